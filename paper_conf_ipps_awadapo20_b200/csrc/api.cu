@@ -1,0 +1,790 @@
+// api.cu — the C ABI (include/dg.h) on top of the sm_100a kernels.
+#include <algorithm>
+#include <cmath>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <new>
+
+#include "graph.h"
+#include "kernels.h"
+#include "router.h"
+
+using dg::u32;
+using dg::u64;
+
+namespace {
+
+constexpr u64 kMaxVertices = 0xFFFFFFFEull;  // Q18: two sentinel values reserved
+constexpr u64 kMaxBatch = 0xFFFFFFFFull;
+
+#define DG_CK(expr)                                                                   \
+  do {                                                                                \
+    cudaError_t e_ = (expr);                                                          \
+    if (e_ != cudaSuccess) {                                                          \
+      if (std::getenv("DG_DEBUG"))                                                    \
+        std::fprintf(stderr, "dg: CUDA error %s at %s:%d\n", cudaGetErrorString(e_), \
+                     __FILE__, __LINE__);                                             \
+      g->bad = true;                                                                  \
+      return DG_ERR_CUDA;                                                             \
+    }                                                                                 \
+  } while (0)
+
+#define DG_TRY(expr)                  \
+  do {                                \
+    dg_status s_ = (expr);            \
+    if (s_ != DG_OK) return s_;       \
+  } while (0)
+
+bool is_device_ptr(const void* p) {
+  if (!p) return false;
+  cudaPointerAttributes a;
+  if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+    cudaGetLastError();
+    return false;
+  }
+  return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged;
+}
+
+// grow-only scratch buffer
+cudaError_t ensure_buf(dg_graph_s::Buf& b, size_t bytes) {
+  if (bytes <= b.bytes) return cudaSuccess;
+  if (b.p) cudaFree(b.p);
+  b.p = nullptr;
+  b.bytes = 0;
+  size_t want = std::max<size_t>(bytes, 1 << 20);
+  cudaError_t e = cudaMalloc(&b.p, want);
+  if (e == cudaSuccess) b.bytes = want;
+  return e;
+}
+
+// Input buffer: device pointers pass through; host memory is copied to a staging
+// buffer (the call then becomes synchronous).
+dg_status stage_in(dg_graph g, int slot, const void* p, size_t bytes, cudaStream_t s,
+                   const void** out, bool* host) {
+  if (!p || bytes == 0 || is_device_ptr(p)) {
+    *out = p;
+    return DG_OK;
+  }
+  *host = true;
+  DG_CK(ensure_buf(g->stage[slot], bytes));
+  DG_CK(cudaMemcpyAsync(g->stage[slot].p, p, bytes, cudaMemcpyHostToDevice, s));
+  *out = g->stage[slot].p;
+  return DG_OK;
+}
+
+// Output buffer: device pointers pass through; host outputs get a staging buffer
+// that finish_out() copies back.
+dg_status stage_out(dg_graph g, int slot, void* p, size_t bytes, void** out, bool* host) {
+  if (!p || bytes == 0 || is_device_ptr(p)) {
+    *out = p;
+    return DG_OK;
+  }
+  *host = true;
+  DG_CK(ensure_buf(g->stage[slot], bytes));
+  *out = g->stage[slot].p;
+  return DG_OK;
+}
+
+dg_status finish_out(dg_graph g, void* host, const void* dev, size_t bytes, cudaStream_t s) {
+  if (host && dev && host != dev && bytes)
+    DG_CK(cudaMemcpyAsync(host, dev, bytes, cudaMemcpyDeviceToHost, s));
+  return DG_OK;
+}
+
+dg_status read_ctl(dg_graph g, cudaStream_t s) {
+  DG_CK(cudaMemcpyAsync(g->hctl, g->ctl, sizeof(dg::DevCtl), cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaStreamSynchronize(s));
+  return DG_OK;
+}
+
+dg_status status_of(dg_graph g, u32 epoch) {
+  return g->hctl->fail_epoch >= epoch && g->hctl->fail_epoch != 0 ? DG_ERR_VERTEX_OUT_OF_RANGE
+                                                                   : DG_OK;
+}
+
+dg_status ensure_bitmap(dg_graph g, u64 nv) {
+  const u64 words = (nv + 31) / 32 + 1;
+  if (words > g->bitmap_words) {
+    if (g->bitmap) cudaFree(g->bitmap);
+    g->bitmap = nullptr;
+    g->bitmap_words = 0;
+    DG_CK(cudaMalloc(&g->bitmap, words * 4));
+    g->bitmap_words = words;
+  }
+  return DG_OK;
+}
+
+dg_status ensure_dedup(dg_graph g, u64 n) {
+  if (n > g->dedup_cap) {
+    if (g->dedup) cudaFree(g->dedup);
+    g->dedup = nullptr;
+    g->dedup_cap = 0;
+    const u64 want = std::max<u64>(n, 4096);
+    DG_CK(cudaMalloc(&g->dedup, want * 4));
+    g->dedup_cap = want;
+  }
+  return DG_OK;
+}
+
+dg_status ensure_retry(dg_graph g, int k, u64 n) {
+  if (n > g->retry_cap[k]) {
+    if (g->retry[k]) cudaFree(g->retry[k]);
+    g->retry[k] = nullptr;
+    g->retry_cap[k] = 0;
+    const u64 want = std::max<u64>(n, 1 << 16);
+    DG_CK(cudaMalloc(&g->retry[k], want * 8));
+    g->retry_cap[k] = want;
+  }
+  return DG_OK;
+}
+
+size_t device_free_bytes() {
+  size_t f = 0, t = 0;
+  if (cudaMemGetInfo(&f, &t) != cudaSuccess) {
+    cudaGetLastError();
+    return 0;
+  }
+  return f;
+}
+
+}  // namespace
+
+namespace dg {
+
+// Map more pool memory so that at least min_buckets buckets exist; new buckets
+// are all-EMPTY (0xFF bytes: EMPTY keys/values, NIL next, NIL owner).
+dg_status grow_pool(dg_graph g, u64 min_buckets, cudaStream_t s) {
+  const u64 max_buckets = std::min<u64>(0xFFFFFFFEull, g->pool.reserved() / g->bucket_bytes);
+  if (min_buckets > max_buckets) return DG_ERR_OUT_OF_MEMORY;
+  if (min_buckets <= g->cap) return DG_OK;
+  cudaError_t e = g->pool.ensure(min_buckets * g->bucket_bytes, 0xFF, s);
+  if (e == cudaErrorMemoryAllocation) {
+    cudaGetLastError();
+    return DG_ERR_OUT_OF_MEMORY;
+  }
+  DG_CK(e);
+  const u64 nb = std::min<u64>(max_buckets, g->pool.mapped() / g->bucket_bytes);
+  e = g->stack.ensure(nb * 4, -1, s);
+  if (e == cudaErrorMemoryAllocation) {
+    cudaGetLastError();
+    return DG_ERR_OUT_OF_MEMORY;
+  }
+  DG_CK(e);
+  g->cap = (u32)nb;
+  return DG_OK;
+}
+
+namespace {
+
+// Make sure an insert launch that may allocate `need` buckets cannot fail, if
+// that is cheap; returns whether the launch must run in retry mode (check for
+// failed ops after the launch and re-run them after growing the pool).
+dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) {
+  *retry_mode = false;
+  if (g->snap_pending && cudaEventQuery(g->snap_event) == cudaSuccess) {
+    g->snap_pending = false;
+    g->bump_ub = g->hctl->bump;  // exact as of the snapshot; nothing launched since
+  }
+  if ((u64)g->cap >= g->bump_ub + need) return DG_OK;
+  // exact free count
+  DG_TRY(read_ctl(g, s));
+  g->snap_pending = false;
+  g->bump_ub = g->hctl->bump;
+  const u64 free_exact = (u64)g->cap - g->hctl->bump + g->hctl->stack_size;
+  if (free_exact >= need) {
+    // pops come from the stack first; the bump cursor moves by at most need - stack
+    return DG_OK;
+  }
+  const u64 missing = need - free_exact;
+  static const bool no_upfront = std::getenv("DG_TEST_RETRY_PATH") != nullptr;
+  const u64 limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
+  if (!no_upfront && missing * g->bucket_bytes <= limit) {
+    const u64 want = (u64)g->cap + missing + std::max<u64>(missing / 4, 65536);
+    dg_status st = grow_pool(g, want, s);
+    if (st == DG_OK) return DG_OK;
+    if (st != DG_ERR_OUT_OF_MEMORY) return st;
+  }
+  *retry_mode = true;
+  return DG_OK;
+}
+
+void note_launch(dg_graph g, u64 need, cudaStream_t s) {
+  g->bump_ub = std::min<u64>(g->cap, g->bump_ub + need);
+  // snapshot the allocator cursors asynchronously when the bound gets tight
+  if ((u64)g->cap < g->bump_ub + need && !g->snap_pending) {
+    if (cudaMemcpyAsync(g->hctl, g->ctl, sizeof(dg::DevCtl), cudaMemcpyDeviceToHost, s) ==
+            cudaSuccess &&
+        cudaEventRecord(g->snap_event, s) == cudaSuccess)
+      g->snap_pending = true;
+    else
+      cudaGetLastError();
+  }
+}
+
+}  // namespace
+
+// insert n edges already resident on this GPU (their sources are local rows)
+dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n, bool mirror,
+                       u32 epoch, cudaStream_t s) {
+  dg::Tables t = g->tables();
+  const u64 n_ops = mirror ? 2 * n : n;
+  if (n_ops == 0) return DG_OK;
+  const u64 need = n_ops + dg::max_groups(g->G, g->sms);
+  bool retry_mode = false;
+  // the snapshot must not be in flight while read_ctl rewrites hctl
+  if (g->snap_pending) {
+    DG_CK(cudaEventSynchronize(g->snap_event));
+  }
+  DG_TRY(plan_capacity(g, need, s, &retry_mode));
+  DG_TRY(ensure_retry(g, 0, n_ops));
+  t = g->tables();
+  dg::EdgeBatch a{};
+  a.src = src;
+  a.dst = dst;
+  a.w = w;
+  a.n = n;
+  a.idx = nullptr;
+  a.n_ops = n_ops;
+  a.retry_out = g->retry[0];
+  a.epoch = epoch;
+  a.nv = g->nv;
+  DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
+  DG_CK(dg::launch_fixup_alloc(t, s));
+  if (!retry_mode) {
+    note_launch(g, need, s);
+    return DG_OK;
+  }
+  // retry mode: re-run the ops that found no free bucket after growing the pool
+  int cur = 0;
+  for (int round = 0;; ++round) {
+    DG_TRY(read_ctl(g, s));
+    g->bump_ub = g->hctl->bump;
+    const u64 failed = g->hctl->retry_count;
+    if (failed == 0) break;
+    if (round > 64) return DG_ERR_OUT_OF_MEMORY;
+    const u64 want = (u64)g->cap + failed + dg::max_groups(g->G, g->sms) + (u64)g->cap / 4;
+    DG_TRY(grow_pool(g, want, s));
+    DG_TRY(ensure_retry(g, cur ^ 1, failed));
+    DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, sizeof(u32), s));
+    t = g->tables();
+    a.idx = g->retry[cur];
+    a.n_ops = failed;
+    a.retry_out = g->retry[cur ^ 1];
+    DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
+    DG_CK(dg::launch_fixup_alloc(t, s));
+    cur ^= 1;
+  }
+  return DG_OK;
+}
+
+dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
+                       cudaStream_t s) {
+  const u64 n_ops = mirror ? 2 * n : n;
+  if (n_ops == 0) return DG_OK;
+  dg::EdgeBatch a{};
+  a.src = src;
+  a.dst = dst;
+  a.n = n;
+  a.n_ops = n_ops;
+  a.epoch = epoch;
+  a.nv = g->nv;
+  DG_CK(dg::launch_delete(g->G, g->tables(), a, g->sms, s));
+  return DG_OK;
+}
+
+dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t* found, u32* wout,
+                      u32 epoch, cudaStream_t s) {
+  if (n == 0) return DG_OK;
+  dg::EdgeBatch a{};
+  a.src = src;
+  a.dst = dst;
+  a.n = n;
+  a.n_ops = n;
+  a.epoch = epoch;
+  a.nv = g->nv;
+  a.found = found;
+  a.wout = wout;
+  DG_CK(dg::launch_query(g->G, g->tables(), a, g->sms, s));
+  return DG_OK;
+}
+
+}  // namespace dg
+
+// ======================================================================= C ABI ==
+extern "C" {
+
+void dg_config_init(dg_config* c) {
+  if (!c) return;
+  std::memset(c, 0, sizeof(*c));
+  c->struct_size = sizeof(dg_config);
+  c->load_factor = 0.7f;
+  c->bucket_bytes = 128;
+  c->directed = 1;
+  c->pool_bytes = 0;
+  c->device = -1;
+  c->rank = 0;
+  c->nranks = 1;
+  c->nccl_unique_id = nullptr;
+}
+
+const char* dg_status_string(dg_status s) {
+  switch (s) {
+    case DG_OK: return "DG_OK";
+    case DG_ERR_INVALID_ARGUMENT: return "DG_ERR_INVALID_ARGUMENT";
+    case DG_ERR_VERTEX_OUT_OF_RANGE: return "DG_ERR_VERTEX_OUT_OF_RANGE";
+    case DG_ERR_OUT_OF_MEMORY: return "DG_ERR_OUT_OF_MEMORY";
+    case DG_ERR_CUDA: return "DG_ERR_CUDA";
+    case DG_ERR_NCCL: return "DG_ERR_NCCL";
+    case DG_ERR_BAD_STATE: return "DG_ERR_BAD_STATE";
+    case DG_ERR_UNSUPPORTED: return "DG_ERR_UNSUPPORTED";
+  }
+  return "DG_ERR_UNKNOWN";
+}
+
+dg_status dg_get_unique_id(void* out128) {
+  if (!out128) return DG_ERR_INVALID_ARGUMENT;
+  return dg::router_unique_id(out128);
+}
+
+static void destroy_graph(dg_graph g) {
+  if (!g) return;
+  cudaSetDevice(g->device);
+  cudaDeviceSynchronize();
+  cudaGetLastError();
+  if (g->router) dg::router_destroy(g->router);
+  g->dir.release();
+  g->pool.release();
+  g->stack.release();
+  if (g->ctl) cudaFree(g->ctl);
+  if (g->hctl) cudaFreeHost(g->hctl);
+  if (g->snap_event) cudaEventDestroy(g->snap_event);
+  if (g->ret_list) cudaFree(g->ret_list);
+  for (auto* p : g->retry)
+    if (p) cudaFree(p);
+  if (g->bitmap) cudaFree(g->bitmap);
+  if (g->dedup) cudaFree(g->dedup);
+  if (g->scan_temp) cudaFree(g->scan_temp);
+  if (g->stats_dev) cudaFree(g->stats_dev);
+  if (g->small_dev) cudaFree(g->small_dev);
+  for (auto& b : g->stage)
+    if (b.p) cudaFree(b.p);
+  cudaGetLastError();
+  delete g;
+}
+
+// Allocate base buckets for rows [row0, row0+count) from the bump region and
+// initialise their directory entries (one bulk allocation).
+static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_global,
+                          const u32* hints_local, u64 slack_buckets, cudaStream_t s) {
+  if (count == 0) return DG_OK;
+  u64* nb = nullptr;
+  u64* off = nullptr;
+  DG_CK(cudaMallocAsync(&nb, (count + 1) * 8, s));
+  DG_CK(cudaMallocAsync(&off, (count + 1) * 8, s));
+  DG_CK(dg::launch_initial_buckets(nb, count, row0, hints_global, hints_local, g->nranks, g->rank,
+                                   g->lf_milli, g->BC, s));
+  DG_CK(dg::scan_exclusive_u64(nb, off, count + 1, &g->scan_temp, &g->scan_bytes, s));
+  u64 total = 0;
+  DG_CK(cudaMemcpyAsync(&total, off + count, 8, cudaMemcpyDeviceToHost, s));
+  DG_TRY(read_ctl(g, s));  // also synchronises
+  const u64 base0 = g->hctl->bump;
+  if (base0 + total + 1 >= 0xFFFFFFFEull) {
+    cudaFreeAsync(nb, s);
+    cudaFreeAsync(off, s);
+    return DG_ERR_OUT_OF_MEMORY;
+  }
+  dg_status st = dg::grow_pool(g, base0 + total + slack_buckets, s);
+  if (st != DG_OK) {
+    cudaFreeAsync(nb, s);
+    cudaFreeAsync(off, s);
+    return st;
+  }
+  cudaError_t e = g->dir.ensure((row0 + count) * sizeof(dg::DirEntry), 0, s);
+  if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
+  DG_CK(e);
+  g->rows = row0 + count;
+  DG_CK(dg::launch_init_rows(g->G, g->tables(), row0, count, off, nb, (u32)base0, s));
+  const u32 newbump = (u32)(base0 + total);
+  DG_CK(cudaMemcpyAsync(&g->ctl->bump, &newbump, 4, cudaMemcpyHostToDevice, s));
+  DG_CK(cudaFreeAsync(nb, s));
+  DG_CK(cudaFreeAsync(off, s));
+  DG_CK(cudaStreamSynchronize(s));
+  g->bump_ub = std::max<u64>(g->bump_ub, newbump);
+  return DG_OK;
+}
+
+dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t* degree_hints,
+                    void* stream, dg_graph* out) {
+  if (!cfg || !out) return DG_ERR_INVALID_ARGUMENT;
+  *out = nullptr;
+  if (cfg->struct_size != sizeof(dg_config)) return DG_ERR_INVALID_ARGUMENT;
+  if (num_vertices > kMaxVertices) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->bucket_bytes != 32 && cfg->bucket_bytes != 64 && cfg->bucket_bytes != 128)
+    return DG_ERR_INVALID_ARGUMENT;
+  if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
+
+  dg_graph g = new (std::nothrow) dg_graph_s();
+  if (!g) return DG_ERR_OUT_OF_MEMORY;
+  g->cfg = *cfg;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  auto fail = [&](dg_status st) {
+    destroy_graph(g);
+    return st;
+  };
+  if (cfg->device >= 0) {
+    if (cudaSetDevice(cfg->device) != cudaSuccess) return fail(DG_ERR_CUDA);
+    g->device = cfg->device;
+  } else if (cudaGetDevice(&g->device) != cudaSuccess) {
+    return fail(DG_ERR_CUDA);
+  }
+  cudaDeviceProp prop;
+  if (cudaGetDeviceProperties(&prop, g->device) != cudaSuccess) return fail(DG_ERR_CUDA);
+  g->sms = prop.multiProcessorCount;
+  g->bucket_bytes = cfg->bucket_bytes;
+  g->G = (int)(cfg->bucket_bytes / 16);
+  g->W = cfg->bucket_bytes / 4;
+  g->BC = cfg->bucket_bytes / 8 - 1;
+  g->lf_milli = std::max<u32>(1, (u32)std::lround((double)cfg->load_factor * 1000.0));
+  g->nranks = (u32)cfg->nranks;
+  g->rank = (u32)cfg->rank;
+  g->directed = cfg->directed != 0;
+  g->nv = num_vertices;
+
+  const size_t total_mem = prop.totalGlobalMem;
+  if (g->pool.reserve(g->device, total_mem) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (g->stack.reserve(g->device, total_mem / g->bucket_bytes * 4 + (2u << 20)) != cudaSuccess)
+    return fail(DG_ERR_CUDA);
+  const u64 max_rows = (kMaxVertices + g->nranks - 1) / g->nranks + 1;
+  if (g->dir.reserve(g->device, max_rows * sizeof(dg::DirEntry)) != cudaSuccess)
+    return fail(DG_ERR_CUDA);
+  if (cudaMalloc(&g->ctl, sizeof(dg::DevCtl)) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (cudaMemsetAsync(g->ctl, 0, sizeof(dg::DevCtl), s) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (cudaMallocHost(&g->hctl, sizeof(dg::DevCtl)) != cudaSuccess) return fail(DG_ERR_CUDA);
+  std::memset(g->hctl, 0, sizeof(dg::DevCtl));
+  if (cudaEventCreateWithFlags(&g->snap_event, cudaEventDisableTiming) != cudaSuccess)
+    return fail(DG_ERR_CUDA);
+  if (cudaMalloc(&g->ret_list, dg::max_groups(g->G, g->sms) * 4 + 64) != cudaSuccess)
+    return fail(DG_ERR_CUDA);
+  if (cudaMalloc(&g->small_dev, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (cudaMalloc(&g->stats_dev, sizeof(dg::StatsOut)) != cudaSuccess) return fail(DG_ERR_CUDA);
+
+  if (g->nranks > 1) {
+    dg_status st = dg::router_create(g, cfg->nccl_unique_id, &g->router);
+    if (st != DG_OK) return fail(st);
+  }
+
+  // hints: indexed by global vertex id
+  const void* hints = nullptr;
+  bool host = false;
+  dg_status st = stage_in(g, 0, degree_hints, degree_hints ? num_vertices * 4 : 0, s, &hints, &host);
+  if (st != DG_OK) return fail(st);
+  const u64 rows = dg::rows_for(num_vertices, g->nranks, g->rank);
+  // overflow slack beyond the base buckets
+  u64 slack = cfg->pool_bytes ? cfg->pool_bytes / g->bucket_bytes : 0;
+  if (!cfg->pool_bytes) slack = std::max<u64>(rows / 4, 1u << 16);
+  if (rows) {
+    st = add_rows(g, 0, rows, reinterpret_cast<const u32*>(hints), nullptr, slack, s);
+  } else {
+    st = dg::grow_pool(g, slack, s);
+  }
+  if (st != DG_OK) return fail(st);
+  if (cudaStreamSynchronize(s) != cudaSuccess) return fail(DG_ERR_CUDA);
+  *out = g;
+  return DG_OK;
+}
+
+dg_status dg_destroy(dg_graph g) {
+  if (!g) return DG_ERR_INVALID_ARGUMENT;
+  destroy_graph(g);
+  return DG_OK;
+}
+
+dg_status dg_num_vertices(dg_graph g, uint64_t* num_vertices, uint64_t* local_rows) {
+  if (!g) return DG_ERR_INVALID_ARGUMENT;
+  if (num_vertices) *num_vertices = g->nv;
+  if (local_rows) *local_rows = g->rows;
+  return DG_OK;
+}
+
+static dg_status check_handle(dg_graph g) {
+  if (!g) return DG_ERR_INVALID_ARGUMENT;
+  if (g->bad) return DG_ERR_BAD_STATE;
+  if (cudaSetDevice(g->device) != cudaSuccess) {
+    g->bad = true;
+    return DG_ERR_CUDA;
+  }
+  return DG_OK;
+}
+
+dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
+                          const uint32_t* weight, uint64_t n, uint64_t* n_added, void* stream) {
+  DG_TRY(check_handle(g));
+  if (n > kMaxBatch) return DG_ERR_INVALID_ARGUMENT;
+  if (n && (!src || !dst)) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  if (n_added) *n_added = 0;
+  const u32 epoch = ++g->epoch;
+  bool host = false;
+  const void *ds = nullptr, *dd = nullptr, *dw = nullptr;
+  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
+  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
+  DG_TRY(stage_in(g, 2, weight, weight ? n * 4 : 0, s, &dw, &host));
+  if (g->nranks > 1) {
+    DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
+  } else {
+    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
+                            epoch, s));
+  }
+  if (n_added || host) {
+    DG_TRY(read_ctl(g, s));
+    u64 cnt = g->hctl->count;
+    if (g->nranks > 1) DG_TRY(dg::router_sum_u64(g, &cnt, s));
+    if (n_added) *n_added = cnt;
+    g->snap_pending = false;
+    g->bump_ub = g->hctl->bump;
+    return status_of(g, epoch);
+  }
+  return DG_OK;
+}
+
+dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
+                          uint64_t* n_removed, void* stream) {
+  DG_TRY(check_handle(g));
+  if (n > kMaxBatch) return DG_ERR_INVALID_ARGUMENT;
+  if (n && (!src || !dst)) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  if (n_removed) *n_removed = 0;
+  const u32 epoch = ++g->epoch;
+  bool host = false;
+  const void *ds = nullptr, *dd = nullptr;
+  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
+  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
+  if (g->nranks > 1) {
+    DG_TRY(dg::router_delete(g, (const u32*)ds, (const u32*)dd, n, epoch, s));
+  } else {
+    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s));
+  }
+  if (n_removed || host) {
+    if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+    g->snap_pending = false;
+    DG_TRY(read_ctl(g, s));
+    u64 cnt = g->hctl->count;
+    if (g->nranks > 1) DG_TRY(dg::router_sum_u64(g, &cnt, s));
+    if (n_removed) *n_removed = cnt;
+    return status_of(g, epoch);
+  }
+  return DG_OK;
+}
+
+dg_status dg_query_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
+                         uint8_t* found, uint32_t* weight_out, void* stream) {
+  DG_TRY(check_handle(g));
+  if (n > kMaxBatch) return DG_ERR_INVALID_ARGUMENT;
+  if (n && (!src || !dst || !found)) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  const u32 epoch = ++g->epoch;
+  bool host = false;
+  const void *ds = nullptr, *dd = nullptr;
+  void *df = nullptr, *dw = nullptr;
+  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
+  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
+  DG_TRY(stage_out(g, 3, found, n, &df, &host));
+  DG_TRY(stage_out(g, 4, weight_out, weight_out ? n * 4 : 0, &dw, &host));
+  if (g->nranks > 1) {
+    DG_TRY(dg::router_query(g, (const u32*)ds, (const u32*)dd, n, (uint8_t*)df, (u32*)dw, epoch, s));
+  } else {
+    DG_TRY(dg::local_query(g, (const u32*)ds, (const u32*)dd, n, (uint8_t*)df, (u32*)dw, epoch, s));
+  }
+  if (host) {
+    DG_TRY(finish_out(g, found, df, n, s));
+    DG_TRY(finish_out(g, weight_out, dw, weight_out ? n * 4 : 0, s));
+    if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+    g->snap_pending = false;
+    DG_TRY(read_ctl(g, s));
+    return status_of(g, epoch);
+  }
+  return DG_OK;
+}
+
+dg_status dg_insert_vertices(dg_graph g, const uint32_t* ids, uint64_t n,
+                             const uint32_t* degree_hints, void* stream) {
+  DG_TRY(check_handle(g));
+  if (n > kMaxBatch) return DG_ERR_INVALID_ARGUMENT;
+  if (n && !ids) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  bool host = false;
+  const void *di = nullptr, *dh = nullptr;
+  DG_TRY(stage_in(g, 5, ids, n * 4, s, &di, &host));
+  DG_TRY(stage_in(g, 6, degree_hints, degree_hints ? n * 4 : 0, s, &dh, &host));
+  u64 maxid = 0;
+  bool any = n > 0;
+  if (any) {
+    DG_CK(dg::launch_max_id((const u32*)di, n, g->small_dev, s));
+    u32 m = 0;
+    DG_CK(cudaMemcpyAsync(&m, g->small_dev, 4, cudaMemcpyDeviceToHost, s));
+    DG_CK(cudaStreamSynchronize(s));
+    maxid = m;
+    if (maxid >= kMaxVertices) return DG_ERR_VERTEX_OUT_OF_RANGE;
+  }
+  u64 new_nv = g->nv;
+  if (any) new_nv = std::max<u64>(new_nv, maxid + 1);
+  if (g->nranks > 1) DG_TRY(dg::router_max_u64(g, &new_nv, s));
+  if (new_nv <= g->nv) return DG_OK;  // Q12: existing IDs are a no-op
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  g->snap_pending = false;
+  const u64 new_rows = dg::rows_for(new_nv, g->nranks, g->rank);
+  const u64 row0 = g->rows;
+  const u64 count = new_rows - row0;
+  if (count) {
+    u32* hint_new = nullptr;
+    DG_CK(cudaMallocAsync(&hint_new, count * 4, s));
+    DG_CK(cudaMemsetAsync(hint_new, 0, count * 4, s));
+    DG_CK(dg::launch_scatter_hints(hint_new, row0, count, (const u32*)di, (const u32*)dh, n,
+                                   g->nranks, g->rank, s));
+    dg_status st = add_rows(g, row0, count, nullptr, hint_new, std::max<u64>(count / 4, 4096), s);
+    cudaFreeAsync(hint_new, s);
+    if (st != DG_OK) return st;
+  }
+  g->nv = new_nv;
+  DG_CK(cudaStreamSynchronize(s));
+  return DG_OK;
+}
+
+dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* stream) {
+  DG_TRY(check_handle(g));
+  if (n > kMaxBatch) return DG_ERR_INVALID_ARGUMENT;
+  if (n && !ids) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  const u32 epoch = ++g->epoch;
+  bool host = false;
+  const void* di = nullptr;
+  DG_TRY(stage_in(g, 5, ids, n * 4, s, &di, &host));
+  const u32* all_ids = (const u32*)di;
+  u64 all_n = n;
+  if (g->nranks > 1) DG_TRY(dg::router_allgather_ids(g, all_ids, n, &all_ids, &all_n, s));
+  if (all_n == 0) return DG_OK;
+  DG_TRY(ensure_bitmap(g, g->nv));
+  DG_TRY(ensure_dedup(g, all_n));
+  DG_CK(cudaMemsetAsync(g->bitmap, 0, ((g->nv + 31) / 32 + 1) * 4, s));
+  DG_CK(cudaMemsetAsync(&g->ctl->queue, 0, 2 * sizeof(u32), s));  // queue, dedup_count
+  const dg::Tables t = g->tables();
+  DG_CK(dg::launch_vdel_mark(all_ids, all_n, g->nv, epoch, g->bitmap, g->dedup, g->ctl, g->nranks,
+                             g->rank, g->sms, s));
+  static const bool force_sweep = std::getenv("DG_FORCE_SWEEP") != nullptr;
+  if (!g->directed && g->nranks == 1 && !force_sweep) {
+    // undirected: Alg. 2 — delete u from the tables of its neighbours
+    DG_CK(dg::launch_vdel_neighbors(g->G, t, g->dedup, epoch, g->sms, s));
+    DG_CK(cudaMemsetAsync(&g->ctl->queue, 0, sizeof(u32), s));
+  } else {
+    // directed: follow-up sweep over all tables
+    DG_CK(dg::launch_vdel_sweep(g->G, t, g->bitmap, epoch, g->sms, s));
+  }
+  DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, epoch, g->sms, s));
+  if (host) {
+    if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+    g->snap_pending = false;
+    DG_TRY(read_ctl(g, s));
+    return status_of(g, epoch);
+  }
+  return DG_OK;
+}
+
+dg_status dg_export_adjacency(dg_graph g, uint64_t* row_offsets, uint32_t* dst, uint32_t* weight,
+                              uint64_t capacity, uint64_t* n_edges, void* stream) {
+  DG_TRY(check_handle(g));
+  if (!row_offsets || !n_edges) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  bool host = false;
+  void* dro = nullptr;
+  DG_TRY(stage_out(g, 3, row_offsets, (g->rows + 1) * 8, &dro, &host));
+  const dg::Tables t = g->tables();
+  DG_CK(dg::launch_export_offsets(t, (u64*)dro, &g->scan_temp, &g->scan_bytes, s));
+  u64 m = 0;
+  DG_CK(cudaMemcpyAsync(&m, (u64*)dro + g->rows, 8, cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaStreamSynchronize(s));
+  *n_edges = m;
+  if (dst) {
+    if (capacity < m) {
+      DG_TRY(finish_out(g, row_offsets, dro, (g->rows + 1) * 8, s));
+      DG_CK(cudaStreamSynchronize(s));
+      return DG_ERR_INVALID_ARGUMENT;
+    }
+    void *dd = nullptr, *dw = nullptr;
+    DG_TRY(stage_out(g, 4, dst, m * 4, &dd, &host));
+    DG_TRY(stage_out(g, 7, weight, weight ? m * 4 : 0, &dw, &host));
+    DG_CK(dg::launch_export_fill(g->G, t, (const u64*)dro, (u32*)dd, (u32*)dw, g->sms, s));
+    DG_TRY(finish_out(g, dst, dd, m * 4, s));
+    DG_TRY(finish_out(g, weight, dw, weight ? m * 4 : 0, s));
+  }
+  DG_TRY(finish_out(g, row_offsets, dro, (g->rows + 1) * 8, s));
+  DG_CK(cudaStreamSynchronize(s));
+  return DG_OK;
+}
+
+dg_status dg_degrees(dg_graph g, uint32_t* out, void* stream) {
+  DG_TRY(check_handle(g));
+  if (!out) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  bool host = false;
+  void* d = nullptr;
+  DG_TRY(stage_out(g, 3, out, g->rows * 4, &d, &host));
+  DG_CK(dg::launch_degrees(g->tables(), (u32*)d, s));
+  if (host) {
+    DG_TRY(finish_out(g, out, d, g->rows * 4, s));
+    DG_CK(cudaStreamSynchronize(s));
+  }
+  return DG_OK;
+}
+
+dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
+  DG_TRY(check_handle(g));
+  if (!out) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  dg::StatsOut h{};
+  auto* d = reinterpret_cast<dg::StatsOut*>(g->stats_dev);
+  DG_CK(dg::launch_stats(g->G, g->tables(), d, g->sms, s));
+  DG_CK(cudaMemcpyAsync(&h, d, sizeof(h), cudaMemcpyDeviceToHost, s));
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  g->snap_pending = false;
+  DG_TRY(read_ctl(g, s));
+  std::memset(out, 0, sizeof(*out));
+  out->local_rows = g->rows;
+  out->base_buckets = h.base_buckets;
+  out->overflow_buckets = h.linked_buckets - h.base_buckets;
+  out->free_buckets = g->hctl->stack_size;
+  out->pool_buckets = g->cap;
+  out->live_pairs = h.live;
+  out->tombstones = h.tombs;
+  out->max_chain = h.max_chain;
+  out->pool_bytes = g->pool.mapped() + g->dir.mapped() + g->stack.mapped();
+  out->load_factor = h.linked_buckets ? (double)h.live / ((double)h.linked_buckets * g->BC) : 0.0;
+  out->utilization =
+      h.linked_buckets ? (double)h.live * 8.0 / ((double)h.linked_buckets * g->bucket_bytes) : 0.0;
+  return DG_OK;
+}
+
+dg_status dg_batch_status(dg_graph g, void* stream) {
+  DG_TRY(check_handle(g));
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  g->snap_pending = false;
+  DG_TRY(read_ctl(g, s));
+  dg_status st = DG_OK;
+  if (g->hctl->fail_epoch > g->checked_epoch) st = DG_ERR_VERTEX_OUT_OF_RANGE;
+  g->checked_epoch = g->epoch;
+  return st;
+}
+
+dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream) {
+  DG_TRY(check_handle(g));
+  (void)count;
+  (void)stream;
+  return DG_ERR_UNSUPPORTED;
+}
+
+}  // extern "C"

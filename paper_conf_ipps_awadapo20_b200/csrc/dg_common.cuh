@@ -1,0 +1,142 @@
+// dg_common.cuh — device-side layout and primitives shared by the kernels.
+//
+// Data layout in HBM:
+//   directory  : DirEntry[local_rows], 16 B per row {base bucket, #buckets, degree, flags}
+//                (the paper's vertex dictionary)
+//   pool       : bucket array; bucket b occupies words [b*W, (b+1)*W), W = bucket_bytes/4.
+//                words 2i, 2i+1 = (key, value) of pair i, i < BC = W/2 - 1
+//                word W-2 = next bucket index of the chain (NIL = 0xFFFFFFFF)
+//                word W-1 = owner row of the bucket (for the streaming purge sweep)
+//                Base buckets of a row are consecutive (Fig. 1 caption P:L357-363);
+//                chained buckets come from the allocator.
+//   free stack : u32[pool capacity] of reclaimed bucket indices + bump cursor
+//   ctl        : DevCtl (allocator cursors, counters, validation epochs)
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace dg {
+
+typedef uint32_t u32;
+typedef uint64_t u64;
+
+constexpr u32 kEmpty = 0xFFFFFFFFu;       // empty key slot (Q18)
+constexpr u32 kTomb = 0xFFFFFFFEu;        // tombstone (deleted key)
+constexpr u32 kNil = 0xFFFFFFFFu;         // end of chain / no bucket
+constexpr u64 kEmptyPair = 0xFFFFFFFFFFFFFFFFull;
+
+struct __align__(16) DirEntry {
+  u32 base;    // first base bucket
+  u32 nb;      // number of base buckets
+  u32 deg;     // exact number of stored neighbours
+  u32 flags;   // reserved
+};
+
+struct DevCtl {
+  u32 pop_count;     // pops taken from the free stack during the current insert phase
+  u32 stack_size;    // reclaimed buckets on the free stack
+  u32 bump;          // next never-used bucket index
+  u32 ret_count;     // unused spare buckets handed back during the current insert phase
+  u32 retry_count;   // ops that found no free bucket (pool exhausted) this launch
+  u32 fail_epoch;    // highest batch epoch rejected by validation (0 = none)
+  u32 queue;         // work-queue cursor (vertex purge, Alg2:L3-6)
+  u32 dedup_count;   // distinct vertices in the current vertex-deletion batch
+  u64 count;         // n_added / n_removed / TC accumulator of the current batch
+  u64 aux;
+};
+
+struct Tables {
+  DirEntry* dir;
+  u32* pool;
+  u32* stack;
+  DevCtl* ctl;
+  u32* ret_list;     // spare buckets returned (<= number of groups launched)
+  u64 rows;          // local rows
+  u32 cap;           // buckets mapped in the pool
+  u32 nranks;        // row = global id / nranks at nranks > 1
+};
+
+// ------------------------------------------------------------------ hashing ----
+// Q16: murmur3 fmix32, then multiply-shift onto [0, nb).  The paper defers the
+// hash to Slab Hash [6]; results are hash-independent.
+__device__ __forceinline__ u32 fmix32(u32 h) {
+  h ^= h >> 16; h *= 0x85ebca6bu;
+  h ^= h >> 13; h *= 0xc2b2ae35u;
+  h ^= h >> 16;
+  return h;
+}
+__device__ __forceinline__ u32 bucket_of(u32 key, u32 nb) {
+  return (u32)(((u64)fmix32(key) * (u64)nb) >> 32);
+}
+
+// ------------------------------------------------------------------ memory ----
+__device__ __forceinline__ uint4 ld_relaxed_v4(const u32* p) {
+  uint4 r;
+  asm volatile("ld.relaxed.gpu.global.v4.u32 {%0,%1,%2,%3}, [%4];"
+               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p) : "memory");
+  return r;
+}
+__device__ __forceinline__ uint4 ld_nc_v4(const u32* p) {
+  uint4 r;
+  asm volatile("ld.global.nc.v4.u32 {%0,%1,%2,%3}, [%4];"
+               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
+  return r;
+}
+__device__ __forceinline__ uint4 ld_nc_dir(const DirEntry* p) {
+  return ld_nc_v4(reinterpret_cast<const u32*>(p));
+}
+__device__ __forceinline__ uint4 ld_dir(const DirEntry* p) {
+  uint4 r;
+  asm volatile("ld.global.v4.u32 {%0,%1,%2,%3}, [%4];"
+               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
+  return r;
+}
+__device__ __forceinline__ u32 ld_relaxed_u32(const u32* p) {
+  u32 r;
+  asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(r) : "l"(p) : "memory");
+  return r;
+}
+__device__ __forceinline__ void st_relaxed_u32(u32* p, u32 v) {
+  asm volatile("st.relaxed.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+__device__ __forceinline__ void st_v4(u32* p, uint4 v) {
+  asm volatile("st.global.v4.u32 [%0], {%1,%2,%3,%4};" ::"l"(p), "r"(v.x), "r"(v.y), "r"(v.z),
+               "r"(v.w) : "memory");
+}
+__device__ __forceinline__ void prefetch_l2(const void* p) {
+  asm volatile("prefetch.global.L2 [%0];" ::"l"(p));
+}
+
+// --------------------------------------------------------------- groups -------
+// A "group" is G consecutive lanes of a warp that together hold one bucket
+// (16 B per lane: G = bucket_bytes/16).  Every group-collective uses the group's
+// own lane mask, so groups of one warp may diverge freely.
+template <int G>
+struct Group {
+  static constexpr int W = 4 * G;         // words per bucket
+  static constexpr int BC = 2 * G - 1;    // pairs per bucket (Q15: 15 / 7 / 3)
+  static constexpr int NEXT = W - 2;
+  static constexpr int OWNER = W - 1;
+  u32 lane;    // lane in warp
+  u32 gl;      // lane in group
+  u32 base;    // first warp lane of the group
+  u32 mask;    // warp mask of the group
+  __device__ __forceinline__ Group() {
+    lane = threadIdx.x & 31u;
+    gl = lane & (G - 1);
+    base = lane & ~(u32)(G - 1);
+    mask = (G == 32 ? 0xFFFFFFFFu : ((1u << G) - 1u)) << base;
+  }
+  __device__ __forceinline__ u32 ballot(bool p) const {
+    return (__ballot_sync(mask, p) >> base) & (G == 32 ? 0xFFFFFFFFu : ((1u << G) - 1u));
+  }
+  template <typename T>
+  __device__ __forceinline__ T shfl(T v, u32 src_gl) const {
+    return __shfl_sync(mask, v, base + src_gl);
+  }
+  __device__ __forceinline__ bool last() const { return gl == (u32)(G - 1); }
+};
+
+__device__ __forceinline__ u64 pack_pair(u32 key, u32 val) { return (u64)key | ((u64)val << 32); }
+
+}  // namespace dg

@@ -1,0 +1,91 @@
+// graph.h — host-side state behind a dg_graph handle.
+#pragma once
+#include <cstddef>
+#include <cstdint>
+
+#include <cuda_runtime.h>
+
+#include "../../include/dg.h"
+#include "dg_common.cuh"
+#include "vmm.h"
+
+namespace dg {
+struct Router;  // multi-GPU batch router (router.cu)
+}
+
+struct dg_graph_s {
+  dg_config cfg{};
+  int device = 0;
+  int sms = 148;
+  int G = 8;              // lanes per bucket (bucket_bytes / 16)
+  uint32_t W = 32;        // words per bucket
+  uint32_t BC = 15;       // pairs per bucket
+  uint32_t bucket_bytes = 128;
+  uint32_t lf_milli = 700;
+  uint32_t nranks = 1, rank = 0;
+  bool directed = true;
+
+  uint64_t nv = 0;        // global vertex capacity
+  uint64_t rows = 0;      // local rows
+
+  dg::VmmArray dir, pool, stack;
+  uint32_t cap = 0;       // buckets mapped in the pool
+  uint64_t bump_ub = 0;   // host upper bound of the device bump cursor
+
+  dg::DevCtl* ctl = nullptr;       // device
+  dg::DevCtl* hctl = nullptr;      // pinned host mirror (snapshots)
+  cudaEvent_t snap_event = nullptr;
+  bool snap_pending = false;
+  uint32_t* ret_list = nullptr;
+  uint64_t* retry[2] = {nullptr, nullptr};
+  uint64_t retry_cap[2] = {0, 0};
+  uint32_t* bitmap = nullptr;
+  uint64_t bitmap_words = 0;
+  uint32_t* dedup = nullptr;
+  uint64_t dedup_cap = 0;
+  void* scan_temp = nullptr;
+  size_t scan_bytes = 0;
+  void* stats_dev = nullptr;
+  uint32_t* small_dev = nullptr;   // scratch words
+
+  uint32_t epoch = 0;
+  uint32_t checked_epoch = 0;
+  bool bad = false;
+
+  struct Buf {
+    void* p = nullptr;
+    size_t bytes = 0;
+  } stage[8];
+
+  dg::Router* router = nullptr;
+
+  dg::Tables tables() const {
+    dg::Tables t;
+    t.dir = reinterpret_cast<dg::DirEntry*>(dir.ptr());
+    t.pool = reinterpret_cast<uint32_t*>(pool.ptr());
+    t.stack = reinterpret_cast<uint32_t*>(stack.ptr());
+    t.ctl = ctl;
+    t.ret_list = ret_list;
+    t.rows = rows;
+    t.cap = cap;
+    t.nranks = nranks;
+    return t;
+  }
+};
+
+namespace dg {
+
+inline uint64_t rows_for(uint64_t nv, uint32_t nranks, uint32_t rank) {
+  return nv > rank ? (nv - rank + nranks - 1) / nranks : 0;
+}
+
+// internal entry points shared by api.cu and router.cu
+dg_status grow_pool(dg_graph g, uint64_t min_buckets, cudaStream_t s);
+dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
+                       uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s);
+dg_status local_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
+                       bool mirror, uint32_t epoch, cudaStream_t s);
+dg_status local_query(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
+                      uint8_t* found, uint32_t* wout, uint32_t epoch, cudaStream_t s);
+
+}  // namespace dg

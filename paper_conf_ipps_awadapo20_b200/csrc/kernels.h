@@ -1,0 +1,78 @@
+// kernels.h — host-callable launchers of the sm_100a kernels.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+#include "dg_common.cuh"
+
+namespace dg {
+
+constexpr int kEdgeBlock = 256;
+
+struct EdgeBatch {
+  const u32* src;
+  const u32* dst;
+  const u32* w;       // insert only, nullable
+  u64 n;              // entries in src/dst/w
+  const u64* idx;     // nullable: op ids to process (retry list)
+  u64 n_ops;          // ops to process (n, 2n for undirected mirror, or |idx|)
+  u64* retry_out;     // insert: op ids that found no free bucket
+  u32 epoch;          // batch epoch (validation)
+  u64 nv;             // global vertex capacity (query range check)
+  uint8_t* found;     // query
+  u32* wout;          // query, nullable
+};
+
+// edge ops (kernels_edges.cu)
+cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
+                            int sms, cudaStream_t s);
+cudaError_t launch_insert(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_delete(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_query(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s);
+u64 max_groups(int G, int sms);
+
+// graph structure (kernels_graph.cu)
+// nb[r] for rows r in [0, count): initial bucket count from a hint.
+//   hint source: hints_global[(row0 + r) * nranks + rank] if hints_global, else
+//   hints_local[r] if hints_local, else 0.
+cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
+                                   const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
+                                   u32 bc, cudaStream_t s);
+// out[i] = sum of in[0..i) for i < count (temp storage grows as needed)
+cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
+                               size_t* temp_bytes, cudaStream_t s);
+// dir[row0 + r] = {base0 + off[r], nb[r], 0, 0}; owner word of each base bucket = row
+cudaError_t launch_init_rows(int G, const Tables& t, u64 row0, u64 count, const u64* off,
+                             const u64* nb, u32 base0, cudaStream_t s);
+// new-row hints for vertex insertion (scatter, max over duplicates)
+cudaError_t launch_scatter_hints(u32* hint_new, u64 row0, u64 count, const u32* ids,
+                                 const u32* hints, u64 n, u32 nranks, u32 rank, cudaStream_t s);
+cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s);
+
+cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s);
+cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
+                                  cudaStream_t s);
+cudaError_t launch_export_fill(int G, const Tables& t, const u64* ro, u32* dst, u32* w,
+                               int sms, cudaStream_t s);
+
+struct StatsOut {
+  unsigned long long base_buckets, linked_buckets, live, tombs, max_chain;
+};
+cudaError_t launch_stats(int G, const Tables& t, StatsOut* out, int sms, cudaStream_t s);
+
+// vertex deletion (kernels_graph.cu)
+cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
+                             DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s);
+cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epoch, int sms,
+                              cudaStream_t s);
+cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
+                                  cudaStream_t s);
+cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
+                              cudaStream_t s);
+
+// triangle counting consumer (kernels_tc.cu)
+cudaError_t launch_tc(int G, const Tables& t, const u64* ro, const u32* adj, u32 part,
+                      u32 nparts, int sms, cudaStream_t s);
+
+}  // namespace dg

@@ -1,0 +1,461 @@
+// kernels_graph.cu — table construction, export, statistics and vertex deletion.
+#include <cub/device/device_scan.cuh>
+#include <thrust/iterator/counting_iterator.h>
+#include <thrust/iterator/transform_iterator.h>
+
+#include "dg_common.cuh"
+#include "kernels.h"
+
+namespace dg {
+
+// ------------------------------------------------------ initial buckets (a0) ----
+// #buckets of a new table = ceil(|A_u| / (lf * Bc)), one bucket when |A_u| is
+// unknown.  lf is carried in thousandths so the
+// ceiling is an exact integer decision (reading R-LF).
+__global__ void k_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
+                                  const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
+                                  u32 bc) {
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r <= count; r += stride) {
+    if (r == count) {
+      nb[r] = 0;
+      continue;
+    }
+    u64 hint = 0;
+    if (hints_global) hint = hints_global[(row0 + r) * nranks + rank];
+    else if (hints_local) hint = hints_local[r];
+    const u64 den = (u64)lf_milli * bc;
+    u64 b = hint ? (hint * 1000 + den - 1) / den : 1;
+    nb[r] = b ? b : 1;
+  }
+}
+
+cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
+                                   const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
+                                   u32 bc, cudaStream_t s) {
+  u64 blocks = (count + 1 + 255) / 256;
+  if (blocks > 65535) blocks = 65535;
+  k_initial_buckets<<<(unsigned)blocks, 256, 0, s>>>(nb, count, row0, hints_global, hints_local,
+                                                     nranks, rank, lf_milli, bc);
+  return cudaGetLastError();
+}
+
+cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
+                               size_t* temp_bytes, cudaStream_t s) {
+  size_t need = 0;
+  cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, in, out, (int64_t)count, s);
+  if (e != cudaSuccess) return e;
+  if (need > *temp_bytes) {
+    if (*temp) cudaFree(*temp);
+    *temp = nullptr;
+    *temp_bytes = 0;
+    e = cudaMalloc(temp, need);
+    if (e != cudaSuccess) return e;
+    *temp_bytes = need;
+  }
+  return cub::DeviceScan::ExclusiveSum(*temp, need, in, out, (int64_t)count, s);
+}
+
+// dir[row0 + r] = {base0 + off[r], nb[r], 0, 0}; each base bucket records its owner row.
+template <int G>
+__global__ void k_init_rows(Tables t, u64 row0, u64 count, const u64* off, const u64* nb,
+                            u32 base0) {
+  constexpr int W = Group<G>::W;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < count; r += stride) {
+    const u32 base = base0 + (u32)off[r];
+    const u32 n = (u32)nb[r];
+    DirEntry e;
+    e.base = base;
+    e.nb = n;
+    e.deg = 0;
+    e.flags = 0;
+    t.dir[row0 + r] = e;
+    for (u32 k = 0; k < n; ++k) t.pool[(u64)(base + k) * W + Group<G>::OWNER] = (u32)(row0 + r);
+  }
+}
+
+cudaError_t launch_init_rows(int G, const Tables& t, u64 row0, u64 count, const u64* off,
+                             const u64* nb, u32 base0, cudaStream_t s) {
+  if (count == 0) return cudaSuccess;
+  u64 blocks = (count + 255) / 256;
+  if (blocks > 65535) blocks = 65535;
+  switch (G) {
+    case 2: k_init_rows<2><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
+    case 4: k_init_rows<4><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
+    case 8: k_init_rows<8><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+// ---------------------------------------------------------- vertex insertion ----
+__global__ void k_scatter_hints(u32* hint_new, u64 row0, u64 count, const u32* ids,
+                                const u32* hints, u64 n, u32 nranks, u32 rank) {
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+    const u32 id = ids[i];
+    if (id % nranks != rank) continue;
+    const u64 row = id / nranks;
+    if (row >= row0 && row < row0 + count) atomicMax(&hint_new[row - row0], hints ? hints[i] : 0u);
+  }
+}
+
+cudaError_t launch_scatter_hints(u32* hint_new, u64 row0, u64 count, const u32* ids,
+                                 const u32* hints, u64 n, u32 nranks, u32 rank, cudaStream_t s) {
+  if (n == 0) return cudaSuccess;
+  u64 blocks = (n + 255) / 256;
+  if (blocks > 65535) blocks = 65535;
+  k_scatter_hints<<<(unsigned)blocks, 256, 0, s>>>(hint_new, row0, count, ids, hints, n, nranks,
+                                                   rank);
+  return cudaGetLastError();
+}
+
+__global__ void k_max_id(const u32* ids, u64 n, u32* out) {
+  u32 m = 0;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) m = max(m, ids[i]);
+  m = __reduce_max_sync(0xFFFFFFFFu, m);
+  if ((threadIdx.x & 31) == 0) atomicMax(out, m);
+}
+
+cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s) {
+  cudaError_t e = cudaMemsetAsync(out, 0, sizeof(u32), s);
+  if (e != cudaSuccess || n == 0) return e;
+  u64 blocks = (n + 255) / 256;
+  if (blocks > 1024) blocks = 1024;
+  k_max_id<<<(unsigned)blocks, 256, 0, s>>>(ids, n, out);
+  return cudaGetLastError();
+}
+
+// ------------------------------------------------------------------ degrees ----
+__global__ void k_degrees(const DirEntry* dir, u64 rows, u32* out) {
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < rows; r += stride)
+    out[r] = dir[r].deg;
+}
+
+cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s) {
+  if (t.rows == 0) return cudaSuccess;
+  u64 blocks = (t.rows + 255) / 256;
+  if (blocks > 65535) blocks = 65535;
+  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.dir, t.rows, out);
+  return cudaGetLastError();
+}
+
+// ------------------------------------------------------------ export (a12) ----
+struct DegAt {
+  const DirEntry* dir;
+  u64 rows;
+  __host__ __device__ u64 operator()(u64 i) const { return i < rows ? (u64)dir[i].deg : 0ull; }
+};
+
+cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
+                                  cudaStream_t s) {
+  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0), DegAt{t.dir, t.rows});
+  size_t need = 0;
+  cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, ro, (int64_t)(t.rows + 1), s);
+  if (e != cudaSuccess) return e;
+  if (need > *temp_bytes) {
+    if (*temp) cudaFree(*temp);
+    *temp = nullptr;
+    *temp_bytes = 0;
+    e = cudaMalloc(temp, need);
+    if (e != cudaSuccess) return e;
+    *temp_bytes = need;
+  }
+  return cub::DeviceScan::ExclusiveSum(*temp, need, it, ro, (int64_t)(t.rows + 1), s);
+}
+
+// One group per row walks every bucket chain of the row (the adjacency iterator,
+// P:L431-436) and writes the live pairs compactly at row_offsets[row].
+template <int G>
+__global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u32* dst, u32* w) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  const u32 below = (1u << g.gl) - 1u;
+  for (u64 row = gid; row < t.rows; row += ng) {
+    const DirEntry de = t.dir[row];
+    u64 pos = ro[row];
+    for (u32 k = 0; k < de.nb; ++k) {
+      u32 b = de.base + k;
+      while (b != kNil) {
+        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
+        const bool l0 = q.x < kTomb;
+        const bool l1 = !g.last() && q.z < kTomb;
+        const u32 m0 = g.ballot(l0), m1 = g.ballot(l1);
+        const u64 before = __popc(m0 & below) + __popc(m1 & below);
+        if (l0) {
+          dst[pos + before] = q.x;
+          if (w) w[pos + before] = q.y;
+        }
+        if (l1) {
+          dst[pos + before + (l0 ? 1 : 0)] = q.z;
+          if (w) w[pos + before + (l0 ? 1 : 0)] = q.w;
+        }
+        pos += __popc(m0) + __popc(m1);
+        b = g.shfl(q.z, G - 1);
+      }
+    }
+  }
+}
+
+cudaError_t launch_export_fill(int G, const Tables& t, const u64* ro, u32* dst, u32* w, int sms,
+                               cudaStream_t s) {
+  if (t.rows == 0) return cudaSuccess;
+  u64 blocks = (t.rows * G + 255) / 256;
+  if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  switch (G) {
+    case 2: k_export_fill<2><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+    case 4: k_export_fill<4><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+    case 8: k_export_fill<8><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+// --------------------------------------------------------------- statistics ----
+template <int G>
+__global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  unsigned long long nbase = 0, linked = 0, live = 0, tombs = 0, maxc = 0;
+  for (u64 row = gid; row < t.rows; row += ng) {
+    const DirEntry de = t.dir[row];
+    nbase += de.nb;
+    for (u32 k = 0; k < de.nb; ++k) {
+      u32 b = de.base + k;
+      unsigned long long len = 0;
+      while (b != kNil) {
+        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
+        const bool l0 = q.x < kTomb, l1 = !g.last() && q.z < kTomb;
+        const bool t0 = q.x == kTomb, t1 = !g.last() && q.z == kTomb;
+        live += __popc(g.ballot(l0)) + __popc(g.ballot(l1));
+        tombs += __popc(g.ballot(t0)) + __popc(g.ballot(t1));
+        ++len;
+        b = g.shfl(q.z, G - 1);
+      }
+      linked += len;
+      if (len > maxc) maxc = len;
+    }
+  }
+  if (g.gl == 0) {
+    atomicAdd(&out->base_buckets, nbase);
+    atomicAdd(&out->linked_buckets, linked);
+    atomicAdd(&out->live, live);
+    atomicAdd(&out->tombs, tombs);
+    atomicMax(&out->max_chain, maxc);
+  }
+}
+
+cudaError_t launch_stats(int G, const Tables& t, StatsOut* out, int sms, cudaStream_t s) {
+  cudaError_t e = cudaMemsetAsync(out, 0, sizeof(StatsOut), s);
+  if (e != cudaSuccess || t.rows == 0) return e;
+  u64 blocks = (t.rows * G + 255) / 256;
+  if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  switch (G) {
+    case 2: k_stats<2><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+    case 4: k_stats<4><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+    case 8: k_stats<8><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+// ------------------------------------------------------- vertex deletion (a9) ----
+// Mark the batch in a |V|-bit bitmap D (all ranks mark every deleted ID, since
+// incoming edges may live on any shard), validate it (Q7/Q11), and list each
+// distinct ID owned by this rank once (duplicates are idempotent).
+__global__ void k_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
+                            DevCtl* ctl, u32 nranks, u32 rank) {
+  bool bad = false;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
+    const u32 id = ids[i];
+    if ((u64)id >= nv) {
+      bad = true;
+      continue;
+    }
+    const u32 bit = 1u << (id & 31);
+    const u32 old = atomicOr(&bitmap[id >> 5], bit);
+    if (!(old & bit) && id % nranks == rank) dedup[atomicAdd(&ctl->dedup_count, 1u)] = id;
+  }
+  if (__any_sync(0xFFFFFFFFu, bad) && (threadIdx.x & 31) == 0) atomicMax(&ctl->fail_epoch, epoch);
+}
+
+cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
+                             DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s) {
+  if (n == 0) return cudaSuccess;
+  u64 blocks = (n + 255) / 256;
+  if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  k_vdel_mark<<<(unsigned)blocks, 256, 0, s>>>(ids, n, nv, epoch, bitmap, dedup, ctl, nranks, rank);
+  return cudaGetLastError();
+}
+
+// Directed purge ("a follow-up lookup and delete of all deleted
+// vertices in all hash tables"): one streaming pass over every allocated bucket
+// of the pool (coalesced, G lanes per bucket); every live key in D becomes a
+// tombstone and the owner row's degree drops by one.
+template <int G>
+__global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
+                                                    u32 epoch) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
+  const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  for (u64 b = gid; b < nbk; b += ng) {
+    u32* bp = t.pool + b * W + 4 * g.gl;
+    const uint4 q = *reinterpret_cast<const uint4*>(bp);
+    const u32 owner = g.shfl(q.w, G - 1);
+    const bool h0 = q.x < kTomb && ((__ldg(bitmap + (q.x >> 5)) >> (q.x & 31)) & 1u);
+    const bool h1 = !g.last() && q.z < kTomb && ((__ldg(bitmap + (q.z >> 5)) >> (q.z & 31)) & 1u);
+    u32 dec = 0;
+    if (h0 && atomicCAS(bp, q.x, kTomb) == q.x) ++dec;
+    if (h1 && atomicCAS(bp + 2, q.z, kTomb) == q.z) ++dec;
+    if (dec) atomicSub(&t.dir[owner].deg, dec);
+  }
+}
+
+cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epoch, int sms,
+                              cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (G) {
+    case 2: k_vdel_sweep<2><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+    case 4: k_vdel_sweep<4><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+    case 8: k_vdel_sweep<8><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+// probe used by the undirected purge: delete key v from the table starting at b
+template <int G>
+__device__ __forceinline__ int purge_delete(const Tables& t, const Group<G>& g, u32 b, u32 v) {
+  constexpr int W = Group<G>::W;
+  while (true) {
+    u32* bp = t.pool + (u64)b * W;
+    const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
+    const bool lastl = g.last();
+    const bool m0 = q.x == v, m1 = !lastl && q.z == v;
+    const u32 hit = g.ballot(m0 || m1);
+    if (hit) {
+      const u32 l = __ffs(hit) - 1;
+      u32 old = 0;
+      if (g.gl == l) old = atomicCAS(bp + 4 * g.gl + (m0 ? 0 : 2), v, kTomb);
+      return g.shfl(old, l) == v ? 1 : 0;
+    }
+    const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
+    if (g.ballot(e0 || e1)) return 0;
+    const u32 next = g.shfl(q.z, G - 1);
+    if (next == kNil) return 0;
+    b = next;
+  }
+}
+
+// Undirected purge, Alg. 2: a group takes the next deleted
+// vertex u from an atomic queue (Alg2:L3-6), iterates over A_u (L11-12) and
+// deletes u from A_v of every neighbour v (L13-17).  Valid only for graphs kept
+// symmetric (directed = 0, single rank).
+template <int G>
+__global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* dedup, u32 epoch) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
+  const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
+  while (true) {
+    u32 qi = 0;
+    if (g.gl == 0) qi = atomicAdd(&t.ctl->queue, 1u);
+    qi = g.shfl(qi, 0);
+    if (qi >= cnt) break;
+    const u32 u = dedup[qi];
+    const DirEntry de = t.dir[u];
+    for (u32 k = 0; k < de.nb; ++k) {
+      u32 b = de.base + k;
+      while (b != kNil) {
+        const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
+        u32 lm0 = g.ballot(q.x < kTomb);
+        u32 lm1 = g.ballot(!g.last() && q.z < kTomb);
+        while (lm0 | lm1) {
+          const u32 l = __ffs(lm0 | lm1) - 1;
+          const bool s0 = (lm0 >> l) & 1u;
+          const u32 x0 = g.shfl(q.x, l), x1 = g.shfl(q.z, l);
+          const u32 v = s0 ? x0 : x1;
+          if (s0) lm0 &= ~(1u << l);
+          else lm1 &= ~(1u << l);
+          const DirEntry dv = t.dir[v];
+          if (purge_delete<G>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
+            atomicSub(&t.dir[v].deg, 1u);
+        }
+        b = g.shfl(q.z, G - 1);
+      }
+    }
+  }
+}
+
+cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
+                                  cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (G) {
+    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+// Owner clear (Alg2:L18-22): walk A_u; chained buckets are reset to EMPTY and
+// pushed on the free stack (dynamic memory reclaimed); base buckets
+// are reset to EMPTY in place (Q9: static memory is kept but must not keep stale
+// keys); degree := 0.
+template <int G>
+__global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, u32 epoch) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
+  const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
+  const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+  while (true) {
+    u32 qi = 0;
+    if (g.gl == 0) qi = atomicAdd(&t.ctl->queue, 1u);
+    qi = g.shfl(qi, 0);
+    if (qi >= cnt) break;
+    const u32 row = dedup[qi] / t.nranks;
+    const DirEntry de = t.dir[row];
+    for (u32 k = 0; k < de.nb; ++k) {
+      u32 b = de.base + k;
+      bool base_bucket = true;
+      while (b != kNil) {
+        u32* bp = t.pool + (u64)b * W + 4 * g.gl;
+        const uint4 q = ld_relaxed_v4(bp);
+        const u32 next = g.shfl(q.z, G - 1);
+        if (g.last()) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
+        else st_v4(bp, empty4);
+        if (!base_bucket && g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
+        base_bucket = false;
+        b = next;
+      }
+    }
+    if (g.gl == 0) t.dir[row].deg = 0;
+  }
+}
+
+cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
+                              cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (G) {
+    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    default: return cudaErrorInvalidValue;
+  }
+  return cudaGetLastError();
+}
+
+}  // namespace dg

@@ -1,0 +1,263 @@
+"""Python handle over the C ABI (include/dg.h).  Argument marshalling only: every
+step of the path runs in libdg.so's sm_100a kernels.
+
+Arrays may be CUDA torch tensors (the calls are then stream-ordered and return
+immediately, like the C ABI with device buffers), CPU torch tensors or numpy arrays
+(host buffers: the library stages them and the call is synchronous).  IDs and
+weights are 32-bit (uint32 or int32 bit patterns).
+"""
+from __future__ import annotations
+
+import ctypes
+
+import numpy as np
+import torch
+
+from . import _lib
+from ._lib import DGError, check, dg_config, dg_stats, lib
+
+_U32_OK = (torch.int32, torch.uint32)
+
+
+def _ptr(a, n_expected=None, dtype_bytes=4, what="array"):
+    """-> (pointer int, length, is_cuda)"""
+    if a is None:
+        return None, 0, False
+    if isinstance(a, torch.Tensor):
+        if a.element_size() != dtype_bytes:
+            raise TypeError(f"{what}: expected {dtype_bytes}-byte elements, got {a.dtype}")
+        if not a.is_contiguous():
+            raise ValueError(f"{what}: tensor must be contiguous")
+        n = a.numel()
+        p = a.data_ptr() if n else None
+        return p, n, a.is_cuda
+    arr = np.asarray(a)
+    if arr.dtype.itemsize != dtype_bytes or not arr.flags.c_contiguous:
+        raise TypeError(f"{what}: expected a contiguous {dtype_bytes}-byte numpy array")
+    n = arr.size
+    return (arr.ctypes.data if n else None), n, False
+
+
+def _as_u32(a):
+    """torch tensors pass through (int32/uint32); anything else becomes contiguous uint32 numpy."""
+    if a is None:
+        return None
+    if isinstance(a, torch.Tensor):
+        if a.dtype not in _U32_OK:
+            raise TypeError(f"expected int32/uint32 tensor, got {a.dtype}")
+        return a.contiguous()
+    return np.ascontiguousarray(np.asarray(a).astype(np.uint32, copy=False))
+
+
+def _stream(stream):
+    if stream is not None:
+        return stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+    if torch.cuda.is_available():
+        return torch.cuda.current_stream().cuda_stream
+    return 0
+
+
+class Graph:
+    """A dynamic graph: one hash table per vertex (§III-IV).
+
+    Parameters mirror ``dg_config`` (include/dg.h).  ``degree_hints`` (length
+    ``num_vertices``) sizes each vertex's initial table; ``None`` gives
+    every vertex one bucket.
+    """
+
+    def __init__(self, num_vertices: int, degree_hints=None, *, load_factor: float = 0.7,
+                 bucket_bytes: int = 128, directed: bool = True, pool_bytes: int = 0,
+                 device: int | None = None, rank: int = 0, nranks: int = 1,
+                 nccl_unique_id: bytes | None = None, stream=None):
+        cfg = dg_config()
+        lib.dg_config_init(ctypes.byref(cfg))
+        cfg.load_factor = float(load_factor)
+        cfg.bucket_bytes = int(bucket_bytes)
+        cfg.directed = 1 if directed else 0
+        cfg.pool_bytes = int(pool_bytes)
+        if device is None:
+            device = torch.cuda.current_device() if torch.cuda.is_available() else -1
+        cfg.device = int(device)
+        cfg.rank = int(rank)
+        cfg.nranks = int(nranks)
+        self._uid = None
+        if nccl_unique_id is not None:
+            self._uid = ctypes.create_string_buffer(bytes(nccl_unique_id), 128)
+            cfg.nccl_unique_id = ctypes.cast(self._uid, ctypes.c_void_p)
+        hints = _as_u32(degree_hints)
+        hp, hn, _ = _ptr(hints, what="degree_hints")
+        if hints is not None and hn != num_vertices:
+            raise ValueError("degree_hints must have num_vertices entries")
+        self.device = torch.device("cuda", int(device)) if device >= 0 else None
+        self._h = ctypes.c_void_p()
+        self.directed = directed
+        self.bucket_bytes = bucket_bytes
+        self.rank, self.nranks = rank, nranks
+        check(lib.dg_create(ctypes.byref(cfg), int(num_vertices), hp, _stream(stream),
+                            ctypes.byref(self._h)), "dg_create")
+
+    # ------------------------------------------------------------------ admin --
+    def close(self):
+        if getattr(self, "_h", None) and self._h.value:
+            lib.dg_destroy(self._h)
+            self._h = ctypes.c_void_p()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *exc):
+        self.close()
+
+    @property
+    def handle(self):
+        return self._h
+
+    @property
+    def num_vertices(self) -> int:
+        nv = ctypes.c_uint64()
+        check(lib.dg_num_vertices(self._h, ctypes.byref(nv), None))
+        return nv.value
+
+    @property
+    def local_rows(self) -> int:
+        r = ctypes.c_uint64()
+        check(lib.dg_num_vertices(self._h, None, ctypes.byref(r)))
+        return r.value
+
+    # ------------------------------------------------------------ edge batches --
+    def insert_edges(self, src, dst, weight=None, *, count: bool = False, stream=None):
+        """Alg. 1.  Returns the number of new keys if ``count``."""
+        src, dst, weight = _as_u32(src), _as_u32(dst), _as_u32(weight)
+        ps, n, _ = _ptr(src, what="src")
+        pd, nd, _ = _ptr(dst, what="dst")
+        pw, nw, _ = _ptr(weight, what="weight")
+        if nd != n or (weight is not None and nw != n):
+            raise ValueError("src/dst/weight lengths differ")
+        out = ctypes.c_uint64(0)
+        check(lib.dg_insert_edges(self._h, ps, pd, pw, n, ctypes.byref(out) if count else None,
+                                  _stream(stream)), "dg_insert_edges")
+        return out.value if count else None
+
+    def delete_edges(self, src, dst, *, count: bool = False, stream=None):
+        """Delete by key.  Returns the number removed if ``count``."""
+        src, dst = _as_u32(src), _as_u32(dst)
+        ps, n, _ = _ptr(src, what="src")
+        pd, nd, _ = _ptr(dst, what="dst")
+        if nd != n:
+            raise ValueError("src/dst lengths differ")
+        out = ctypes.c_uint64(0)
+        check(lib.dg_delete_edges(self._h, ps, pd, n, ctypes.byref(out) if count else None,
+                                  _stream(stream)), "dg_delete_edges")
+        return out.value if count else None
+
+    def query_edges(self, src, dst, *, weights: bool = True, found_out=None, weight_out=None,
+                    stream=None):
+        """edgeExist -> (found uint8, weight uint32 or None)."""
+        src, dst = _as_u32(src), _as_u32(dst)
+        ps, n, cuda = _ptr(src, what="src")
+        pd, nd, _ = _ptr(dst, what="dst")
+        if nd != n:
+            raise ValueError("src/dst lengths differ")
+        if found_out is None:
+            if cuda:
+                found_out = torch.empty(n, dtype=torch.uint8, device=src.device)
+                if weights:
+                    weight_out = torch.empty(n, dtype=torch.uint32, device=src.device)
+            else:
+                found_out = np.empty(n, np.uint8)
+                if weights:
+                    weight_out = np.empty(n, np.uint32)
+        pf, _, _ = _ptr(found_out, dtype_bytes=1, what="found")
+        pw, _, _ = _ptr(weight_out, what="weight_out")
+        check(lib.dg_query_edges(self._h, ps, pd, n, pf, pw, _stream(stream)), "dg_query_edges")
+        return found_out, weight_out
+
+    # --------------------------------------------------------- vertex batches --
+    def insert_vertices(self, ids, degree_hints=None, stream=None):
+        ids, hints = _as_u32(ids), _as_u32(degree_hints)
+        pi, n, _ = _ptr(ids, what="ids")
+        ph, nh, _ = _ptr(hints, what="degree_hints")
+        if hints is not None and nh != n:
+            raise ValueError("ids/degree_hints lengths differ")
+        check(lib.dg_insert_vertices(self._h, pi, n, ph, _stream(stream)), "dg_insert_vertices")
+
+    def delete_vertices(self, ids, stream=None):
+        ids = _as_u32(ids)
+        pi, n, _ = _ptr(ids, what="ids")
+        check(lib.dg_delete_vertices(self._h, pi, n, _stream(stream)), "dg_delete_vertices")
+
+    # ------------------------------------------------------------------ reads --
+    def export(self, device: bool = True, stream=None):
+        """Adjacency lists of the local rows as CSR (row_offsets u64, dst u32, w u32).
+        Rows are unsorted within themselves."""
+        rows = self.local_rows
+        m = ctypes.c_uint64()
+        st = _stream(stream)
+        if device and self.device is not None:
+            ro = torch.empty(rows + 1, dtype=torch.uint64, device=self.device)
+            pro = ro.data_ptr()
+        else:
+            ro = np.empty(rows + 1, np.uint64)
+            pro = ro.ctypes.data
+        check(lib.dg_export_adjacency(self._h, pro, None, None, 0, ctypes.byref(m), st),
+              "dg_export_adjacency")
+        n = m.value
+        if device and self.device is not None:
+            d = torch.empty(max(n, 1), dtype=torch.uint32, device=self.device)
+            w = torch.empty(max(n, 1), dtype=torch.uint32, device=self.device)
+            pd, pw = d.data_ptr(), w.data_ptr()
+        else:
+            d = np.empty(max(n, 1), np.uint32)
+            w = np.empty(max(n, 1), np.uint32)
+            pd, pw = d.ctypes.data, w.ctypes.data
+        check(lib.dg_export_adjacency(self._h, pro, pd, pw, max(n, 1), ctypes.byref(m), st),
+              "dg_export_adjacency")
+        return ro, d[:n], w[:n]
+
+    def export_numpy(self):
+        ro, d, w = self.export(device=False)
+        return ro, d, w
+
+    def degrees(self, device: bool = True, stream=None):
+        rows = self.local_rows
+        if device and self.device is not None:
+            out = torch.empty(max(rows, 1), dtype=torch.uint32, device=self.device)
+            p = out.data_ptr()
+        else:
+            out = np.empty(max(rows, 1), np.uint32)
+            p = out.ctypes.data
+        check(lib.dg_degrees(self._h, p, _stream(stream)), "dg_degrees")
+        return out[:rows]
+
+    def stats(self, stream=None) -> dict:
+        s = dg_stats()
+        check(lib.dg_get_stats(self._h, ctypes.byref(s), _stream(stream)), "dg_get_stats")
+        return {name: getattr(s, name) for name, _ in dg_stats._fields_}
+
+    def batch_status(self, stream=None) -> int:
+        """0, or DG_ERR_VERTEX_OUT_OF_RANGE if an async batch since the last call was rejected."""
+        st = lib.dg_batch_status(self._h, _stream(stream))
+        if st not in (_lib.DG_OK, _lib.DG_ERR_VERTEX_OUT_OF_RANGE):
+            check(st, "dg_batch_status")
+        return st
+
+    def triangle_count(self, stream=None) -> int:
+        c = ctypes.c_uint64()
+        check(lib.dg_triangle_count(self._h, ctypes.byref(c), _stream(stream)),
+              "dg_triangle_count")
+        return c.value
+
+
+def get_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    check(lib.dg_get_unique_id(buf), "dg_get_unique_id")
+    return buf.raw
+
+
+__all__ = ["Graph", "DGError", "get_unique_id"]

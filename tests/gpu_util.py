@@ -1,0 +1,76 @@
+"""Helpers shared by the GPU parity tests (-m gpu)."""
+from __future__ import annotations
+
+import numpy as np
+import torch
+
+from oracle import Oracle
+from oracle.compare import Candidates, check_invariants, compare_export, compare_queries
+
+
+def cuda(a):
+    if a is None:
+        return None
+    return torch.from_numpy(np.ascontiguousarray(a, np.uint32)).to("cuda")
+
+
+class GpuAdapter:
+    """Oracle-shaped facade over the CUDA path (for the golden-script runner)."""
+
+    def __init__(self, n, directed=True, **kw):
+        from paper_conf_ipps_awadapo20_b200 import Graph
+        self.g = Graph(n, directed=directed, **kw)
+
+    def _call(self, fn, *a, **k):
+        from paper_conf_ipps_awadapo20_b200 import DGError
+        try:
+            return 0, fn(*a, **k)
+        except DGError as e:
+            return e.status, 0
+
+    def insert_edges(self, s, d, w=None):
+        return self._call(self.g.insert_edges, cuda(s), cuda(d), cuda(w), count=True)
+
+    def delete_edges(self, s, d):
+        return self._call(self.g.delete_edges, cuda(s), cuda(d), count=True)
+
+    def query_edges(self, s, d):
+        f, w = self.g.query_edges(cuda(s), cuda(d))
+        st = self.g.batch_status()
+        return st, f.cpu().numpy(), w.cpu().numpy()
+
+    def delete_vertices(self, ids):
+        self.g.delete_vertices(cuda(ids))
+        return self.g.batch_status()
+
+    def insert_vertices(self, ids):
+        st, _ = self._call(self.g.insert_vertices, cuda(ids))
+        return st
+
+    def export(self):
+        ro, d, w = self.g.export()
+        return ro.cpu().numpy(), d.cpu().numpy(), w.cpu().numpy()
+
+
+def check_against_oracle(g, o: Oracle, where=""):
+    """Full export + degree + invariant comparison of a Graph with the oracle."""
+    ro, d, w = g.export()
+    ro, d, w = ro.cpu().numpy(), d.cpu().numpy(), w.cpu().numpy()
+    ref = o.export()
+    cand = Candidates(*o.candidates())
+    errs = compare_export((ro, d, w), ref, cand)
+    assert not errs, f"{where}: {errs}"
+    deg = g.degrees().cpu().numpy()
+    assert np.array_equal(deg, o.degrees()), f"{where}: degrees differ"
+    errs = check_invariants(ro, d, deg)
+    assert not errs, f"{where}: {errs}"
+    return cand
+
+
+def check_queries(g, o: Oracle, qs, qd, cand=None, where=""):
+    f, w = g.query_edges(cuda(qs), cuda(qd))
+    st, rf, rw = o.query_edges(qs, qd)
+    if cand is None:
+        cand = Candidates(*o.candidates())
+    errs = compare_queries(qs, qd, f.cpu().numpy(), w.cpu().numpy(), rf, rw, cand)
+    assert not errs, f"{where}: {errs}"

@@ -1,0 +1,291 @@
+"""GPU-vs-oracle parity through the C ABI (-m gpu).
+
+Bit-exact on exports (canonicalised), degrees, counts and query answers; a key
+duplicated inside its most recent insert batch may hold any of that batch's
+weights for it (Q1).  Sizes span many warp tiles with ragged tails.
+"""
+import os
+import subprocess
+import sys
+
+import numpy as np
+import pytest
+import torch
+
+import workloads as wl
+from oracle import Oracle
+from tests.golden_script import load, run_script
+from tests.gpu_util import GpuAdapter, check_against_oracle, check_queries, cuda
+
+pytestmark = pytest.mark.gpu
+
+GEOMS = [32, 64, 128]
+
+
+@pytest.fixture(autouse=True)
+def _dev(cuda_ok):
+    torch.cuda.set_device(0)
+    yield
+    torch.cuda.synchronize()
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("name", ["edge_ops_directed.txt", "edge_ops_undirected.txt"])
+def test_golden_scripts_on_gpu(name, bb):
+    run_script(load(name), lambda n, directed: GpuAdapter(n, directed, bucket_bytes=bb))
+
+
+def _config1_stream(bb, hints, directed, seed=1):
+    """Config 1 (BASELINE.json configs[0]; SURVEY §8(d) cfg 1): |V| = 1,024;
+    16 insert batches of 1,024 (5% forced intra-batch duplicates with distinct
+    weights), queries, deletes, vertex deletions, re-insertion, growth and an
+    out-of-range batch — compared with the oracle after every batch."""
+    from paper_conf_ipps_awadapo20_b200 import DGError, DG_ERR_VERTEX_OUT_OF_RANGE, Graph
+    nv = 1024
+    hint = wl.out_degrees(wl.uniform_edges(seed, 0, 16 * 1024, nv)[0], nv) if hints else None
+    g = Graph(nv, hint, bucket_bytes=bb, directed=directed)
+    o = Oracle(nv, directed)
+    stream = 1000
+    for b in range(16):
+        s, d, w = wl.uniform_edges(seed, stream + b, 1024, nv)
+        k = 51  # 5%: repeat earlier keys of the same batch with distinct weights
+        s[-k:], d[-k:] = s[:k], d[:k]
+        st, added = o.insert_edges(s, d, w)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
+        cand = check_against_oracle(g, o, f"insert batch {b}")
+        # queries: half live (from the oracle's export), half uniform
+        ro, dd, _ = o.export()
+        rows = np.repeat(np.arange(nv, dtype=np.uint32), np.diff(ro).astype(np.int64))
+        pick = wl.uniform_index(seed, 5000 + b, 512, max(dd.size, 1))
+        qs = np.concatenate([rows[pick], wl.uniform_edges(seed, 6000 + b, 512, nv)[0]])
+        qd = np.concatenate([dd[pick], wl.uniform_edges(seed, 6000 + b, 512, nv)[1]])
+        check_queries(g, o, qs, qd, cand, f"query batch {b}")
+    for b in range(4):
+        ro, dd, _ = o.export()
+        rows = np.repeat(np.arange(nv, dtype=np.uint32), np.diff(ro).astype(np.int64))
+        pick = wl.uniform_index(seed, 7000 + b, 512, dd.size)
+        us, ud, _ = wl.uniform_edges(seed, 8000 + b, 512, nv)
+        s = np.concatenate([rows[pick], us]); d = np.concatenate([dd[pick], ud])
+        assert g.delete_edges(cuda(s), cuda(d), count=True) == o.delete_edges(s, d)[1]
+        check_against_oracle(g, o, f"delete batch {b}")
+    for b in range(4):
+        ids = wl.uniform_u32(seed, 9000 + b, 16, nv)
+        g.delete_vertices(cuda(ids))
+        assert g.batch_status() == 0
+        o.delete_vertices(ids)
+        check_against_oracle(g, o, f"vertex deletion {b}")
+        # re-insert edges touching the deleted IDs (vertex re-insertion)
+        s, d, w = wl.uniform_edges(seed, 9500 + b, 256, nv)
+        s[:128] = ids[np.arange(128) % ids.size]
+        d[128:] = ids[np.arange(128) % ids.size]
+        st, added = o.insert_edges(s, d, w)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
+        check_against_oracle(g, o, f"re-insert {b}")
+    # growth: vertex insertion 1024..1279, then 1,024 edges over [0, 1280)
+    new = np.arange(1024, 1280, dtype=np.uint32)
+    g.insert_vertices(cuda(new), cuda(np.full(new.size, 20, np.uint32)))
+    o.insert_vertices(new)
+    assert g.num_vertices == 1280
+    s, d, w = wl.uniform_edges(seed, 9900, 1024, 1280)
+    st, added = o.insert_edges(s, d, w)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
+    check_against_oracle(g, o, "after growth")
+    # out-of-range batch: rejected, graph unchanged (Q7)
+    s, d, w = wl.uniform_edges(seed, 9901, 1024, 1280)
+    s[500] = 1280
+    with pytest.raises(DGError) as e:
+        g.insert_edges(cuda(s), cuda(d), cuda(w), count=True)
+    assert e.value.status == DG_ERR_VERTEX_OUT_OF_RANGE
+    with pytest.raises(DGError):
+        g.delete_edges(cuda(s), cuda(d), count=True)
+    g.delete_vertices(cuda(np.array([5, 5000], np.uint32)))
+    assert g.batch_status() == DG_ERR_VERTEX_OUT_OF_RANGE
+    check_against_oracle(g, o, "after rejected batches")
+    st = g.stats()
+    assert st["live_pairs"] == o.num_edges()
+    g.close()
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("hints", [False, True])
+def test_config1_directed(bb, hints):
+    _config1_stream(bb, hints, True)
+
+
+@pytest.mark.parametrize("bb", [32, 128])
+def test_config1_undirected(bb):
+    _config1_stream(bb, False, False, seed=3)
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+def test_large_random_ragged(bb):
+    """|V| = 100,000; 3 insert batches of 700,001 (ragged tail), queries, deletes."""
+    nv = 100_000
+    g = __import__("paper_conf_ipps_awadapo20_b200").Graph(nv, bucket_bytes=bb)
+    o = Oracle(nv)
+    for b in range(3):
+        s, d, w = wl.uniform_edges(11, b, 700_001, nv)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+    cand = check_against_oracle(g, o, "inserted")
+    qs, qd, _ = wl.uniform_edges(11, 50, 300_007, nv)
+    s, d, _ = wl.uniform_edges(11, 1, 300_007, nv)  # live keys from batch 1
+    check_queries(g, o, np.concatenate([qs, s]), np.concatenate([qd, d]), cand, "queries")
+    assert g.delete_edges(cuda(s), cuda(d), count=True) == o.delete_edges(s, d)[1]
+    check_against_oracle(g, o, "deleted")
+
+
+@pytest.mark.parametrize("bb", [32, 128])
+def test_rmat_hubs_without_hints(bb):
+    """Scale-free input with one bucket per vertex (Tab. VI-style incremental build):
+    long chains, many concurrent chain extensions and same-key races."""
+    scale = 16
+    nv = 1 << scale
+    s, d = wl.rmat_edges(5, 0, 1_000_000, scale, wl.GRAPH500)
+    w = wl.weights(5, 0, s.size)
+    g = __import__("paper_conf_ipps_awadapo20_b200").Graph(nv, bucket_bytes=bb, pool_bytes=1 << 20)
+    o = Oracle(nv)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+    cand = check_against_oracle(g, o, "rmat")
+    st = g.stats()
+    assert st["max_chain"] > 10 and st["live_pairs"] == o.num_edges()
+    check_queries(g, o, s[::7], d[::7], cand, "rmat queries")
+    # hub deletion frees chained buckets; re-insertion reuses them from the free stack
+    deg = np.bincount(s, minlength=nv)
+    hubs = np.argsort(deg)[-8:].astype(np.uint32)
+    g.delete_vertices(cuda(hubs))
+    o.delete_vertices(hubs)
+    check_against_oracle(g, o, "hubs deleted")
+    st2 = g.stats()
+    assert st2["free_buckets"] > 0
+    m = (np.isin(s, hubs))
+    assert g.insert_edges(cuda(s[m]), cuda(d[m]), cuda(w[m]), count=True) == \
+        o.insert_edges(s[m], d[m], w[m])[1]
+    check_against_oracle(g, o, "hubs re-inserted")
+    assert g.stats()["free_buckets"] < st2["free_buckets"]
+
+
+def test_heavy_intra_batch_duplicates():
+    nv = 64
+    s = np.full(50_000, 7, np.uint32)
+    d = (np.arange(50_000) % 5 + 1).astype(np.uint32)
+    w = np.arange(50_000, dtype=np.uint32)
+    g = __import__("paper_conf_ipps_awadapo20_b200").Graph(nv)
+    o = Oracle(nv)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1] == 5
+    check_against_oracle(g, o, "dups")
+    # deleting the same key many times removes it once
+    assert g.delete_edges(cuda(s), cuda(d), count=True) == 5
+
+
+def test_host_buffers_match_device_buffers():
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 5000
+    s, d, w = wl.uniform_edges(21, 0, 100_000, nv)
+    a, b = Graph(nv), Graph(nv)
+    assert a.insert_edges(s, d, w, count=True) == b.insert_edges(cuda(s), cuda(d), cuda(w), count=True)
+    qs, qd, _ = wl.uniform_edges(21, 1, 50_000, nv)
+    fa, wa = a.query_edges(qs, qd)
+    fb, wb = b.query_edges(cuda(qs), cuda(qd))
+    assert isinstance(fa, np.ndarray)
+    assert np.array_equal(fa, fb.cpu().numpy()) and np.array_equal(wa, wb.cpu().numpy())
+    ea, eb = a.export_numpy(), b.export()
+    assert np.array_equal(ea[0], eb[0].cpu().numpy())
+
+
+@pytest.mark.parametrize("directed", [True, False])
+def test_vertex_deletion_modes(directed):
+    """Directed: streaming purge sweep; undirected: Alg. 2."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 20_000
+    s, d = wl.rmat_edges(8, 0, 200_000, 15, wl.GRAPH500, nv=nv)
+    g = Graph(nv, directed=directed)
+    o = Oracle(nv, directed)
+    g.insert_edges(cuda(s), cuda(d))
+    o.insert_edges(s, d)
+    for r in range(3):
+        ids = np.concatenate([wl.uniform_u32(8, 100 + r, 300, nv), s[:5]])  # hubs + duplicates
+        g.delete_vertices(cuda(ids))
+        o.delete_vertices(ids)
+        check_against_oracle(g, o, f"round {r}")
+        qs = np.repeat(ids[:50], 40)
+        qd = wl.uniform_u32(8, 200 + r, qs.size, nv)
+        check_queries(g, o, np.concatenate([qs, qd]), np.concatenate([qd, qs]), None, "incident")
+
+
+def test_empty_batches():
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    g = Graph(10)
+    e = torch.empty(0, dtype=torch.uint32, device="cuda")
+    assert g.insert_edges(e, e, count=True) == 0
+    assert g.delete_edges(e, e, count=True) == 0
+    f, w = g.query_edges(e, e)
+    assert f.numel() == 0
+    g.delete_vertices(e)
+    g.insert_vertices(e)
+    ro, d, w = g.export()
+    assert d.numel() == 0 and ro.numel() == 11
+    g0 = Graph(0)
+    assert g0.export()[1].numel() == 0
+
+
+def test_geometry_invariance():
+    """Deterministic weights -> identical exports across bucket size, load factor and
+    hints (hints/load factor affect only performance)."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 30_000
+    s, d = wl.rmat_edges(9, 0, 400_000, 15, wl.LJLIKE, nv=nv)
+    w = (s.astype(np.uint64) * 2654435761 ^ d).astype(np.uint32)  # equal weights for equal keys
+    hint = wl.out_degrees(s, nv)
+    ref = None
+    for bb in GEOMS:
+        for lf in (0.35, 0.7, 2.0):
+            for h in (None, hint):
+                g = Graph(nv, h, bucket_bytes=bb, load_factor=lf)
+                g.insert_edges(cuda(s), cuda(d), cuda(w))
+                g.delete_edges(cuda(s[::3]), cuda(d[::3]))
+                ro, dd, ww = g.export()
+                from oracle.compare import canonical
+                out = canonical(ro.cpu().numpy(), dd.cpu().numpy(), ww.cpu().numpy())
+                if ref is None:
+                    ref = out
+                else:
+                    assert all(np.array_equal(a, b) for a, b in zip(ref, out)), (bb, lf, h is None)
+                g.close()
+
+
+def test_initial_bucket_rule_matches_oracle():
+    """dg_create's base-bucket count equals the paper's closed form
+    as computed by the oracle, for every vertex."""
+    from oracle import initial_buckets
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    hints = np.array([0, 1, 10, 11, 100, 105, 106, 1000, 20000, 7, 3], np.uint32)
+    for bb, bc in ((128, 15), (64, 7), (32, 3)):
+        for lf in (0.7, 0.5, 1.0):
+            g = Graph(hints.size, hints, bucket_bytes=bb, load_factor=lf)
+            want = sum(initial_buckets(int(h), int(round(lf * 1000)), bc) for h in hints)
+            assert g.stats()["base_buckets"] == want
+
+
+def test_pool_exhaustion_retry_path():
+    """Pool exhaustion mid-kernel: failed ops are re-run after the pool grows
+    (forced with DG_TEST_RETRY_PATH, which disables up-front growth)."""
+    code = r"""
+import numpy as np, torch, sys
+sys.path.insert(0, %r)
+import workloads as wl
+from oracle import Oracle
+from tests.gpu_util import check_against_oracle, cuda
+from paper_conf_ipps_awadapo20_b200 import Graph
+nv = 4096
+g = Graph(nv, pool_bytes=4096)
+o = Oracle(nv)
+for b in range(3):
+    s, d, w = wl.uniform_edges(2, b, 400_000, nv)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+check_against_oracle(g, o, "retry")
+print("OK", g.stats()["pool_buckets"])
+""" % os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, DG_TEST_RETRY_PATH="1")
+    r = subprocess.run([sys.executable, "-c", code], env=env, capture_output=True, text=True,
+                       timeout=600)
+    assert r.returncode == 0 and "OK" in r.stdout, r.stderr[-3000:]
