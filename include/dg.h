@@ -89,10 +89,16 @@ typedef struct dg_config {
   int32_t device;         /* CUDA device ordinal; -1 = current device */
   int32_t rank;           /* this process's rank, 0 <= rank < nranks */
   int32_t nranks;         /* number of GPUs the graph is sharded over (1 = single GPU) */
-  uint32_t reserved0;
+  uint32_t flags;         /* DG_FLAG_* bits, default 0 */
   const void* nccl_unique_id; /* 128-byte ncclUniqueId from dg_get_unique_id() on rank 0,
                                  broadcast by the caller; NULL when nranks == 1 */
 } dg_config;
+
+/* dg_config.flags: new keys are installed in the first tombstone of their chain by
+ * default (the two-stage insert the paper offers as an option; results
+ * are identical, chains stop growing under insert/delete churn).  This flag selects
+ * the paper's default append-only policy: tombstones are never reused. */
+#define DG_FLAG_NO_TOMBSTONE_REUSE 1u
 
 /* Memory / structure statistics (Fig. 2b/c quantities). */
 typedef struct dg_stats {
@@ -101,6 +107,7 @@ typedef struct dg_stats {
   uint64_t overflow_buckets;  /* chained buckets currently linked into tables */
   uint64_t free_buckets;      /* buckets on the free stack */
   uint64_t pool_buckets;      /* buckets mapped in the pool */
+  uint64_t bump_buckets;      /* high-water mark: buckets ever handed out (base + chained) */
   uint64_t live_pairs;        /* stored edges (sum of degrees) */
   uint64_t tombstones;        /* deleted-key slots not yet reclaimed */
   uint64_t max_chain;         /* longest bucket chain (in buckets) */
@@ -204,6 +211,22 @@ DG_API dg_status dg_batch_status(dg_graph g, void* stream);
  * triangle is counted once.  *count (host) receives the total; synchronises.
  * Requires nranks == 1 (multi-GPU triangle counting runs one replica per GPU). */
 DG_API dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream);
+
+/* ------------------------------------------------------------ instrumentation --
+ * Off by default; used by bench.py.  While enabled, every probe-kernel launch of an
+ * edge batch (and the purge kernels of a vertex-deletion batch) is bracketed by
+ * CUDA events on the call's stream. */
+typedef struct dg_profile {
+  uint64_t launches;          /* kernels launched by libdg in this process since enable */
+  uint64_t kernel_launches[4];/* timed launches: [0] insert, [1] delete, [2] query, [3] vertex purge */
+  double kernel_ms[4];        /* their summed device durations in ms */
+  uint64_t last_count;        /* n_added / n_removed of the most recent insert/delete batch */
+} dg_profile;
+
+/* enable != 0 starts (and resets) instrumentation; 0 stops it. */
+DG_API dg_status dg_profile_enable(dg_graph g, int enable);
+/* Reads the counters (synchronises `stream`). */
+DG_API dg_status dg_profile_read(dg_graph g, dg_profile* out, void* stream);
 
 #ifdef __cplusplus
 }

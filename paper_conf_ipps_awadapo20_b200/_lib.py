@@ -20,6 +20,7 @@ DG_ERR_CUDA = 4
 DG_ERR_NCCL = 5
 DG_ERR_BAD_STATE = 6
 DG_ERR_UNSUPPORTED = 7
+DG_FLAG_NO_TOMBSTONE_REUSE = 1
 
 VP = ctypes.c_void_p
 U64 = ctypes.c_uint64
@@ -37,7 +38,7 @@ class dg_config(ctypes.Structure):
         ("device", ctypes.c_int32),
         ("rank", ctypes.c_int32),
         ("nranks", ctypes.c_int32),
-        ("reserved0", ctypes.c_uint32),
+        ("flags", ctypes.c_uint32),
         ("nccl_unique_id", ctypes.c_void_p),
     ]
 
@@ -49,12 +50,22 @@ class dg_stats(ctypes.Structure):
         ("overflow_buckets", ctypes.c_uint64),
         ("free_buckets", ctypes.c_uint64),
         ("pool_buckets", ctypes.c_uint64),
+        ("bump_buckets", ctypes.c_uint64),
         ("live_pairs", ctypes.c_uint64),
         ("tombstones", ctypes.c_uint64),
         ("max_chain", ctypes.c_uint64),
         ("pool_bytes", ctypes.c_uint64),
         ("load_factor", ctypes.c_double),
         ("utilization", ctypes.c_double),
+    ]
+
+
+class dg_profile(ctypes.Structure):
+    _fields_ = [
+        ("launches", ctypes.c_uint64),
+        ("kernel_launches", ctypes.c_uint64 * 4),
+        ("kernel_ms", ctypes.c_double * 4),
+        ("last_count", ctypes.c_uint64),
     ]
 
 
@@ -76,6 +87,8 @@ SIGNATURES = [
     ("dg_get_stats", ctypes.c_int, [VP, ctypes.POINTER(dg_stats), VP]),
     ("dg_batch_status", ctypes.c_int, [VP, VP]),
     ("dg_triangle_count", ctypes.c_int, [VP, P_U64, VP]),
+    ("dg_profile_enable", ctypes.c_int, [VP, ctypes.c_int]),
+    ("dg_profile_read", ctypes.c_int, [VP, ctypes.POINTER(dg_profile), VP]),
 ]
 
 

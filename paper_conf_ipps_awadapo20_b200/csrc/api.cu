@@ -152,6 +152,17 @@ size_t device_free_bytes() {
 
 namespace dg {
 
+void prof_mark(dg_graph g, int k, cudaStream_t s) {
+  if (!g->prof) return;
+  cudaEvent_t e;
+  if (cudaEventCreate(&e) != cudaSuccess) {
+    cudaGetLastError();
+    return;
+  }
+  cudaEventRecord(e, s);
+  g->prof_ev[k].push_back(e);
+}
+
 // Map more pool memory so that at least min_buckets buckets exist; new buckets
 // are all-EMPTY (0xFF bytes: EMPTY keys/values, NIL next, NIL owner).
 dg_status grow_pool(dg_graph g, u64 min_buckets, cudaStream_t s) {
@@ -247,9 +258,12 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   a.idx = nullptr;
   a.n_ops = n_ops;
   a.retry_out = g->retry[0];
+  a.reuse_tombstones = g->reuse_tombstones ? 1u : 0u;
   a.epoch = epoch;
   a.nv = g->nv;
+  prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
+  prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_fixup_alloc(t, s));
   if (!retry_mode) {
     note_launch(g, need, s);
@@ -289,7 +303,9 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
   a.n_ops = n_ops;
   a.epoch = epoch;
   a.nv = g->nv;
+  prof_mark(g, PROF_DELETE, s);
   DG_CK(dg::launch_delete(g->G, g->tables(), a, g->sms, s));
+  prof_mark(g, PROF_DELETE, s);
   return DG_OK;
 }
 
@@ -305,7 +321,9 @@ dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t
   a.nv = g->nv;
   a.found = found;
   a.wout = wout;
+  prof_mark(g, PROF_QUERY, s);
   DG_CK(dg::launch_query(g->G, g->tables(), a, g->sms, s));
+  prof_mark(g, PROF_QUERY, s);
   return DG_OK;
 }
 
@@ -347,11 +365,19 @@ dg_status dg_get_unique_id(void* out128) {
   return dg::router_unique_id(out128);
 }
 
+static void prof_clear(dg_graph g) {
+  for (auto& v : g->prof_ev) {
+    for (cudaEvent_t e : v) cudaEventDestroy(e);
+    v.clear();
+  }
+}
+
 static void destroy_graph(dg_graph g) {
   if (!g) return;
   cudaSetDevice(g->device);
   cudaDeviceSynchronize();
   cudaGetLastError();
+  prof_clear(g);
   if (g->router) dg::router_destroy(g->router);
   g->dir.release();
   g->pool.release();
@@ -425,6 +451,7 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->flags & ~DG_FLAG_NO_TOMBSTONE_REUSE) return DG_ERR_INVALID_ARGUMENT;
 
   dg_graph g = new (std::nothrow) dg_graph_s();
   if (!g) return DG_ERR_OUT_OF_MEMORY;
@@ -451,6 +478,7 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   g->nranks = (u32)cfg->nranks;
   g->rank = (u32)cfg->rank;
   g->directed = cfg->directed != 0;
+  g->reuse_tombstones = (cfg->flags & DG_FLAG_NO_TOMBSTONE_REUSE) == 0;
   g->nv = num_vertices;
 
   const size_t total_mem = prop.totalGlobalMem;
@@ -676,6 +704,7 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
   DG_CK(dg::launch_vdel_mark(all_ids, all_n, g->nv, epoch, g->bitmap, g->dedup, g->ctl, g->nranks,
                              g->rank, g->sms, s));
   static const bool force_sweep = std::getenv("DG_FORCE_SWEEP") != nullptr;
+  dg::prof_mark(g, dg::PROF_VDEL, s);
   if (!g->directed && g->nranks == 1 && !force_sweep) {
     // undirected: Alg. 2 — delete u from the tables of its neighbours
     DG_CK(dg::launch_vdel_neighbors(g->G, t, g->dedup, epoch, g->sms, s));
@@ -685,6 +714,7 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
     DG_CK(dg::launch_vdel_sweep(g->G, t, g->bitmap, epoch, g->sms, s));
   }
   DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, epoch, g->sms, s));
+  dg::prof_mark(g, dg::PROF_VDEL, s);
   if (host) {
     if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
     g->snap_pending = false;
@@ -758,6 +788,7 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   out->overflow_buckets = h.linked_buckets - h.base_buckets;
   out->free_buckets = g->hctl->stack_size;
   out->pool_buckets = g->cap;
+  out->bump_buckets = g->hctl->bump;
   out->live_pairs = h.live;
   out->tombstones = h.tombs;
   out->max_chain = h.max_chain;
@@ -785,6 +816,38 @@ dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream) {
   (void)count;
   (void)stream;
   return DG_ERR_UNSUPPORTED;
+}
+
+dg_status dg_profile_enable(dg_graph g, int enable) {
+  DG_TRY(check_handle(g));
+  cudaDeviceSynchronize();
+  prof_clear(g);
+  g->prof = enable != 0;
+  g->prof_launch0 = dg::kernel_launches();
+  return DG_OK;
+}
+
+dg_status dg_profile_read(dg_graph g, dg_profile* out, void* stream) {
+  DG_TRY(check_handle(g));
+  if (!out) return DG_ERR_INVALID_ARGUMENT;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  std::memset(out, 0, sizeof(*out));
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  g->snap_pending = false;
+  DG_TRY(read_ctl(g, s));
+  for (int k = 0; k < 4; ++k) {
+    auto& v = g->prof_ev[k];
+    for (size_t i = 0; i + 1 < v.size(); i += 2) {
+      float ms = 0.f;
+      DG_CK(cudaEventSynchronize(v[i + 1]));
+      DG_CK(cudaEventElapsedTime(&ms, v[i], v[i + 1]));
+      out->kernel_ms[k] += ms;
+      out->kernel_launches[k] += 1;
+    }
+  }
+  out->launches = dg::kernel_launches() - g->prof_launch0;
+  out->last_count = g->hctl->count;
+  return DG_OK;
 }
 
 }  // extern "C"

@@ -70,17 +70,17 @@ __device__ __forceinline__ u32 bucket_of(u32 key, u32 nb) {
 }
 
 // ------------------------------------------------------------------ memory ----
+// 16-B loads are issued as v2.u64 so ptxas keeps ONE 128-bit load even when only
+// the key words are consumed (a v4.u32 with dead lanes is split into 32-bit loads).
 __device__ __forceinline__ uint4 ld_relaxed_v4(const u32* p) {
-  uint4 r;
-  asm volatile("ld.relaxed.gpu.global.v4.u32 {%0,%1,%2,%3}, [%4];"
-               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p) : "memory");
-  return r;
+  unsigned long long a, b;
+  asm volatile("ld.relaxed.gpu.global.v2.u64 {%0,%1}, [%2];" : "=l"(a), "=l"(b) : "l"(p) : "memory");
+  return make_uint4((u32)a, (u32)(a >> 32), (u32)b, (u32)(b >> 32));
 }
 __device__ __forceinline__ uint4 ld_nc_v4(const u32* p) {
-  uint4 r;
-  asm volatile("ld.global.nc.v4.u32 {%0,%1,%2,%3}, [%4];"
-               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
-  return r;
+  unsigned long long a, b;
+  asm volatile("ld.global.nc.v2.u64 {%0,%1}, [%2];" : "=l"(a), "=l"(b) : "l"(p));
+  return make_uint4((u32)a, (u32)(a >> 32), (u32)b, (u32)(b >> 32));
 }
 __device__ __forceinline__ uint4 ld_nc_dir(const DirEntry* p) {
   return ld_nc_v4(reinterpret_cast<const u32*>(p));

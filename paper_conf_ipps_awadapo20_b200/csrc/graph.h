@@ -2,6 +2,7 @@
 #pragma once
 #include <cstddef>
 #include <cstdint>
+#include <vector>
 
 #include <cuda_runtime.h>
 
@@ -24,6 +25,7 @@ struct dg_graph_s {
   uint32_t lf_milli = 700;
   uint32_t nranks = 1, rank = 0;
   bool directed = true;
+  bool reuse_tombstones = true;
 
   uint64_t nv = 0;        // global vertex capacity
   uint64_t rows = 0;      // local rows
@@ -59,6 +61,11 @@ struct dg_graph_s {
 
   dg::Router* router = nullptr;
 
+  // instrumentation (dg_profile_*)
+  bool prof = false;
+  uint64_t prof_launch0 = 0;
+  std::vector<cudaEvent_t> prof_ev[4];  // start/stop pairs per kernel kind
+
   dg::Tables tables() const {
     dg::Tables t;
     t.dir = reinterpret_cast<dg::DirEntry*>(dir.ptr());
@@ -78,6 +85,10 @@ namespace dg {
 inline uint64_t rows_for(uint64_t nv, uint32_t nranks, uint32_t rank) {
   return nv > rank ? (nv - rank + nranks - 1) / nranks : 0;
 }
+
+enum ProfKind { PROF_INSERT = 0, PROF_DELETE = 1, PROF_QUERY = 2, PROF_VDEL = 3 };
+// record an event of kind k on s if instrumentation is enabled
+void prof_mark(dg_graph g, int k, cudaStream_t s);
 
 // internal entry points shared by api.cu and router.cu
 dg_status grow_pool(dg_graph g, uint64_t min_buckets, cudaStream_t s);

@@ -9,6 +9,10 @@ namespace dg {
 
 constexpr int kEdgeBlock = 256;
 
+// process-wide count of kernels launched by the library (dg_profile.launches)
+void note_kernel(int n);
+uint64_t kernel_launches();
+
 struct EdgeBatch {
   const u32* src;
   const u32* dst;
@@ -21,6 +25,7 @@ struct EdgeBatch {
   u64 nv;             // global vertex capacity (query range check)
   uint8_t* found;     // query
   u32* wout;          // query, nullable
+  u32 reuse_tombstones;  // insert: install new keys in the first tombstone
 };
 
 // edge ops (kernels_edges.cu)

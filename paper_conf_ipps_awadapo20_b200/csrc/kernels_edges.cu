@@ -24,10 +24,16 @@
 //     and degrees stay exact (Alg1:L9-10);
 //   * degree updates are one fire-and-forget atomic per added/removed key; batch
 //     counters are reduced per warp.
+#include <atomic>
+
 #include "dg_common.cuh"
 #include "kernels.h"
 
 namespace dg {
+
+static std::atomic<unsigned long long> g_launches{0};
+void note_kernel(int n) { g_launches.fetch_add((unsigned long long)n, std::memory_order_relaxed); }
+uint64_t kernel_launches() { return g_launches.load(std::memory_order_relaxed); }
 
 enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 
@@ -43,11 +49,22 @@ __device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 stack_size) {
 }
 
 // ------------------------------------------------------------ probe: insert ----
+// Full chain walk from the head bucket b (slow path; the fast path in k_edges
+// handles single-bucket chains).  The key must be absent from the whole chain
+// before it is installed (uniqueness); it is installed with
+// a 64-bit CAS in the FIRST free slot of the chain: the first tombstone when
+// tombstones are reused (the paper's two-stage option), else the
+// first EMPTY.  Any failed slot CAS re-scans the chain from the head:
+// two inserts of one key then always contend for the same slot.
 // returns 1 = key added, 0 = existing key replaced, -1 = no bucket available
 template <int G>
-__device__ __forceinline__ int probe_insert(const Tables& t, const Group<G>& g, u32 row, u32 b,
-                                            u32 v, u32 w, u32& spare, u32 stack_size) {
+__device__ __forceinline__ int probe_insert(const Tables& t, const Group<G>& g, u32 row,
+                                            const u32 head, u32 v, u32 w, u32& spare,
+                                            u32 stack_size, bool reuse) {
   constexpr int W = Group<G>::W;
+  u32 b = head;
+  u32* ff = nullptr;         // first free slot seen (pair address), group-uniform
+  unsigned long long ffo = 0;  // its current contents
   while (true) {
     u32* bp = t.pool + (u64)b * W;
     const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
@@ -61,45 +78,58 @@ __device__ __forceinline__ int probe_insert(const Tables& t, const Group<G>& g, 
     }
     const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
     const u32 em = g.ballot(e0 || e1);
-    if (em) {  // first EMPTY slot of the chain: install (v, w)
-      const u32 l = __ffs(em) - 1;
-      const u32 woff = 4 * g.gl + (e0 ? 0 : 2);
-      unsigned long long old = 0;
-      if (g.gl == l)
-        old = atomicCAS(reinterpret_cast<unsigned long long*>(bp + woff), kEmptyPair,
-                        (unsigned long long)pack_pair(v, w));
-      old = g.shfl(old, l);
-      if (old == kEmptyPair) return 1;
-      if ((u32)old == v) {  // a racing op installed the same key: replace
-        if (g.gl == l) st_relaxed_u32(bp + woff + 1, w);
-        return 0;
+    if (!ff) {
+      const bool f0 = e0 || (reuse && q.x == kTomb);
+      const bool f1 = e1 || (reuse && !lastl && q.z == kTomb);
+      const u32 fm = g.ballot(f0 || f1);
+      if (fm) {
+        const u32 l = __ffs(fm) - 1;
+        const u64 addr = (u64)(bp + 4 * g.gl + (f0 ? 0 : 2));
+        const unsigned long long cur = f0 ? pack_pair(q.x, q.y) : pack_pair(q.z, q.w);
+        ff = reinterpret_cast<u32*>(g.shfl(addr, l));
+        ffo = g.shfl(cur, l);
       }
-      continue;  // slot taken by another key: re-read this bucket
     }
     const u32 next = g.shfl(q.z, G - 1);
-    if (next != kNil) {
-      b = next;
+    if (em || next == kNil) {
+      // end of the chain: the key is absent
+      if (ff) {
+        unsigned long long old = 0;
+        if (g.gl == 0)
+          old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
+                          (unsigned long long)pack_pair(v, w));
+        old = g.shfl(old, 0);
+        if (old == ffo) return 1;
+        if ((u32)old == v) {  // a racing op installed the same key there: replace
+          if (g.gl == 0) st_relaxed_u32(ff + 1, w);
+          return 0;
+        }
+        ff = nullptr;  // slot taken by another key: re-scan from the head
+        b = head;
+        continue;
+      }
+      // chain full: link a new bucket at the tail
+      if (spare == kNil) {
+        u32 s = 0;
+        if (g.gl == 0) s = alloc_bucket(t, stack_size);
+        spare = g.shfl(s, 0);
+        if (spare == kNil) return -1;
+      }
+      u32 old = 0;
+      if (lastl) {
+        st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
+        old = atomicCAS(bp + Group<G>::NEXT, kNil, spare);
+      }
+      old = g.shfl(old, G - 1);
+      if (old == kNil) {
+        b = spare;
+        spare = kNil;
+      } else {
+        b = old;  // another op linked first (earlier slots cannot free up); keep our spare
+      }
       continue;
     }
-    // chain full: link a new bucket at the tail
-    if (spare == kNil) {
-      u32 s = 0;
-      if (g.gl == 0) s = alloc_bucket(t, stack_size);
-      spare = g.shfl(s, 0);
-      if (spare == kNil) return -1;
-    }
-    u32 old = 0;
-    if (lastl) {
-      st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
-      old = atomicCAS(bp + Group<G>::NEXT, kNil, spare);
-    }
-    old = g.shfl(old, G - 1);
-    if (old == kNil) {
-      b = spare;
-      spare = kNil;
-    } else {
-      b = old;  // another op linked first; keep our spare for later
-    }
+    b = next;
   }
 }
 
@@ -152,21 +182,34 @@ __device__ __forceinline__ bool probe_query(const Tables& t, const Group<G>& g, 
 }
 
 // ------------------------------------------------------------- main kernel ----
+// Per warp iteration (32 ops):
+//   1. lane L stages op L (coalesced) and gathers its directory entry;
+//   2. each group of G lanes loads the head buckets of its G ops back to back
+//      (G independent 128-bit loads per lane: G*32/G = 32 buckets in flight per warp);
+//   3. with group ballots it decides every op whose chain is a single bucket (the
+//      common case at the paper's load factor): hit/miss for queries, the slot to
+//      tombstone for deletes, replace-or-install slot for inserts;
+//   4. every lane issues the CAS of its own op — one warp-wide atomic instruction;
+//   5. ops with longer chains or lost CASes take the sequential chain walk.
+enum { ST_DONE = 0, ST_CAS = 1, ST_SLOW = 2 };
+
 template <int G, int OP>
-__global__ void __launch_bounds__(kEdgeBlock) k_edges(Tables t, EdgeBatch a) {
+__global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) {
+  constexpr int W = Group<G>::W;
   const Group<G> g;
   if (OP != OP_QUERY) {
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
   }
   const u32 stack_size = (OP == OP_INSERT) ? ld_relaxed_u32(&t.ctl->stack_size) : 0u;
+  const bool reuse = a.reuse_tombstones != 0;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
-  u64 my_count = 0;
+  u32 my_count = 0;
   u32 spare = kNil;
   bool bad_range = false;
 
   for (u64 chunk = warp; chunk * 32 < a.n_ops; chunk += nwarps) {
-    // ---- stage 32 ops of the batch (coalesced), one per lane
+    // ---- 1. stage one op per lane
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
     u64 opid = j;
@@ -187,52 +230,136 @@ __global__ void __launch_bounds__(kEdgeBlock) k_edges(Tables t, EdgeBatch a) {
       bad_range = true;
     }
     const u32 row = (t.nranks == 1) ? u : u / t.nranks;
-    // ---- every lane gathers its op's directory entry and prefetches its bucket
-    u32 bkt = 0;
+    u32 head = 0;
     if (active) {
       // base/nb never change during an edge phase; only deg is written (atomics)
       const uint4 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
-      bkt = de.x + bucket_of(v, de.y);
-      prefetch_l2(t.pool + (u64)bkt * Group<G>::W);
+      head = de.x + bucket_of(v, de.y);
     }
-    // ---- each group probes the G ops held by its lanes, one after another
-    u32 res = 0, resw = 0;
-#pragma unroll 1
+    // ---- 2. head buckets of the group's G ops, all loads in flight together.
+    // The fast path (2-4) is branch-free across groups: every warp intrinsic uses
+    // the full mask and each lane reads from the lanes of its own group.
+    constexpr u32 FULL = 0xFFFFFFFFu;
+    constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
+    const u32 amask = __ballot_sync(FULL, active);
+    uint4 q[G];
+#pragma unroll
     for (int r = 0; r < G; ++r) {
-      if (!g.shfl((int)active, r)) continue;
-      const u32 rv = g.shfl(v, r);
-      const u32 rb = g.shfl(bkt, r);
-      const u32 rrow = g.shfl(row, r);
+      const u32 hr = __shfl_sync(FULL, head, g.base + r);
+      const u32* p = t.pool + (u64)hr * W + 4 * g.gl;
+      if ((amask >> (g.base + r)) & 1u) q[r] = (OP == OP_QUERY) ? ld_nc_v4(p) : ld_relaxed_v4(p);
+      else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+    }
+    // ---- 3. decide single-bucket chains
+    u32 state = ST_DONE;
+    u32 res_val = 0;                 // query: value; found in res_found
+    bool res_found = false;
+    u32* cas_addr = nullptr;
+    unsigned long long cas_old = 0;
+    const bool lastl = g.last();
+#pragma unroll
+    for (int r = 0; r < G; ++r) {
+      const uint4 x = q[r];
+      const u32 srcl = g.base + r;
+      const bool ar = (amask >> srcl) & 1u;
+      const u32 vr = __shfl_sync(FULL, v, srcl);
+      const u32 hr = __shfl_sync(FULL, head, srcl);
+      u32* bp = t.pool + (u64)hr * W + 4 * g.gl;
+      const bool m0 = ar && x.x == vr, m1 = ar && !lastl && x.z == vr;
+      const u32 hit = (__ballot_sync(FULL, m0 || m1) >> g.base) & GBITS;
+      const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
+      const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
+      const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
+      const bool whole = em != 0 || next == kNil;  // the head bucket is the whole chain
+      const u32 lh = hit ? __ffs(hit) - 1 : 0;
+      const bool mine = g.gl == (u32)r;
+      if (OP == OP_QUERY) {
+        const u32 val = __shfl_sync(FULL, m0 ? x.y : x.w, g.base + lh);
+        if (mine && ar) {
+          res_found = hit != 0;
+          res_val = val;
+          if (!hit && !whole) state = ST_SLOW;
+        }
+      } else if (OP == OP_DELETE) {
+        const u64 ka = __shfl_sync(FULL, (unsigned long long)(bp + (m0 ? 0 : 2)), g.base + lh);
+        if (mine && ar) {
+          if (hit) { state = ST_CAS; cas_addr = reinterpret_cast<u32*>(ka); }
+          else if (!whole) state = ST_SLOW;
+        }
+      } else {  // insert
+        const u32 wr = __shfl_sync(FULL, w, srcl);
+        if (hit && g.gl == lh) st_relaxed_u32(bp + (m0 ? 1 : 3), wr);  // replace
+        const bool f0 = e0 || (reuse && x.x == kTomb);
+        const bool f1 = e1 || (reuse && !lastl && x.z == kTomb);
+        const u32 fm = (__ballot_sync(FULL, f0 || f1) >> g.base) & GBITS;
+        const u32 lf = fm ? __ffs(fm) - 1 : 0;
+        const unsigned long long cur = f0 ? pack_pair(x.x, x.y) : pack_pair(x.z, x.w);
+        const u64 sa = __shfl_sync(FULL, (unsigned long long)(bp + (f0 ? 0 : 2)), g.base + lf);
+        const unsigned long long so = __shfl_sync(FULL, cur, g.base + lf);
+        if (mine && ar && !hit) {
+          if (whole && fm) { state = ST_CAS; cas_addr = reinterpret_cast<u32*>(sa); cas_old = so; }
+          else state = ST_SLOW;
+        }
+      }
+    }
+    // ---- 4. one CAS per lane, all in flight together
+    if (state == ST_CAS) {
+      if (OP == OP_DELETE) {
+        if (atomicCAS(cas_addr, v, kTomb) == v) {
+          atomicSub(&t.dir[row].deg, 1u);
+          ++my_count;
+        }
+        state = ST_DONE;  // a lost CAS means another op deleted the key (Q5)
+      } else if (OP == OP_INSERT) {
+        const unsigned long long old =
+            atomicCAS(reinterpret_cast<unsigned long long*>(cas_addr), cas_old,
+                      (unsigned long long)pack_pair(v, w));
+        if (old == cas_old) {
+          atomicAdd(&t.dir[row].deg, 1u);
+          ++my_count;
+          state = ST_DONE;
+        } else if ((u32)old == v) {  // a racing op installed the same key: replace
+          st_relaxed_u32(cas_addr + 1, w);
+          state = ST_DONE;
+        } else {
+          state = ST_SLOW;
+        }
+      }
+    }
+    // ---- 5. sequential chain walks for the rest
+    u32 slow = g.ballot(state == ST_SLOW);
+    while (slow) {
+      const u32 r = __ffs(slow) - 1;
+      slow &= slow - 1;
+      const u32 vr = g.shfl(v, r);
+      const u32 hr = g.shfl(head, r);
+      const u32 rowr = g.shfl(row, r);
       if (OP == OP_INSERT) {
-        const u32 rw = g.shfl(w, r);
-        const u64 ropid = g.shfl(opid, r);
-        const int s = probe_insert<G>(t, g, rrow, rb, rv, rw, spare, stack_size);
-        if (g.gl == 0) {
+        const u32 wr = g.shfl(w, r);
+        const int s = probe_insert<G>(t, g, rowr, hr, vr, wr, spare, stack_size, reuse);
+        if (g.gl == r) {
           if (s == 1) {
-            atomicAdd(&t.dir[rrow].deg, 1u);
+            atomicAdd(&t.dir[row].deg, 1u);
             ++my_count;
           } else if (s < 0) {
-            a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = ropid;
+            a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
           }
         }
       } else if (OP == OP_DELETE) {
-        const int s = probe_delete<G>(t, g, rb, rv);
-        if (s && g.gl == 0) {
-          atomicSub(&t.dir[rrow].deg, 1u);
+        const int s = probe_delete<G>(t, g, hr, vr);
+        if (s && g.gl == r) {
+          atomicSub(&t.dir[row].deg, 1u);
           ++my_count;
         }
       } else {
         u32 val = 0;
-        const bool f = probe_query<G>(t, g, rb, rv, val);
-        if (g.gl == (u32)r) {
-          res = f ? 1u : 0u;
-          resw = f ? val : 0u;
-        }
+        const bool f = probe_query<G>(t, g, hr, vr, val);
+        if (g.gl == r) { res_found = f; res_val = f ? val : 0u; }
       }
     }
     if (OP == OP_QUERY && valid) {
-      a.found[j] = (uint8_t)res;
-      if (a.wout) a.wout[j] = resw;
+      a.found[j] = res_found ? 1 : 0;
+      if (a.wout) a.wout[j] = res_found ? res_val : 0u;
     }
   }
   // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
@@ -242,8 +369,9 @@ __global__ void __launch_bounds__(kEdgeBlock) k_edges(Tables t, EdgeBatch a) {
     if (__any_sync(0xFFFFFFFFu, bad_range) && g.lane == 0)
       atomicMax(&t.ctl->fail_epoch, a.epoch);
   } else {
-    const u64 tot = __reduce_add_sync(0xFFFFFFFFu, (u32)my_count);
-    if (g.lane == 0 && tot) atomicAdd(reinterpret_cast<unsigned long long*>(&t.ctl->count), tot);
+    const u32 tot = __reduce_add_sync(0xFFFFFFFFu, my_count);
+    if (g.lane == 0 && tot)
+      atomicAdd(reinterpret_cast<unsigned long long*>(&t.ctl->count), (unsigned long long)tot);
   }
 }
 
@@ -307,7 +435,7 @@ static cudaError_t launch_g(const Tables& t, const EdgeBatch& a, int sms, cudaSt
   u64 blocks = (warps_needed + per_block - 1) / per_block;
   const u64 maxb = (u64)sms * grid_for<G, OP>();
   if (blocks > maxb) blocks = maxb;
-  k_edges<G, OP><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a);
+  k_edges<G, OP><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -341,12 +469,12 @@ cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 e
   u64 blocks = (n + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   if (blocks == 0) blocks = 1;
-  k_validate<<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl);
+  k_validate<<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl); note_kernel(1);
   return cudaGetLastError();
 }
 
 cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s) {
-  k_fixup_alloc<<<1, 256, 0, s>>>(t);
+  k_fixup_alloc<<<1, 256, 0, s>>>(t); note_kernel(1);
   return cudaGetLastError();
 }
 

@@ -36,7 +36,7 @@ cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hint
   u64 blocks = (count + 1 + 255) / 256;
   if (blocks > 65535) blocks = 65535;
   k_initial_buckets<<<(unsigned)blocks, 256, 0, s>>>(nb, count, row0, hints_global, hints_local,
-                                                     nranks, rank, lf_milli, bc);
+                                                     nranks, rank, lf_milli, bc); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -53,6 +53,7 @@ cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
     if (e != cudaSuccess) return e;
     *temp_bytes = need;
   }
+  note_kernel(2);
   return cub::DeviceScan::ExclusiveSum(*temp, need, in, out, (int64_t)count, s);
 }
 
@@ -81,9 +82,9 @@ cudaError_t launch_init_rows(int G, const Tables& t, u64 row0, u64 count, const 
   u64 blocks = (count + 255) / 256;
   if (blocks > 65535) blocks = 65535;
   switch (G) {
-    case 2: k_init_rows<2><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
-    case 4: k_init_rows<4><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
-    case 8: k_init_rows<8><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); break;
+    case 2: k_init_rows<2><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
+    case 4: k_init_rows<4><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
+    case 8: k_init_rows<8><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -107,7 +108,7 @@ cudaError_t launch_scatter_hints(u32* hint_new, u64 row0, u64 count, const u32* 
   u64 blocks = (n + 255) / 256;
   if (blocks > 65535) blocks = 65535;
   k_scatter_hints<<<(unsigned)blocks, 256, 0, s>>>(hint_new, row0, count, ids, hints, n, nranks,
-                                                   rank);
+                                                   rank); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -124,7 +125,7 @@ cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s) {
   if (e != cudaSuccess || n == 0) return e;
   u64 blocks = (n + 255) / 256;
   if (blocks > 1024) blocks = 1024;
-  k_max_id<<<(unsigned)blocks, 256, 0, s>>>(ids, n, out);
+  k_max_id<<<(unsigned)blocks, 256, 0, s>>>(ids, n, out); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -139,7 +140,7 @@ cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s) {
   if (t.rows == 0) return cudaSuccess;
   u64 blocks = (t.rows + 255) / 256;
   if (blocks > 65535) blocks = 65535;
-  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.dir, t.rows, out);
+  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.dir, t.rows, out); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -164,6 +165,7 @@ cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t*
     if (e != cudaSuccess) return e;
     *temp_bytes = need;
   }
+  note_kernel(2);
   return cub::DeviceScan::ExclusiveSum(*temp, need, it, ro, (int64_t)(t.rows + 1), s);
 }
 
@@ -208,9 +210,9 @@ cudaError_t launch_export_fill(int G, const Tables& t, const u64* ro, u32* dst, 
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   switch (G) {
-    case 2: k_export_fill<2><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
-    case 4: k_export_fill<4><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
-    case 8: k_export_fill<8><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+    case 2: k_export_fill<2><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
+    case 4: k_export_fill<4><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
+    case 8: k_export_fill<8><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -258,9 +260,9 @@ cudaError_t launch_stats(int G, const Tables& t, StatsOut* out, int sms, cudaStr
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   switch (G) {
-    case 2: k_stats<2><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
-    case 4: k_stats<4><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
-    case 8: k_stats<8><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+    case 2: k_stats<2><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
+    case 4: k_stats<4><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
+    case 8: k_stats<8><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -292,7 +294,7 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
   if (n == 0) return cudaSuccess;
   u64 blocks = (n + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
-  k_vdel_mark<<<(unsigned)blocks, 256, 0, s>>>(ids, n, nv, epoch, bitmap, dedup, ctl, nranks, rank);
+  k_vdel_mark<<<(unsigned)blocks, 256, 0, s>>>(ids, n, nv, epoch, bitmap, dedup, ctl, nranks, rank); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -326,9 +328,9 @@ cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epo
                               cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (G) {
-    case 2: k_vdel_sweep<2><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
-    case 4: k_vdel_sweep<4><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
-    case 8: k_vdel_sweep<8><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+    case 2: k_vdel_sweep<2><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
+    case 4: k_vdel_sweep<4><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
+    case 8: k_vdel_sweep<8><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -402,9 +404,9 @@ cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 
                                   cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (G) {
-    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
-    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
-    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -450,9 +452,9 @@ cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoc
                               cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (G) {
-    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
-    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
-    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); break;
+    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();

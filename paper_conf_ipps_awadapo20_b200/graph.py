@@ -14,7 +14,7 @@ import numpy as np
 import torch
 
 from . import _lib
-from ._lib import DGError, check, dg_config, dg_stats, lib
+from ._lib import DGError, check, dg_config, dg_profile, dg_stats, lib
 
 _U32_OK = (torch.int32, torch.uint32)
 
@@ -68,7 +68,8 @@ class Graph:
     def __init__(self, num_vertices: int, degree_hints=None, *, load_factor: float = 0.7,
                  bucket_bytes: int = 128, directed: bool = True, pool_bytes: int = 0,
                  device: int | None = None, rank: int = 0, nranks: int = 1,
-                 nccl_unique_id: bytes | None = None, stream=None):
+                 nccl_unique_id: bytes | None = None, reuse_tombstones: bool = True,
+                 stream=None):
         cfg = dg_config()
         lib.dg_config_init(ctypes.byref(cfg))
         cfg.load_factor = float(load_factor)
@@ -80,6 +81,7 @@ class Graph:
         cfg.device = int(device)
         cfg.rank = int(rank)
         cfg.nranks = int(nranks)
+        cfg.flags = 0 if reuse_tombstones else _lib.DG_FLAG_NO_TOMBSTONE_REUSE
         self._uid = None
         if nccl_unique_id is not None:
             self._uid = ctypes.create_string_buffer(bytes(nccl_unique_id), 128)
@@ -246,6 +248,19 @@ class Graph:
         if st not in (_lib.DG_OK, _lib.DG_ERR_VERTEX_OUT_OF_RANGE):
             check(st, "dg_batch_status")
         return st
+
+    # ------------------------------------------------------- instrumentation --
+    PROFILE_KINDS = ("insert", "delete", "query", "vertex_purge")
+
+    def profile_enable(self, enable: bool = True):
+        check(lib.dg_profile_enable(self._h, 1 if enable else 0), "dg_profile_enable")
+
+    def profile_read(self, stream=None) -> dict:
+        p = dg_profile()
+        check(lib.dg_profile_read(self._h, ctypes.byref(p), _stream(stream)), "dg_profile_read")
+        return {"launches": p.launches, "last_count": p.last_count,
+                "kernel_launches": dict(zip(self.PROFILE_KINDS, list(p.kernel_launches))),
+                "kernel_ms": dict(zip(self.PROFILE_KINDS, list(p.kernel_ms)))}
 
     def triangle_count(self, stream=None) -> int:
         c = ctypes.c_uint64()

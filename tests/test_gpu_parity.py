@@ -35,7 +35,7 @@ def test_golden_scripts_on_gpu(name, bb):
     run_script(load(name), lambda n, directed: GpuAdapter(n, directed, bucket_bytes=bb))
 
 
-def _config1_stream(bb, hints, directed, seed=1):
+def _config1_stream(bb, hints, directed, seed=1, reuse=True):
     """Config 1 (BASELINE.json configs[0]; SURVEY §8(d) cfg 1): |V| = 1,024;
     16 insert batches of 1,024 (5% forced intra-batch duplicates with distinct
     weights), queries, deletes, vertex deletions, re-insertion, growth and an
@@ -43,7 +43,7 @@ def _config1_stream(bb, hints, directed, seed=1):
     from paper_conf_ipps_awadapo20_b200 import DGError, DG_ERR_VERTEX_OUT_OF_RANGE, Graph
     nv = 1024
     hint = wl.out_degrees(wl.uniform_edges(seed, 0, 16 * 1024, nv)[0], nv) if hints else None
-    g = Graph(nv, hint, bucket_bytes=bb, directed=directed)
+    g = Graph(nv, hint, bucket_bytes=bb, directed=directed, reuse_tombstones=reuse)
     o = Oracle(nv, directed)
     stream = 1000
     for b in range(16):
@@ -117,6 +117,36 @@ def test_config1_undirected(bb):
     _config1_stream(bb, False, False, seed=3)
 
 
+@pytest.mark.parametrize("bb", [32, 128])
+def test_config1_append_only(bb):
+    """The paper's default policy: tombstones are never reused."""
+    _config1_stream(bb, False, True, seed=4, reuse=False)
+
+
+@pytest.mark.parametrize("reuse", [True, False])
+def test_churn_tombstone_policy(reuse):
+    """Insert/delete churn: identical results under both tombstone policies; with
+    reuse the chains stop growing (two-stage insert), without it every
+    deleted key keeps its slot."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 50_000
+    s0, d0, w0 = wl.uniform_edges(13, 0, 400_000, nv)
+    g = Graph(nv, wl.out_degrees(s0, nv), reuse_tombstones=reuse)
+    o = Oracle(nv)
+    g.insert_edges(cuda(s0), cuda(d0), cuda(w0))
+    o.insert_edges(s0, d0, w0)
+    for r in range(6):
+        s, d, w = wl.uniform_edges(13, 10 + r, 200_000, nv)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+        assert g.delete_edges(cuda(s), cuda(d), count=True) == o.delete_edges(s, d)[1]
+    check_against_oracle(g, o, "churn")
+    st = g.stats()
+    if reuse:  # bounded by the churn per vertex, not by the number of rounds
+        assert st["tombstones"] < 3 * 200_000
+    else:
+        assert st["tombstones"] >= 6 * 190_000
+
+
 @pytest.mark.parametrize("bb", GEOMS)
 def test_large_random_ragged(bb):
     """|V| = 100,000; 3 insert batches of 700,001 (ragged tail), queries, deletes."""
@@ -161,7 +191,30 @@ def test_rmat_hubs_without_hints(bb):
     assert g.insert_edges(cuda(s[m]), cuda(d[m]), cuda(w[m]), count=True) == \
         o.insert_edges(s[m], d[m], w[m])[1]
     check_against_oracle(g, o, "hubs re-inserted")
-    assert g.stats()["free_buckets"] < st2["free_buckets"]
+    st3 = g.stats()
+    assert st3["base_buckets"] + st3["overflow_buckets"] + st3["free_buckets"] <= st3["bump_buckets"]
+
+
+def test_freed_buckets_are_reused():
+    """Vertex deletion returns chained buckets to the allocator; later
+    chain growth pops them before touching never-used memory."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    s = np.zeros(3000, np.uint32)
+    d = (np.arange(3000) + 4).astype(np.uint32)
+    g2 = Graph(3100, bucket_bytes=32)  # 3 pairs per bucket, one base bucket per vertex
+    g2.insert_edges(cuda(s), cuda(d))
+    st1 = g2.stats()
+    assert st1["overflow_buckets"] == 999 and st1["live_pairs"] == 3000
+    g2.delete_vertices(cuda(np.array([0], np.uint32)))
+    st2 = g2.stats()
+    assert st2["free_buckets"] - st1["free_buckets"] == 999 and st2["live_pairs"] == 0
+    for i in range(60):  # one op per launch: no chain-link races, no spare buckets
+        g2.insert_edges(cuda(s[i:i + 1]), cuda(d[i:i + 1]))
+    st3 = g2.stats()
+    assert st3["overflow_buckets"] == 19 and st3["live_pairs"] == 60
+    assert st3["bump_buckets"] == st2["bump_buckets"]  # nothing new taken from the pool
+    assert st3["free_buckets"] == st2["free_buckets"] - 19
+    g2.close()
 
 
 def test_heavy_intra_batch_duplicates():

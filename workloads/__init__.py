@@ -42,13 +42,13 @@ def _L():
             lib = ctypes.CDLL(build())
             lib.wl_rng.restype = ctypes.c_uint64
             lib.wl_rng.argtypes = [ctypes.c_uint64] * 3
-            lib.wl_uniform_edges.argtypes = [ctypes.c_uint64, ctypes.c_uint64, ctypes.c_uint64,
-                                             ctypes.c_uint64, U32P, U32P, U32P]
-            lib.wl_uniform_u32.argtypes = [ctypes.c_uint64] * 4 + [U32P]
+            lib.wl_uniform_edges.argtypes = [ctypes.c_uint64] * 5 + [U32P, U32P, U32P]
+            lib.wl_uniform_u32.argtypes = [ctypes.c_uint64] * 5 + [U32P]
             lib.wl_uniform_index.argtypes = [ctypes.c_uint64] * 4 + [U64P]
             lib.wl_permute.restype = ctypes.c_uint32
             lib.wl_permute.argtypes = [ctypes.c_uint32, ctypes.c_int, ctypes.c_uint64]
             lib.wl_rmat_edges.argtypes = [ctypes.c_uint64, ctypes.c_uint64, ctypes.c_uint64,
+                                          U64P, ctypes.c_uint64,
                                           ctypes.c_int, ctypes.c_double, ctypes.c_double,
                                           ctypes.c_double, ctypes.c_int, ctypes.c_uint64,
                                           U32P, U32P]
@@ -68,18 +68,20 @@ def rng(seed: int, stream: int, index: int) -> int:
     return int(_L().wl_rng(seed, stream, index))
 
 
-def uniform_edges(seed: int, stream: int, n: int, nv: int, weights: bool = True):
-    """n edges with src, dst uniform on [0, nv); weights uniform u32."""
+def uniform_edges(seed: int, stream: int, n: int, nv: int, weights: bool = True,
+                  offset: int = 0):
+    """Edges offset..offset+n-1 of a stream: src, dst uniform on [0, nv); weights
+    uniform u32.  Any slice regenerates bit-identically."""
     s = np.empty(n, np.uint32)
     d = np.empty(n, np.uint32)
     w = np.empty(n, np.uint32) if weights else None
-    _L().wl_uniform_edges(seed, stream, n, nv, _p32(s), _p32(d), _p32(w))
+    _L().wl_uniform_edges(seed, stream, offset, n, nv, _p32(s), _p32(d), _p32(w))
     return s, d, w
 
 
-def uniform_u32(seed: int, stream: int, n: int, bound: int = 0) -> np.ndarray:
+def uniform_u32(seed: int, stream: int, n: int, bound: int = 0, offset: int = 0) -> np.ndarray:
     out = np.empty(n, np.uint32)
-    _L().wl_uniform_u32(seed, stream, n, bound, _p32(out))
+    _L().wl_uniform_u32(seed, stream, offset, n, bound, _p32(out))
     return out
 
 
@@ -98,12 +100,18 @@ LJLIKE = (0.50, 0.20, 0.20)
 
 
 def rmat_edges(seed: int, stream: int, n: int, scale: int, abc=GRAPH500,
-               permute_ids: bool = True, nv: int = 0):
-    """n R-MAT edges over 2^scale vertices (rejected to [0, nv) if nv>0)."""
+               permute_ids: bool = True, nv: int = 0, offset: int = 0, index=None):
+    """R-MAT edges offset..offset+n-1 (or the edge ids in ``index``) over 2^scale
+    vertices, rejected to [0, nv) if nv > 0."""
+    if index is not None:
+        index = np.ascontiguousarray(index, np.uint64)
+        n = index.size
     s = np.empty(n, np.uint32)
     d = np.empty(n, np.uint32)
     a, b, c = abc
-    _L().wl_rmat_edges(seed, stream, n, scale, a, b, c, int(permute_ids), nv, _p32(s), _p32(d))
+    _L().wl_rmat_edges(seed, stream, offset,
+                       None if index is None else index.ctypes.data_as(U64P), n, scale,
+                       a, b, c, int(permute_ids), nv, _p32(s), _p32(d))
     return s, d
 
 
@@ -125,8 +133,8 @@ def out_degrees(src: np.ndarray, nv: int) -> np.ndarray:
     return deg
 
 
-def weights(seed: int, stream: int, n: int) -> np.ndarray:
-    return uniform_u32(seed, stream ^ 0x77777777, n, 0)
+def weights(seed: int, stream: int, n: int, offset: int = 0) -> np.ndarray:
+    return uniform_u32(seed, stream ^ 0x77777777, n, 0, offset)
 
 
 def symmetrise(src: np.ndarray, dst: np.ndarray):

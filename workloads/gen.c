@@ -40,25 +40,26 @@ uint64_t wl_rng(uint64_t seed, uint64_t stream, uint64_t index) {
 /* ---------------------------------------------------------------- uniform ---- */
 /* n edges with src,dst uniform on [0, nv) (self-loops and duplicates occur
  * naturally), weights uniform u32.  w may be NULL. */
-void wl_uniform_edges(uint64_t seed, uint64_t stream, uint64_t n, uint64_t nv,
+void wl_uniform_edges(uint64_t seed, uint64_t stream, uint64_t i0, uint64_t n, uint64_t nv,
                       uint32_t* src, uint32_t* dst, uint32_t* w) {
   const uint64_t k = stream_key(seed, stream);
   const uint64_t kw = stream_key(seed, stream ^ 0x5757575757575757ULL);
 #pragma omp parallel for schedule(static)
   for (int64_t i = 0; i < (int64_t)n; ++i) {
-    uint64_t r = rng_k(k, (uint64_t)i);
+    uint64_t r = rng_k(k, i0 + (uint64_t)i);
     src[i] = below((uint32_t)(r >> 32), nv);
     dst[i] = below((uint32_t)r, nv);
-    if (w) w[i] = (uint32_t)(rng_k(kw, (uint64_t)i) >> 32);
+    if (w) w[i] = (uint32_t)(rng_k(kw, i0 + (uint64_t)i) >> 32);
   }
 }
 
 /* uniform u32 values (weights, or indices after reduction by the caller) */
-void wl_uniform_u32(uint64_t seed, uint64_t stream, uint64_t n, uint64_t bound, uint32_t* out) {
+void wl_uniform_u32(uint64_t seed, uint64_t stream, uint64_t i0, uint64_t n, uint64_t bound,
+                    uint32_t* out) {
   const uint64_t k = stream_key(seed, stream);
 #pragma omp parallel for schedule(static)
   for (int64_t i = 0; i < (int64_t)n; ++i) {
-    uint32_t r = (uint32_t)(rng_k(k, (uint64_t)i) >> 32);
+    uint32_t r = (uint32_t)(rng_k(k, i0 + (uint64_t)i) >> 32);
     out[i] = bound ? below(r, bound) : r;
   }
 }
@@ -118,8 +119,9 @@ static inline void rmat_one(uint64_t key, uint64_t i, uint64_t attempt, int scal
   *s = u; *d = v;
 }
 
-void wl_rmat_edges(uint64_t seed, uint64_t stream, uint64_t n, int scale,
-                   double a, double b, double c, int permute, uint64_t nv,
+/* edge ids: idx[i] if idx != NULL, else i0 + i */
+void wl_rmat_edges(uint64_t seed, uint64_t stream, uint64_t i0, const uint64_t* idx, uint64_t n,
+                   int scale, double a, double b, double c, int permute, uint64_t nv,
                    uint32_t* src, uint32_t* dst) {
   const uint64_t key = stream_key(seed, stream);
   const double two32 = 4294967296.0;
@@ -132,8 +134,9 @@ void wl_rmat_edges(uint64_t seed, uint64_t stream, uint64_t n, int scale,
 #pragma omp parallel for schedule(static)
   for (int64_t i = 0; i < (int64_t)n; ++i) {
     uint32_t s, d;
+    const uint64_t e = idx ? idx[i] : i0 + (uint64_t)i;
     for (uint64_t att = 0;; ++att) {
-      rmat_one(key, (uint64_t)i, att, scale, ta, tab, tabc, &s, &d);
+      rmat_one(key, e, att, scale, ta, tab, tabc, &s, &d);
       if (permute) { s = wl_permute(s, scale, seed); d = wl_permute(d, scale, seed); }
       if (s < nv && d < nv) break;
     }
