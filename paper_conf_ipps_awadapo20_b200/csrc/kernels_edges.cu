@@ -48,164 +48,43 @@ __device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 stack_size) {
   return j < t.cap ? j : kNil;
 }
 
-// ------------------------------------------------------------ probe: insert ----
-// Full chain walk from the head bucket b (slow path; the fast path in k_edges
-// handles single-bucket chains).  The key must be absent from the whole chain
-// before it is installed (uniqueness); it is installed with
-// a 64-bit CAS in the FIRST free slot of the chain: the first tombstone when
-// tombstones are reused (the paper's two-stage option), else the
-// first EMPTY.  Any failed slot CAS re-scans the chain from the head:
-// two inserts of one key then always contend for the same slot.
-// returns 1 = key added, 0 = existing key replaced, -1 = no bucket available
-template <int G>
-__device__ __forceinline__ int probe_insert(const Tables& t, const Group<G>& g, u32 row,
-                                            const u32 head, u32 v, u32 w, u32& spare,
-                                            u32 stack_size, bool reuse) {
-  constexpr int W = Group<G>::W;
-  u32 b = head;
-  u32* ff = nullptr;         // first free slot seen (pair address), group-uniform
-  unsigned long long ffo = 0;  // its current contents
-  while (true) {
-    u32* bp = t.pool + (u64)b * W;
-    const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
-    const bool lastl = g.last();
-    const bool m0 = q.x == v, m1 = !lastl && q.z == v;
-    const u32 hit = g.ballot(m0 || m1);
-    if (hit) {  // replace: key exists
-      const u32 l = __ffs(hit) - 1;
-      if (g.gl == l) st_relaxed_u32(bp + 4 * g.gl + (m0 ? 1 : 3), w);
-      return 0;
-    }
-    const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
-    const u32 em = g.ballot(e0 || e1);
-    if (!ff) {
-      const bool f0 = e0 || (reuse && q.x == kTomb);
-      const bool f1 = e1 || (reuse && !lastl && q.z == kTomb);
-      const u32 fm = g.ballot(f0 || f1);
-      if (fm) {
-        const u32 l = __ffs(fm) - 1;
-        const u64 addr = (u64)(bp + 4 * g.gl + (f0 ? 0 : 2));
-        const unsigned long long cur = f0 ? pack_pair(q.x, q.y) : pack_pair(q.z, q.w);
-        ff = reinterpret_cast<u32*>(g.shfl(addr, l));
-        ffo = g.shfl(cur, l);
-      }
-    }
-    const u32 next = g.shfl(q.z, G - 1);
-    if (em || next == kNil) {
-      // end of the chain: the key is absent
-      if (ff) {
-        unsigned long long old = 0;
-        if (g.gl == 0)
-          old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
-                          (unsigned long long)pack_pair(v, w));
-        old = g.shfl(old, 0);
-        if (old == ffo) return 1;
-        if ((u32)old == v) {  // a racing op installed the same key there: replace
-          if (g.gl == 0) st_relaxed_u32(ff + 1, w);
-          return 0;
-        }
-        ff = nullptr;  // slot taken by another key: re-scan from the head
-        b = head;
-        continue;
-      }
-      // chain full: link a new bucket at the tail
-      if (spare == kNil) {
-        u32 s = 0;
-        if (g.gl == 0) s = alloc_bucket(t, stack_size);
-        spare = g.shfl(s, 0);
-        if (spare == kNil) return -1;
-      }
-      u32 old = 0;
-      if (lastl) {
-        st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
-        old = atomicCAS(bp + Group<G>::NEXT, kNil, spare);
-      }
-      old = g.shfl(old, G - 1);
-      if (old == kNil) {
-        b = spare;
-        spare = kNil;
-      } else {
-        b = old;  // another op linked first (earlier slots cannot free up); keep our spare
-      }
-      continue;
-    }
-    b = next;
-  }
-}
-
-// ------------------------------------------------------------ probe: delete ----
-template <int G>
-__device__ __forceinline__ int probe_delete(const Tables& t, const Group<G>& g, u32 b, u32 v) {
-  constexpr int W = Group<G>::W;
-  while (true) {
-    u32* bp = t.pool + (u64)b * W;
-    const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
-    const bool lastl = g.last();
-    const bool m0 = q.x == v, m1 = !lastl && q.z == v;
-    const u32 hit = g.ballot(m0 || m1);
-    if (hit) {
-      const u32 l = __ffs(hit) - 1;
-      u32 old = 0;
-      if (g.gl == l) old = atomicCAS(bp + 4 * g.gl + (m0 ? 0 : 2), v, kTomb);
-      return g.shfl(old, l) == v ? 1 : 0;
-    }
-    const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
-    if (g.ballot(e0 || e1)) return 0;
-    const u32 next = g.shfl(q.z, G - 1);
-    if (next == kNil) return 0;
-    b = next;
-  }
-}
-
-// ------------------------------------------------------------- probe: query ----
-template <int G>
-__device__ __forceinline__ bool probe_query(const Tables& t, const Group<G>& g, u32 b, u32 v,
-                                            u32& val) {
-  constexpr int W = Group<G>::W;
-  while (true) {
-    const u32* bp = t.pool + (u64)b * W;
-    const uint4 q = ld_nc_v4(bp + 4 * g.gl);
-    const bool lastl = g.last();
-    const bool m0 = q.x == v, m1 = !lastl && q.z == v;
-    const u32 hit = g.ballot(m0 || m1);
-    if (hit) {
-      const u32 l = __ffs(hit) - 1;
-      val = g.shfl(m0 ? q.y : q.w, l);
-      return true;
-    }
-    const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
-    if (g.ballot(e0 || e1)) return false;
-    const u32 next = g.shfl(q.z, G - 1);
-    if (next == kNil) return false;
-    b = next;
-  }
-}
-
 // ------------------------------------------------------------- main kernel ----
-// Per warp iteration (32 ops):
-//   1. lane L stages op L (coalesced) and gathers its directory entry;
-//   2. each group of G lanes loads the head buckets of its G ops back to back
-//      (G independent 128-bit loads per lane: G*32/G = 32 buckets in flight per warp);
-//   3. with group ballots it decides every op whose chain is a single bucket (the
-//      common case at the paper's load factor): hit/miss for queries, the slot to
-//      tombstone for deletes, replace-or-install slot for inserts;
-//   4. every lane issues the CAS of its own op — one warp-wide atomic instruction;
-//   5. ops with longer chains or lost CASes take the sequential chain walk.
-enum { ST_DONE = 0, ST_CAS = 1, ST_SLOW = 2 };
+// Per warp iteration (32 ops of the batch):
+//   1. lane L stages op L (coalesced loads) and gathers its directory entry; its
+//      op starts at the head bucket b = base + hash(v) mod nb of A_u;
+//   2. rounds, until no op of the warp is pending:
+//      a. each group of G lanes loads the CURRENT bucket of each of its G pending ops
+//         (G independent 16-B loads per lane: up to 32 buckets in flight per warp);
+//      b. with full-warp ballots/shuffles (each lane reads its own group's lanes;
+//         no divergence, no group-masked syncs) every op is decided from its
+//         bucket: key found / chain ended / continue to `next`;
+//      c. the lane that owns an op performs its atomic: the delete CAS
+//         key -> tombstone, the insert CAS of (key, value) into the chain's first
+//         free slot, or the allocation + CAS-link of a new tail bucket — all lanes
+//         of the warp in one instruction.
+//   The insert follows Alg. 1's replace: the whole chain is scanned
+//   for the key before a new pair is installed; the install targets the FIRST free
+//   slot (first tombstone when tombstones are reused, else the first
+//   EMPTY) and a failed install CAS re-scans from the head, so two
+//   inserts of one key always contend for the same slot.
+enum { ACT_NONE = 0, ACT_CAS_DEL = 1, ACT_CAS_INS = 2, ACT_EXTEND = 3 };
 
 template <int G, int OP>
 __global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) {
   constexpr int W = Group<G>::W;
+  constexpr u32 FULL = 0xFFFFFFFFu;
+  constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
   const Group<G> g;
   if (OP != OP_QUERY) {
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
   }
   const u32 stack_size = (OP == OP_INSERT) ? ld_relaxed_u32(&t.ctl->stack_size) : 0u;
   const bool reuse = a.reuse_tombstones != 0;
+  const bool lastl = g.last();
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
   u32 my_count = 0;
-  u32 spare = kNil;
+  u32 spare = kNil;  // a fresh bucket this lane allocated but could not link
   bool bad_range = false;
 
   for (u64 chunk = warp; chunk * 32 < a.n_ops; chunk += nwarps) {
@@ -224,152 +103,142 @@ __global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) 
       if (OP == OP_INSERT && a.w) w = a.w[i];
       if (rev) { const u32 x = u; u = v; v = x; }
     }
-    bool active = valid && u != v;  // self-loops are never stored (Alg1:L3)
+    bool pend = valid && u != v;  // self-loops are never stored (Alg1:L3)
     if (OP == OP_QUERY && valid && ((u64)u >= a.nv || (u64)v >= a.nv)) {
-      active = false;
+      pend = false;
       bad_range = true;
     }
     const u32 row = (t.nranks == 1) ? u : u / t.nranks;
     u32 head = 0;
-    if (active) {
+    if (pend) {
       // base/nb never change during an edge phase; only deg is written (atomics)
       const uint4 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
       head = de.x + bucket_of(v, de.y);
     }
-    // ---- 2. head buckets of the group's G ops, all loads in flight together.
-    // The fast path (2-4) is branch-free across groups: every warp intrinsic uses
-    // the full mask and each lane reads from the lanes of its own group.
-    constexpr u32 FULL = 0xFFFFFFFFu;
-    constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
-    const u32 amask = __ballot_sync(FULL, active);
-    uint4 q[G];
+    u32 cur = head;
+    bool found = false;
+    u32 val = 0;
+    u32* ff = nullptr;               // insert: first free slot of the chain (pair address)
+    unsigned long long ffo = 0;      //         and its contents when scanned
+
+    // ---- 2. rounds
+    while (true) {
+      const u32 pm = __ballot_sync(FULL, pend);
+      if (pm == 0) break;
+      // a. current buckets of the group's pending ops
+      uint4 q[G];
 #pragma unroll
-    for (int r = 0; r < G; ++r) {
-      const u32 hr = __shfl_sync(FULL, head, g.base + r);
-      const u32* p = t.pool + (u64)hr * W + 4 * g.gl;
-      if ((amask >> (g.base + r)) & 1u) q[r] = (OP == OP_QUERY) ? ld_nc_v4(p) : ld_relaxed_v4(p);
-      else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
-    }
-    // ---- 3. decide single-bucket chains
-    u32 state = ST_DONE;
-    u32 res_val = 0;                 // query: value; found in res_found
-    bool res_found = false;
-    u32* cas_addr = nullptr;
-    unsigned long long cas_old = 0;
-    const bool lastl = g.last();
+      for (int r = 0; r < G; ++r) {
+        const u32 cr = __shfl_sync(FULL, cur, g.base + r);
+        const u32* p = t.pool + (u64)cr * W + 4 * g.gl;
+        if ((pm >> (g.base + r)) & 1u) q[r] = (OP == OP_QUERY) ? ld_nc_v4(p) : ld_relaxed_v4(p);
+        else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+      }
+      // b. decide
+      int act = ACT_NONE;
 #pragma unroll
-    for (int r = 0; r < G; ++r) {
-      const uint4 x = q[r];
-      const u32 srcl = g.base + r;
-      const bool ar = (amask >> srcl) & 1u;
-      const u32 vr = __shfl_sync(FULL, v, srcl);
-      const u32 hr = __shfl_sync(FULL, head, srcl);
-      u32* bp = t.pool + (u64)hr * W + 4 * g.gl;
-      const bool m0 = ar && x.x == vr, m1 = ar && !lastl && x.z == vr;
-      const u32 hit = (__ballot_sync(FULL, m0 || m1) >> g.base) & GBITS;
-      const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
-      const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
-      const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
-      const bool whole = em != 0 || next == kNil;  // the head bucket is the whole chain
-      const u32 lh = hit ? __ffs(hit) - 1 : 0;
-      const bool mine = g.gl == (u32)r;
-      if (OP == OP_QUERY) {
-        const u32 val = __shfl_sync(FULL, m0 ? x.y : x.w, g.base + lh);
-        if (mine && ar) {
-          res_found = hit != 0;
-          res_val = val;
-          if (!hit && !whole) state = ST_SLOW;
-        }
-      } else if (OP == OP_DELETE) {
-        const u64 ka = __shfl_sync(FULL, (unsigned long long)(bp + (m0 ? 0 : 2)), g.base + lh);
-        if (mine && ar) {
-          if (hit) { state = ST_CAS; cas_addr = reinterpret_cast<u32*>(ka); }
-          else if (!whole) state = ST_SLOW;
-        }
-      } else {  // insert
-        const u32 wr = __shfl_sync(FULL, w, srcl);
-        if (hit && g.gl == lh) st_relaxed_u32(bp + (m0 ? 1 : 3), wr);  // replace
-        const bool f0 = e0 || (reuse && x.x == kTomb);
-        const bool f1 = e1 || (reuse && !lastl && x.z == kTomb);
-        const u32 fm = (__ballot_sync(FULL, f0 || f1) >> g.base) & GBITS;
-        const u32 lf = fm ? __ffs(fm) - 1 : 0;
-        const unsigned long long cur = f0 ? pack_pair(x.x, x.y) : pack_pair(x.z, x.w);
-        const u64 sa = __shfl_sync(FULL, (unsigned long long)(bp + (f0 ? 0 : 2)), g.base + lf);
-        const unsigned long long so = __shfl_sync(FULL, cur, g.base + lf);
-        if (mine && ar && !hit) {
-          if (whole && fm) { state = ST_CAS; cas_addr = reinterpret_cast<u32*>(sa); cas_old = so; }
-          else state = ST_SLOW;
-        }
-      }
-    }
-    // ---- 4. one CAS per lane, all in flight together
-    if (state == ST_CAS) {
-      if (OP == OP_DELETE) {
-        if (atomicCAS(cas_addr, v, kTomb) == v) {
-          atomicSub(&t.dir[row].deg, 1u);
-          ++my_count;
-        }
-        state = ST_DONE;  // a lost CAS means another op deleted the key (Q5)
-      } else if (OP == OP_INSERT) {
-        const unsigned long long old =
-            atomicCAS(reinterpret_cast<unsigned long long*>(cas_addr), cas_old,
-                      (unsigned long long)pack_pair(v, w));
-        if (old == cas_old) {
-          atomicAdd(&t.dir[row].deg, 1u);
-          ++my_count;
-          state = ST_DONE;
-        } else if ((u32)old == v) {  // a racing op installed the same key: replace
-          st_relaxed_u32(cas_addr + 1, w);
-          state = ST_DONE;
-        } else {
-          state = ST_SLOW;
-        }
-      }
-    }
-    // ---- 5. sequential chain walks for the rest
-    u32 slow = g.ballot(state == ST_SLOW);
-    while (slow) {
-      const u32 r = __ffs(slow) - 1;
-      slow &= slow - 1;
-      const u32 vr = g.shfl(v, r);
-      const u32 hr = g.shfl(head, r);
-      const u32 rowr = g.shfl(row, r);
-      if (OP == OP_INSERT) {
-        const u32 wr = g.shfl(w, r);
-        const int s = probe_insert<G>(t, g, rowr, hr, vr, wr, spare, stack_size, reuse);
-        if (g.gl == r) {
-          if (s == 1) {
-            atomicAdd(&t.dir[row].deg, 1u);
-            ++my_count;
-          } else if (s < 0) {
-            a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
+      for (int r = 0; r < G; ++r) {
+        const uint4 x = q[r];
+        const u32 srcl = g.base + r;
+        const bool pr = (pm >> srcl) & 1u;
+        const u32 vr = __shfl_sync(FULL, v, srcl);
+        const u32 cr = __shfl_sync(FULL, cur, srcl);
+        u32* bp = t.pool + (u64)cr * W + 4 * g.gl;
+        const bool m0 = pr && x.x == vr, m1 = pr && !lastl && x.z == vr;
+        const u32 hit = (__ballot_sync(FULL, m0 || m1) >> g.base) & GBITS;
+        const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
+        const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
+        const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
+        const bool end = em != 0 || next == kNil;  // EMPTY slots only exist at the tail
+        const u32 lh = hit ? __ffs(hit) - 1 : 0;
+        const bool mine = pr && g.gl == (u32)r;
+        if (OP == OP_QUERY) {
+          const u32 hv = __shfl_sync(FULL, m0 ? x.y : x.w, g.base + lh);
+          if (mine) {
+            if (hit) { found = true; val = hv; pend = false; }
+            else if (end) pend = false;
+            else cur = next;
+          }
+        } else if (OP == OP_DELETE) {
+          const u64 ka = __shfl_sync(FULL, (unsigned long long)(bp + (m0 ? 0 : 2)), g.base + lh);
+          if (mine) {
+            if (hit) { act = ACT_CAS_DEL; ff = reinterpret_cast<u32*>(ka); }
+            else if (end) pend = false;
+            else cur = next;
+          }
+        } else {  // insert
+          const u32 wr = __shfl_sync(FULL, w, srcl);
+          if (hit && g.gl == lh) st_relaxed_u32(bp + (m0 ? 1 : 3), wr);  // replace
+          const bool f0 = e0 || (reuse && x.x == kTomb);
+          const bool f1 = e1 || (reuse && !lastl && x.z == kTomb);
+          const u32 fm = (__ballot_sync(FULL, f0 || f1) >> g.base) & GBITS;
+          const u32 lf = fm ? __ffs(fm) - 1 : 0;
+          const unsigned long long cont = f0 ? pack_pair(x.x, x.y) : pack_pair(x.z, x.w);
+          const u64 sa = __shfl_sync(FULL, (unsigned long long)(bp + (f0 ? 0 : 2)), g.base + lf);
+          const unsigned long long so = __shfl_sync(FULL, cont, g.base + lf);
+          if (mine) {
+            if (hit) {
+              pend = false;
+            } else {
+              if (!ff && fm) { ff = reinterpret_cast<u32*>(sa); ffo = so; }
+              if (end) act = ff ? ACT_CAS_INS : ACT_EXTEND;
+              else cur = next;
+            }
           }
         }
-      } else if (OP == OP_DELETE) {
-        const int s = probe_delete<G>(t, g, hr, vr);
-        if (s && g.gl == r) {
+      }
+      // c. one atomic per lane, all in flight together
+      if (OP == OP_DELETE && act == ACT_CAS_DEL) {
+        if (atomicCAS(ff, v, kTomb) == v) {
           atomicSub(&t.dir[row].deg, 1u);
           ++my_count;
         }
-      } else {
-        u32 val = 0;
-        const bool f = probe_query<G>(t, g, hr, vr, val);
-        if (g.gl == r) { res_found = f; res_val = f ? val : 0u; }
+        pend = false;  // a lost CAS means another op deleted the key (Q5)
+      }
+      if (OP == OP_INSERT && act == ACT_CAS_INS) {
+        const unsigned long long old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
+                                                 (unsigned long long)pack_pair(v, w));
+        if (old == ffo) {
+          atomicAdd(&t.dir[row].deg, 1u);
+          ++my_count;
+          pend = false;
+        } else if ((u32)old == v) {  // a racing op installed the same key: replace
+          st_relaxed_u32(ff + 1, w);
+          pend = false;
+        } else {  // the slot went to another key: re-scan from the head
+          cur = head;
+          ff = nullptr;
+        }
+      }
+      if (OP == OP_INSERT && act == ACT_EXTEND) {
+        // chain full: link a new bucket at the tail (a8)
+        if (spare == kNil) spare = alloc_bucket(t, stack_size);
+        if (spare == kNil) {  // pool exhausted: the host grows it and re-runs this op
+          a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
+          pend = false;
+        } else {
+          st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
+          const u32 old = atomicCAS(t.pool + (u64)cur * W + Group<G>::NEXT, kNil, spare);
+          if (old == kNil) {
+            cur = spare;
+            spare = kNil;
+          } else {
+            cur = old;  // another op linked first (no earlier slot can free up); keep ours
+          }
+        }
       }
     }
     if (OP == OP_QUERY && valid) {
-      a.found[j] = res_found ? 1 : 0;
-      if (a.wout) a.wout[j] = res_found ? res_val : 0u;
+      a.found[j] = found ? 1 : 0;
+      if (a.wout) a.wout[j] = found ? val : 0u;
     }
   }
   // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
-  if (OP == OP_INSERT && spare != kNil && g.gl == 0)
-    t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
+  if (OP == OP_INSERT && spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
   if (OP == OP_QUERY) {
-    if (__any_sync(0xFFFFFFFFu, bad_range) && g.lane == 0)
-      atomicMax(&t.ctl->fail_epoch, a.epoch);
+    if (__any_sync(FULL, bad_range) && g.lane == 0) atomicMax(&t.ctl->fail_epoch, a.epoch);
   } else {
-    const u32 tot = __reduce_add_sync(0xFFFFFFFFu, my_count);
+    const u32 tot = __reduce_add_sync(FULL, my_count);
     if (g.lane == 0 && tot)
       atomicAdd(reinterpret_cast<unsigned long long*>(&t.ctl->count), (unsigned long long)tot);
   }
@@ -460,8 +329,9 @@ cudaError_t launch_query(int G, const Tables& t, const EdgeBatch& a, int sms, cu
 }
 
 u64 max_groups(int G, int sms) {
-  // upper bound on groups resident in one launch (bounds the spare-return list)
-  return (u64)sms * 2048 / (u64)G;
+  // upper bound on threads resident in one launch: each may hold one spare bucket
+  (void)G;
+  return (u64)sms * 2048;
 }
 
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
