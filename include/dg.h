@@ -99,6 +99,10 @@ typedef struct dg_config {
  * are identical, chains stop growing under insert/delete churn).  This flag selects
  * the paper's default append-only policy: tombstones are never reused. */
 #define DG_FLAG_NO_TOMBSTONE_REUSE 1u
+/* Diagnostic: route a single-GPU graph (nranks == 1) through the multi-GPU batch
+ * router over a 1-rank NCCL communicator (exercises partition / exchange / answer
+ * return on one GPU). */
+#define DG_FLAG_FORCE_ROUTER 2u
 
 /* Memory / structure statistics (Fig. 2b/c quantities). */
 typedef struct dg_stats {

@@ -23,8 +23,22 @@ OBJ = os.path.join(ROOT, "build", "dg")
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
+
+
+def _nccl_include():
+    """Headers of the NCCL that torch links (2.28.x wheel); libnccl itself is dlopen'ed."""
+    for p in sys.path + [os.path.dirname(os.path.dirname(os.__file__)) + "/site-packages"]:
+        cand = os.path.join(p, "nvidia", "nccl", "include")
+        if os.path.exists(os.path.join(cand, "nccl.h")):
+            return cand
+    if os.path.exists("/usr/include/nccl.h"):
+        return "/usr/include"
+    raise RuntimeError("nccl.h not found")
+
+
 FLAGS = ["-O3", "-lineinfo", "-std=c++17", "--expt-relaxed-constexpr", "-Xcompiler", "-fPIC",
-         "-Xcompiler", "-fvisibility=hidden", "-I", os.path.join(ROOT, "include")]
+         "-Xcompiler", "-fvisibility=hidden", "-I", os.path.join(ROOT, "include"),
+         "-I", _nccl_include()]
 
 
 def _sources():

@@ -451,7 +451,7 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
-  if (cfg->flags & ~DG_FLAG_NO_TOMBSTONE_REUSE) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->flags & ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER)) return DG_ERR_INVALID_ARGUMENT;
 
   dg_graph g = new (std::nothrow) dg_graph_s();
   if (!g) return DG_ERR_OUT_OF_MEMORY;
@@ -501,6 +501,12 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
 
   if (g->nranks > 1) {
     dg_status st = dg::router_create(g, cfg->nccl_unique_id, &g->router);
+    if (st != DG_OK) return fail(st);
+  } else if (cfg->flags & DG_FLAG_FORCE_ROUTER) {
+    // diagnostic: route a single-GPU graph through the NCCL path (1-rank communicator)
+    char id[128];
+    dg_status st = dg::router_unique_id(id);
+    if (st == DG_OK) st = dg::router_create(g, id, &g->router);
     if (st != DG_OK) return fail(st);
   }
 
@@ -560,7 +566,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
   DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
   DG_TRY(stage_in(g, 2, weight, weight ? n * 4 : 0, s, &dw, &host));
-  if (g->nranks > 1) {
+  if (g->router) {
     DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
   } else {
     DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
@@ -570,7 +576,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   if (n_added || host) {
     DG_TRY(read_ctl(g, s));
     u64 cnt = g->hctl->count;
-    if (g->nranks > 1) DG_TRY(dg::router_sum_u64(g, &cnt, s));
+    if (g->router) DG_TRY(dg::router_sum_u64(g, &cnt, s));
     if (n_added) *n_added = cnt;
     g->snap_pending = false;
     g->bump_ub = g->hctl->bump;
@@ -591,7 +597,7 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
   const void *ds = nullptr, *dd = nullptr;
   DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
   DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
-  if (g->nranks > 1) {
+  if (g->router) {
     DG_TRY(dg::router_delete(g, (const u32*)ds, (const u32*)dd, n, epoch, s));
   } else {
     DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
@@ -602,7 +608,7 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
     g->snap_pending = false;
     DG_TRY(read_ctl(g, s));
     u64 cnt = g->hctl->count;
-    if (g->nranks > 1) DG_TRY(dg::router_sum_u64(g, &cnt, s));
+    if (g->router) DG_TRY(dg::router_sum_u64(g, &cnt, s));
     if (n_removed) *n_removed = cnt;
     return status_of(g, epoch);
   }
@@ -623,7 +629,7 @@ dg_status dg_query_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, u
   DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
   DG_TRY(stage_out(g, 3, found, n, &df, &host));
   DG_TRY(stage_out(g, 4, weight_out, weight_out ? n * 4 : 0, &dw, &host));
-  if (g->nranks > 1) {
+  if (g->router) {
     DG_TRY(dg::router_query(g, (const u32*)ds, (const u32*)dd, n, (uint8_t*)df, (u32*)dw, epoch, s));
   } else {
     DG_TRY(dg::local_query(g, (const u32*)ds, (const u32*)dd, n, (uint8_t*)df, (u32*)dw, epoch, s));
@@ -649,6 +655,22 @@ dg_status dg_insert_vertices(dg_graph g, const uint32_t* ids, uint64_t n,
   const void *di = nullptr, *dh = nullptr;
   DG_TRY(stage_in(g, 5, ids, n * 4, s, &di, &host));
   DG_TRY(stage_in(g, 6, degree_hints, degree_hints ? n * 4 : 0, s, &dh, &host));
+  if (g->router) {
+    // every rank needs every (id, hint): the rows of an ID live on its owner
+    const u32* all_ids = nullptr;
+    const u32* all_h = nullptr;
+    u64 all_n = 0, hn = 0;
+    DG_TRY(dg::router_allgather_u32(g, (const u32*)di, n, 0, &all_ids, &all_n, s));
+    if (!dh && n) {  // a rank without hints contributes zeros (= unknown degree)
+      DG_CK(ensure_buf(g->stage[6], n * 4));
+      DG_CK(cudaMemsetAsync(g->stage[6].p, 0, n * 4, s));
+      dh = g->stage[6].p;
+    }
+    DG_TRY(dg::router_allgather_u32(g, (const u32*)dh, n, 1, &all_h, &hn, s));
+    di = all_ids;
+    dh = all_h;
+    n = all_n;
+  }
   u64 maxid = 0;
   bool any = n > 0;
   if (any) {
@@ -661,7 +683,7 @@ dg_status dg_insert_vertices(dg_graph g, const uint32_t* ids, uint64_t n,
   }
   u64 new_nv = g->nv;
   if (any) new_nv = std::max<u64>(new_nv, maxid + 1);
-  if (g->nranks > 1) DG_TRY(dg::router_max_u64(g, &new_nv, s));
+  if (g->router) DG_TRY(dg::router_max_u64(g, &new_nv, s));
   if (new_nv <= g->nv) return DG_OK;  // Q12: existing IDs are a no-op
   if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   g->snap_pending = false;
@@ -694,7 +716,7 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
   DG_TRY(stage_in(g, 5, ids, n * 4, s, &di, &host));
   const u32* all_ids = (const u32*)di;
   u64 all_n = n;
-  if (g->nranks > 1) DG_TRY(dg::router_allgather_ids(g, all_ids, n, &all_ids, &all_n, s));
+  if (g->router) DG_TRY(dg::router_allgather_u32(g, all_ids, n, 0, &all_ids, &all_n, s));
   if (all_n == 0) return DG_OK;
   DG_TRY(ensure_bitmap(g, g->nv));
   DG_TRY(ensure_dedup(g, all_n));

@@ -24,9 +24,10 @@ dg_status router_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, ui
                         uint32_t epoch, cudaStream_t s);
 dg_status router_query(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
                        uint8_t* found, uint32_t* wout, uint32_t epoch, cudaStream_t s);
-// all ranks' deleted IDs (the union is the batch)
-dg_status router_allgather_ids(dg_graph g, const uint32_t* ids, uint64_t n, const uint32_t** all,
-                               uint64_t* all_n, cudaStream_t s);
+// concatenation of every rank's array (rank order); slot selects one of two
+// router-owned output buffers (0: ids, 1: a parallel array such as hints)
+dg_status router_allgather_u32(dg_graph g, const uint32_t* data, uint64_t n, int slot,
+                               const uint32_t** all, uint64_t* all_n, cudaStream_t s);
 dg_status router_sum_u64(dg_graph g, uint64_t* v, cudaStream_t s);
 dg_status router_max_u64(dg_graph g, uint64_t* v, cudaStream_t s);
 

@@ -69,7 +69,7 @@ class Graph:
                  bucket_bytes: int = 128, directed: bool = True, pool_bytes: int = 0,
                  device: int | None = None, rank: int = 0, nranks: int = 1,
                  nccl_unique_id: bytes | None = None, reuse_tombstones: bool = True,
-                 stream=None):
+                 force_router: bool = False, stream=None):
         cfg = dg_config()
         lib.dg_config_init(ctypes.byref(cfg))
         cfg.load_factor = float(load_factor)
@@ -81,7 +81,8 @@ class Graph:
         cfg.device = int(device)
         cfg.rank = int(rank)
         cfg.nranks = int(nranks)
-        cfg.flags = 0 if reuse_tombstones else _lib.DG_FLAG_NO_TOMBSTONE_REUSE
+        cfg.flags = (0 if reuse_tombstones else _lib.DG_FLAG_NO_TOMBSTONE_REUSE) | \
+            (_lib.DG_FLAG_FORCE_ROUTER if force_router else 0)
         self._uid = None
         if nccl_unique_id is not None:
             self._uid = ctypes.create_string_buffer(bytes(nccl_unique_id), 128)

@@ -1,0 +1,112 @@
+"""Multi-rank host logic on CPU (gloo, world_size 2; -m "not gpu").
+
+Pins the router's semantics before any GPU runs (SURVEY §8(c) "sharded ==
+unsharded"): every edge op is executed only by owner(u) = u mod P, each rank feeds
+its own slice of every batch, ops travel by an all-to-all exchange, vertex
+deletions are all-gathered; the union of the P shards must equal the unsharded
+oracle on the same stream.  Also checks the NCCL-id bootstrap the Python binding
+uses (rank 0's dg_get_unique_id broadcast over the process group)."""
+import os
+import socket
+
+import numpy as np
+import pytest
+import torch
+import torch.distributed as dist
+import torch.multiprocessing as mp
+
+import workloads as wl
+
+
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _exchange(arrs, owner, P):
+    """all-to-all of the SoA arrays by owner rank (gloo)."""
+    order = np.argsort(owner, kind="stable")
+    counts = np.bincount(owner, minlength=P)
+    send_counts = torch.tensor(counts, dtype=torch.int64)
+    recv_counts = torch.empty(P, dtype=torch.int64)
+    dist.all_to_all_single(recv_counts, send_counts)
+    out = []
+    for a in arrs:
+        src = torch.from_numpy(a[order].astype(np.int64))
+        dst = torch.empty(int(recv_counts.sum()), dtype=torch.int64)
+        dist.all_to_all_single(dst, src, recv_counts.tolist(), counts.tolist())
+        out.append(dst.numpy().astype(np.uint32))
+    return out
+
+
+def _worker(rank, P, port, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=P)
+    try:
+        from oracle import Oracle
+        # NCCL id bootstrap as done by bench.py / the binding
+        from paper_conf_ipps_awadapo20_b200 import get_unique_id
+        obj = [get_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        assert isinstance(obj[0], bytes) and len(obj[0]) == 128
+        nv = 3000
+        o = Oracle(nv)  # holds only rows u with u % P == rank
+        for b in range(4):
+            n = 20_000
+            off, cnt = n * rank // P, n * (rank + 1) // P - n * rank // P
+            s, d, w = wl.uniform_edges(41, b, cnt, nv, offset=off)
+            rs, rd, rw = _exchange([s, d, w], s % P, P)
+            assert (rs % P == rank).all()
+            o.insert_edges(rs, rd, rw)
+        ds, dd, _ = wl.uniform_edges(41, 1, 5000, nv, offset=rank * 5000)
+        rs, rd = _exchange([ds, dd], ds % P, P)
+        o.delete_edges(rs, rd)
+        ids = wl.uniform_u32(41, 7, 20, nv, offset=rank * 20)
+        allids = [None] * P
+        dist.all_gather_object(allids, ids)
+        o.delete_vertices(np.concatenate(allids))
+        ro, dd_, ww = o.export()
+        q.put((rank, ro, dd_, ww))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_sharded_oracle_equals_unsharded():
+    from oracle import Oracle
+    P = 2
+    port = _free_port()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_worker, args=(r, P, port, q)) for r in range(P)]
+    for p in procs:
+        p.start()
+    res = {}
+    for _ in range(P):
+        r, ro, dd, ww = q.get(timeout=300)
+        res[r] = (ro, dd, ww)
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    nv = 3000
+    o = Oracle(nv)
+    for b in range(4):
+        s, d, w = wl.uniform_edges(41, b, 20_000, nv)
+        o.insert_edges(s, d, w)
+    ds, dd, _ = wl.uniform_edges(41, 1, 5000 * P, nv)
+    o.delete_edges(ds, dd)
+    o.delete_vertices(wl.uniform_u32(41, 7, 20 * P, nv))
+    ro_g, d_g, w_g = o.export()
+    for u in range(nv):
+        k = u % P
+        ro, dd_, ww = res[k]
+        a, b = int(ro[u]), int(ro[u + 1])
+        ga, gb = int(ro_g[u]), int(ro_g[u + 1])
+        assert np.array_equal(dd_[a:b], d_g[ga:gb]), u
+        assert np.array_equal(ww[a:b], w_g[ga:gb]), u
+        # rows not owned by k are empty on k
+        other = res[1 - k][0]
+        assert other[u + 1] == other[u]
