@@ -209,12 +209,16 @@ DG_API dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream);
  * (synchronises): DG_ERR_VERTEX_OUT_OF_RANGE if any was rejected, else DG_OK. */
 DG_API dg_status dg_batch_status(dg_graph g, void* stream);
 
-/* Triangle count of an undirected (directed = 0) graph by per-vertex hash
- * intersection (§VI-C): for every vertex u and every pair v, w of
- * its higher-ranked neighbours (rank = (degree, id)), probe A_v for w.  Each
- * triangle is counted once.  *count (host) receives the total; synchronises.
- * Requires nranks == 1 (multi-GPU triangle counting runs one replica per GPU). */
-DG_API dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream);
+/* Triangle count of a symmetric graph (undirected mode, directed = 0) by per-vertex
+ * hash intersection (§VI-C): orient every edge from lower to higher rank,
+ * rank(x) = (degree, id); for every vertex u and every pair v, w of its
+ * higher-ranked neighbours, probe the hash table of v for w.  Each triangle is
+ * counted once.  Work is split by u mod nparts: *count (host) receives the count
+ * of part `part` (0 <= part < nparts); the sum over all parts is the total (one
+ * replica per GPU, the caller sums, e.g. with an all-reduce).  Synchronises.
+ * Requires nranks == 1 (each GPU holds a whole replica). */
+DG_API dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t* count,
+                                   void* stream);
 
 /* ------------------------------------------------------------ instrumentation --
  * Off by default; used by bench.py.  While enabled, every probe-kernel launch of an
@@ -222,8 +226,9 @@ DG_API dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream);
  * CUDA events on the call's stream. */
 typedef struct dg_profile {
   uint64_t launches;          /* kernels launched by libdg in this process since enable */
-  uint64_t kernel_launches[4];/* timed launches: [0] insert, [1] delete, [2] query, [3] vertex purge */
-  double kernel_ms[4];        /* their summed device durations in ms */
+  uint64_t kernel_launches[5];/* timed launches: [0] insert, [1] delete, [2] query,
+                                 [3] vertex purge, [4] triangle-count wedge probes */
+  double kernel_ms[5];        /* their summed device durations in ms */
   uint64_t last_count;        /* n_added / n_removed of the most recent insert/delete batch */
 } dg_profile;
 

@@ -64,8 +64,8 @@ class dg_stats(ctypes.Structure):
 class dg_profile(ctypes.Structure):
     _fields_ = [
         ("launches", ctypes.c_uint64),
-        ("kernel_launches", ctypes.c_uint64 * 4),
-        ("kernel_ms", ctypes.c_double * 4),
+        ("kernel_launches", ctypes.c_uint64 * 5),
+        ("kernel_ms", ctypes.c_double * 5),
         ("last_count", ctypes.c_uint64),
     ]
 
@@ -87,7 +87,7 @@ SIGNATURES = [
     ("dg_degrees", ctypes.c_int, [VP, VP, VP]),
     ("dg_get_stats", ctypes.c_int, [VP, ctypes.POINTER(dg_stats), VP]),
     ("dg_batch_status", ctypes.c_int, [VP, VP]),
-    ("dg_triangle_count", ctypes.c_int, [VP, P_U64, VP]),
+    ("dg_triangle_count", ctypes.c_int, [VP, U32, U32, P_U64, VP]),
     ("dg_profile_enable", ctypes.c_int, [VP, ctypes.c_int]),
     ("dg_profile_read", ctypes.c_int, [VP, ctypes.POINTER(dg_profile), VP]),
 ]

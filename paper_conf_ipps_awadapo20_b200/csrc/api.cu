@@ -395,6 +395,8 @@ static void destroy_graph(dg_graph g) {
   if (g->small_dev) cudaFree(g->small_dev);
   for (auto& b : g->stage)
     if (b.p) cudaFree(b.p);
+  for (auto& b : g->tc)
+    if (b.p) cudaFree(b.p);
   cudaGetLastError();
   delete g;
 }
@@ -833,11 +835,50 @@ dg_status dg_batch_status(dg_graph g, void* stream) {
   return st;
 }
 
-dg_status dg_triangle_count(dg_graph g, uint64_t* count, void* stream) {
+dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t* count,
+                            void* stream) {
   DG_TRY(check_handle(g));
-  (void)count;
-  (void)stream;
-  return DG_ERR_UNSUPPORTED;
+  if (!count || nparts == 0 || part >= nparts) return DG_ERR_INVALID_ARGUMENT;
+  if (g->nranks != 1) return DG_ERR_UNSUPPORTED;
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  *count = 0;
+  const dg::Tables t = g->tables();
+  const u64 rows = g->rows;
+  // (1) adjacency export (a12): CSR of every A_u
+  DG_CK(ensure_buf(g->tc[0], (rows + 1) * 8));
+  u64* ro = reinterpret_cast<u64*>(g->tc[0].p);
+  DG_CK(dg::launch_export_offsets(t, ro, &g->scan_temp, &g->scan_bytes, s));
+  u64 m = 0;
+  DG_CK(cudaMemcpyAsync(&m, ro + rows, 8, cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaStreamSynchronize(s));
+  if (m >= 0xFFFFFFFFull) return DG_ERR_UNSUPPORTED;
+  DG_CK(ensure_buf(g->tc[1], m * 4 + 4));
+  u32* dst = reinterpret_cast<u32*>(g->tc[1].p);
+  DG_CK(dg::launch_export_fill(g->G, t, ro, dst, nullptr, g->sms, s));
+  // (2) orientation by rank = (degree, id)
+  DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8));
+  DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8));
+  u64* ocnt = reinterpret_cast<u64*>(g->tc[2].p);
+  u64* oro = reinterpret_cast<u64*>(g->tc[3].p);
+  DG_CK(dg::launch_tc_orient_count(t, ro, dst, part, nparts, ocnt, g->sms, s));
+  DG_CK(dg::scan_exclusive_u64(ocnt, oro, rows + 1, &g->scan_temp, &g->scan_bytes, s));
+  u64 mo = 0;
+  DG_CK(cudaMemcpyAsync(&mo, oro + rows, 8, cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaStreamSynchronize(s));
+  DG_CK(ensure_buf(g->tc[4], mo * 4 + 4));
+  DG_CK(ensure_buf(g->tc[5], mo * 4 + 4));
+  u32* oadj = reinterpret_cast<u32*>(g->tc[4].p);
+  u32* oend = reinterpret_cast<u32*>(g->tc[5].p);
+  DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, g->sms, s));
+  // (3) one edgeExist per wedge
+  DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
+  dg::prof_mark(g, dg::PROF_TC, s);
+  DG_CK(dg::launch_tc_wedges(g->G, t, oadj, oend, mo,
+                             reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
+  dg::prof_mark(g, dg::PROF_TC, s);
+  DG_TRY(read_ctl(g, s));
+  *count = g->hctl->count;
+  return DG_OK;
 }
 
 dg_status dg_profile_enable(dg_graph g, int enable) {
@@ -857,7 +898,7 @@ dg_status dg_profile_read(dg_graph g, dg_profile* out, void* stream) {
   if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   g->snap_pending = false;
   DG_TRY(read_ctl(g, s));
-  for (int k = 0; k < 4; ++k) {
+  for (int k = 0; k < 5; ++k) {
     auto& v = g->prof_ev[k];
     for (size_t i = 0; i + 1 < v.size(); i += 2) {
       float ms = 0.f;

@@ -58,13 +58,14 @@ struct dg_graph_s {
     void* p = nullptr;
     size_t bytes = 0;
   } stage[8];
+  Buf tc[6];  // triangle counting scratch (CSR, orientation)
 
   dg::Router* router = nullptr;
 
   // instrumentation (dg_profile_*)
   bool prof = false;
   uint64_t prof_launch0 = 0;
-  std::vector<cudaEvent_t> prof_ev[4];  // start/stop pairs per kernel kind
+  std::vector<cudaEvent_t> prof_ev[5];  // start/stop pairs per kernel kind
 
   dg::Tables tables() const {
     dg::Tables t;
@@ -86,7 +87,7 @@ inline uint64_t rows_for(uint64_t nv, uint32_t nranks, uint32_t rank) {
   return nv > rank ? (nv - rank + nranks - 1) / nranks : 0;
 }
 
-enum ProfKind { PROF_INSERT = 0, PROF_DELETE = 1, PROF_QUERY = 2, PROF_VDEL = 3 };
+enum ProfKind { PROF_INSERT = 0, PROF_DELETE = 1, PROF_QUERY = 2, PROF_VDEL = 3, PROF_TC = 4 };
 // record an event of kind k on s if instrumentation is enabled
 void prof_mark(dg_graph g, int k, cudaStream_t s);
 

@@ -77,7 +77,12 @@ cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoc
                               cudaStream_t s);
 
 // triangle counting consumer (kernels_tc.cu)
-cudaError_t launch_tc(int G, const Tables& t, const u64* ro, const u32* adj, u32 part,
-                      u32 nparts, int sms, cudaStream_t s);
+cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* dst, u32 part,
+                                   u32 nparts, u64* ocnt, int sms, cudaStream_t s);
+cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
+                                  u32 nparts, const u64* oro, u32* oadj, u32* oend, int sms,
+                                  cudaStream_t s);
+cudaError_t launch_tc_wedges(int G, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
+                             unsigned long long* count, int sms, cudaStream_t s);
 
 }  // namespace dg

@@ -251,7 +251,7 @@ class Graph:
         return st
 
     # ------------------------------------------------------- instrumentation --
-    PROFILE_KINDS = ("insert", "delete", "query", "vertex_purge")
+    PROFILE_KINDS = ("insert", "delete", "query", "vertex_purge", "tc")
 
     def profile_enable(self, enable: bool = True):
         check(lib.dg_profile_enable(self._h, 1 if enable else 0), "dg_profile_enable")
@@ -263,9 +263,10 @@ class Graph:
                 "kernel_launches": dict(zip(self.PROFILE_KINDS, list(p.kernel_launches))),
                 "kernel_ms": dict(zip(self.PROFILE_KINDS, list(p.kernel_ms)))}
 
-    def triangle_count(self, stream=None) -> int:
+    def triangle_count(self, part: int = 0, nparts: int = 1, stream=None) -> int:
+        """Triangles by hash intersection (§VI-C); part/nparts split the work by u mod nparts."""
         c = ctypes.c_uint64()
-        check(lib.dg_triangle_count(self._h, ctypes.byref(c), _stream(stream)),
+        check(lib.dg_triangle_count(self._h, part, nparts, ctypes.byref(c), _stream(stream)),
               "dg_triangle_count")
         return c.value
 

@@ -390,3 +390,52 @@ def test_multi_gpu_torchrun():
                         os.path.join(root, "tests", "multigpu_worker.py")],
                        capture_output=True, text=True, timeout=900, cwd=root)
     assert r.returncode == 0 and "MULTIGPU OK" in r.stdout, r.stdout[-2000:] + r.stderr[-4000:]
+
+
+# ------------------------------------------------------------- triangle count --
+def _golden_triangles():
+    from tests.golden_script import load as _load
+    out = []
+    for ln in _load("triangles.txt"):
+        f = ln.split()
+        out.append((f[0], int(f[1]), int(f[2]), [tuple(int(x) for x in e.split("-")) for e in f[3:]]))
+    return out
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+def test_tc_golden_and_closed_forms(bb):
+    import math
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    for name, n, want, edges in _golden_triangles():
+        g = Graph(n, directed=False, bucket_bytes=bb)
+        g.insert_edges(cuda([e[0] for e in edges]), cuda([e[1] for e in edges]))
+        assert g.triangle_count() == want, name
+    for n in (3, 10, 47):
+        iu, ju = np.triu_indices(n, 1)
+        g = Graph(n, directed=False, bucket_bytes=bb)
+        g.insert_edges(cuda(iu), cuda(ju))
+        assert g.triangle_count() == math.comb(n, 3)
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+def test_tc_matches_oracle_rmat(bb):
+    """Hash-intersection TC (GPU) vs the forward algorithm on sorted lists (oracle)
+    on a symmetrised R-MAT graph; the part/nparts split sums to the total."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    scale = 15
+    nv = 1 << scale
+    s, d = wl.rmat_edges(5, 0, 400_000, scale, wl.GRAPH500)
+    g = Graph(nv, wl.out_degrees(np.concatenate([s, d]), nv), directed=False, bucket_bytes=bb)
+    o = Oracle(nv, directed=False)
+    g.insert_edges(cuda(s), cuda(d))
+    o.insert_edges(s, d)
+    check_against_oracle(g, o, "sym rmat")
+    want = o.triangle_count()
+    assert want > 1000
+    assert g.triangle_count() == want
+    assert sum(g.triangle_count(p, 3) for p in range(3)) == want
+    # dynamic: insert a new batch, recount (config 5 iteration)
+    s2, d2 = wl.rmat_edges(5, 1, 100_000, scale, wl.GRAPH500)
+    g.insert_edges(cuda(s2), cuda(d2))
+    o.insert_edges(s2, d2)
+    assert g.triangle_count() == o.triangle_count()
