@@ -728,16 +728,21 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
   DG_CK(dg::launch_vdel_mark(all_ids, all_n, g->nv, epoch, g->bitmap, g->dedup, g->ctl, g->nranks,
                              g->rank, g->sms, s));
   static const bool force_sweep = std::getenv("DG_FORCE_SWEEP") != nullptr;
+  // base-bucket offsets of the distinct deleted vertices (flattened purge work)
+  DG_CK(ensure_buf(g->stage[7], (all_n + 1) * 8 * 2));
+  u64* nbarr = reinterpret_cast<u64*>(g->stage[7].p);
+  u64* boff = nbarr + (all_n + 1);
+  DG_CK(dg::launch_vdel_nb(t, g->dedup, all_n, nbarr, g->sms, s));
+  DG_CK(dg::scan_exclusive_u64(nbarr, boff, all_n + 1, &g->scan_temp, &g->scan_bytes, s));
   dg::prof_mark(g, dg::PROF_VDEL, s);
   if (!g->directed && g->nranks == 1 && !force_sweep) {
     // undirected: Alg. 2 — delete u from the tables of its neighbours
-    DG_CK(dg::launch_vdel_neighbors(g->G, t, g->dedup, epoch, g->sms, s));
-    DG_CK(cudaMemsetAsync(&g->ctl->queue, 0, sizeof(u32), s));
+    DG_CK(dg::launch_vdel_neighbors(g->G, t, g->dedup, boff, epoch, g->sms, s));
   } else {
     // directed: follow-up sweep over all tables
     DG_CK(dg::launch_vdel_sweep(g->G, t, g->bitmap, epoch, g->sms, s));
   }
-  DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, epoch, g->sms, s));
+  DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, boff, epoch, g->sms, s));
   dg::prof_mark(g, dg::PROF_VDEL, s);
   if (host) {
     if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));

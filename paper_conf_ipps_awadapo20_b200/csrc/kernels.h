@@ -71,10 +71,13 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
                              DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s);
 cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epoch, int sms,
                               cudaStream_t s);
-cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
-                                  cudaStream_t s);
-cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
-                              cudaStream_t s);
+// nbarr[k] = base buckets of the k-th distinct deleted vertex (0 past the count), k <= n_max
+cudaError_t launch_vdel_nb(const Tables& t, const u32* dedup, u64 n_max, u64* nbarr, int sms,
+                           cudaStream_t s);
+cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, const u64* boff,
+                                  u32 epoch, int sms, cudaStream_t s);
+cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
+                              int sms, cudaStream_t s);
 
 // triangle counting consumer (kernels_tc.cu)
 cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* dst, u32 part,

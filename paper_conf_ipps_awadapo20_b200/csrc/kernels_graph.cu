@@ -306,21 +306,34 @@ template <int G>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     u32 epoch) {
   constexpr int W = Group<G>::W;
+  constexpr int U = 4;  // buckets in flight per group (memory-level parallelism)
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
-  for (u64 b = gid; b < nbk; b += ng) {
-    u32* bp = t.pool + b * W + 4 * g.gl;
-    const uint4 q = *reinterpret_cast<const uint4*>(bp);
-    const u32 owner = g.shfl(q.w, G - 1);
-    const bool h0 = q.x < kTomb && ((__ldg(bitmap + (q.x >> 5)) >> (q.x & 31)) & 1u);
-    const bool h1 = !g.last() && q.z < kTomb && ((__ldg(bitmap + (q.z >> 5)) >> (q.z & 31)) & 1u);
-    u32 dec = 0;
-    if (h0 && atomicCAS(bp, q.x, kTomb) == q.x) ++dec;
-    if (h1 && atomicCAS(bp + 2, q.z, kTomb) == q.z) ++dec;
-    if (dec) atomicSub(&t.dir[owner].deg, dec);
+  for (u64 b0 = gid; b0 < nbk; b0 += ng * U) {
+    uint4 q[U];
+#pragma unroll
+    for (int k = 0; k < U; ++k) {
+      const u64 b = b0 + (u64)k * ng;
+      q[k] = b < nbk ? *reinterpret_cast<const uint4*>(t.pool + b * W + 4 * g.gl)
+                     : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+    }
+#pragma unroll
+    for (int k = 0; k < U; ++k) {
+      const u64 b = b0 + (u64)k * ng;
+      u32* bp = t.pool + b * W + 4 * g.gl;
+      const uint4 x = q[k];
+      const u32 owner = g.shfl(x.w, G - 1);
+      const bool h0 = x.x < kTomb && ((__ldg(bitmap + (x.x >> 5)) >> (x.x & 31)) & 1u);
+      const bool h1 =
+          !g.last() && x.z < kTomb && ((__ldg(bitmap + (x.z >> 5)) >> (x.z & 31)) & 1u);
+      u32 dec = 0;
+      if (h0 && atomicCAS(bp, x.x, kTomb) == x.x) ++dec;
+      if (h1 && atomicCAS(bp + 2, x.z, kTomb) == x.z) ++dec;
+      if (dec) atomicSub(&t.dir[owner].deg, dec);
+    }
   }
 }
 
@@ -360,53 +373,83 @@ __device__ __forceinline__ int purge_delete(const Tables& t, const Group<G>& g, 
   }
 }
 
-// Undirected purge, Alg. 2: a group takes the next deleted
-// vertex u from an atomic queue (Alg2:L3-6), iterates over A_u (L11-12) and
-// deletes u from A_v of every neighbour v (L13-17).  Valid only for graphs kept
-// symmetric (directed = 0, single rank).
+// The per-vertex purge kernels below are flattened to one group per (deleted
+// vertex, base bucket): boff[k] = sum of the base-bucket counts of the first k
+// distinct deleted vertices, so a hub's thousands of base buckets are cleared in
+// parallel instead of by one group (the paper balances per vertex with an atomic
+// queue, Alg2:L3-6; a bucket-granular split also balances hubs).
+__global__ void k_vdel_nb(const u32* dedup, const DevCtl* ctl, u64 n_max, const DirEntry* dir,
+                          u32 nranks, u64* nbarr) {
+  const u32 cnt = ctl->dedup_count;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k <= n_max; k += stride)
+    nbarr[k] = k < cnt ? (u64)dir[dedup[k] / nranks].nb : 0ull;
+}
+
+cudaError_t launch_vdel_nb(const Tables& t, const u32* dedup, u64 n_max, u64* nbarr, int sms,
+                           cudaStream_t s) {
+  u64 blocks = (n_max + 1 + 255) / 256;
+  if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  k_vdel_nb<<<(unsigned)blocks, 256, 0, s>>>(dedup, t.ctl, n_max, t.dir, t.nranks, nbarr); note_kernel(1);
+  return cudaGetLastError();
+}
+
+// largest k < cnt with boff[k] <= x
+__device__ __forceinline__ u32 owner_of(const u64* boff, u32 cnt, u64 x) {
+  u32 lo = 0, hi = cnt;  // boff[lo] <= x < boff[hi] (boff[cnt] = total)
+  while (hi - lo > 1) {
+    const u32 mid = (lo + hi) >> 1;
+    if (boff[mid] <= x) lo = mid;
+    else hi = mid;
+  }
+  return lo;
+}
+
+// Undirected purge, Alg. 2: for every deleted vertex u,
+// iterate over A_u (L11-12) and delete u from A_v of every neighbour v (L13-17).
+// Valid only for graphs kept symmetric (directed = 0, single rank).
 template <int G>
-__global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* dedup, u32 epoch) {
+__global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* dedup,
+                                                        const u64* boff, u32 epoch) {
   constexpr int W = Group<G>::W;
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
-  while (true) {
-    u32 qi = 0;
-    if (g.gl == 0) qi = atomicAdd(&t.ctl->queue, 1u);
-    qi = g.shfl(qi, 0);
-    if (qi >= cnt) break;
-    const u32 u = dedup[qi];
-    const DirEntry de = t.dir[u];
-    for (u32 k = 0; k < de.nb; ++k) {
-      u32 b = de.base + k;
-      while (b != kNil) {
-        const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
-        u32 lm0 = g.ballot(q.x < kTomb);
-        u32 lm1 = g.ballot(!g.last() && q.z < kTomb);
-        while (lm0 | lm1) {
-          const u32 l = __ffs(lm0 | lm1) - 1;
-          const bool s0 = (lm0 >> l) & 1u;
-          const u32 x0 = g.shfl(q.x, l), x1 = g.shfl(q.z, l);
-          const u32 v = s0 ? x0 : x1;
-          if (s0) lm0 &= ~(1u << l);
-          else lm1 &= ~(1u << l);
-          const DirEntry dv = t.dir[v];
-          if (purge_delete<G>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
-            atomicSub(&t.dir[v].deg, 1u);
-        }
-        b = g.shfl(q.z, G - 1);
+  if (cnt == 0) return;
+  const u64 total = boff[cnt];
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  for (u64 x = gid; x < total; x += ng) {
+    const u32 k = owner_of(boff, cnt, x);
+    const u32 u = dedup[k];
+    u32 b = t.dir[u].base + (u32)(x - boff[k]);
+    while (b != kNil) {
+      const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
+      u32 lm0 = g.ballot(q.x < kTomb);
+      u32 lm1 = g.ballot(!g.last() && q.z < kTomb);
+      while (lm0 | lm1) {
+        const u32 l = __ffs(lm0 | lm1) - 1;
+        const bool s0 = (lm0 >> l) & 1u;
+        const u32 x0 = g.shfl(q.x, l), x1 = g.shfl(q.z, l);
+        const u32 v = s0 ? x0 : x1;
+        if (s0) lm0 &= ~(1u << l);
+        else lm1 &= ~(1u << l);
+        const DirEntry dv = t.dir[v];
+        if (purge_delete<G>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
+          atomicSub(&t.dir[v].deg, 1u);
       }
+      b = g.shfl(q.z, G - 1);
     }
   }
 }
 
-cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
-                                  cudaStream_t s) {
+cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, const u64* boff,
+                                  u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (G) {
-    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
-    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
-    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
@@ -415,46 +458,46 @@ cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, u32 
 // Owner clear (Alg2:L18-22): walk A_u; chained buckets are reset to EMPTY and
 // pushed on the free stack (dynamic memory reclaimed); base buckets
 // are reset to EMPTY in place (Q9: static memory is kept but must not keep stale
-// keys); degree := 0.
+// keys); degree := 0.  One group per (vertex, base bucket).
 template <int G>
-__global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, u32 epoch) {
+__global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, const u64* boff,
+                                                    u32 epoch) {
   constexpr int W = Group<G>::W;
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
+  if (cnt == 0) return;
+  const u64 total = boff[cnt];
   const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
-  while (true) {
-    u32 qi = 0;
-    if (g.gl == 0) qi = atomicAdd(&t.ctl->queue, 1u);
-    qi = g.shfl(qi, 0);
-    if (qi >= cnt) break;
-    const u32 row = dedup[qi] / t.nranks;
-    const DirEntry de = t.dir[row];
-    for (u32 k = 0; k < de.nb; ++k) {
-      u32 b = de.base + k;
-      bool base_bucket = true;
-      while (b != kNil) {
-        u32* bp = t.pool + (u64)b * W + 4 * g.gl;
-        const uint4 q = ld_relaxed_v4(bp);
-        const u32 next = g.shfl(q.z, G - 1);
-        if (g.last()) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
-        else st_v4(bp, empty4);
-        if (!base_bucket && g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
-        base_bucket = false;
-        b = next;
-      }
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  for (u64 x = gid; x < total; x += ng) {
+    const u32 k = owner_of(boff, cnt, x);
+    const u32 row = dedup[k] / t.nranks;
+    const u32 j = (u32)(x - boff[k]);
+    u32 b = t.dir[row].base + j;
+    bool base_bucket = true;
+    while (b != kNil) {
+      u32* bp = t.pool + (u64)b * W + 4 * g.gl;
+      const uint4 q = ld_relaxed_v4(bp);
+      const u32 next = g.shfl(q.z, G - 1);
+      if (g.last()) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
+      else st_v4(bp, empty4);
+      if (!base_bucket && g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
+      base_bucket = false;
+      b = next;
     }
-    if (g.gl == 0) t.dir[row].deg = 0;
+    if (j == 0 && g.gl == 0) t.dir[row].deg = 0;
   }
 }
 
-cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, u32 epoch, int sms,
-                              cudaStream_t s) {
+cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
+                              int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (G) {
-    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
-    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
-    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, epoch); note_kernel(1); break;
+    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();
