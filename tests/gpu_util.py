@@ -74,3 +74,31 @@ def check_queries(g, o: Oracle, qs, qd, cand=None, where=""):
         cand = Candidates(*o.candidates())
     errs = compare_queries(qs, qd, f.cpu().numpy(), w.cpu().numpy(), rf, rw, cand)
     assert not errs, f"{where}: {errs}"
+
+
+def gpu_invariants(ro, dst, deg):
+    """Size-independent invariants on a full export, computed with torch on the GPU
+    (test-side checking only): no duplicate (u, v), no self-loop, degree == row length.
+    ro: uint64 [V+1], dst: uint32 [E], deg: uint32 [V] (device tensors)."""
+    ro64 = ro.to(torch.int64)
+    lens = ro64[1:] - ro64[:-1]
+    errs = []
+    if not torch.equal(lens, deg.to(torch.int64)):
+        errs.append("degree != row length")
+    rows = torch.repeat_interleave(torch.arange(lens.numel(), device=ro.device), lens)
+    d64 = dst.to(torch.int64)
+    if bool((rows == d64).any()):
+        errs.append("self-loop stored")
+    keys = torch.sort((rows << 32) | d64).values
+    if keys.numel() > 1 and bool((keys[1:] == keys[:-1]).any()):
+        errs.append("duplicate edge stored")
+    return errs
+
+
+def distinct_nonloop(s, d):
+    """number of distinct (u, v) keys with u != v (torch.unique on the GPU)."""
+    ts = torch.from_numpy(np.ascontiguousarray(s).astype(np.int64)).cuda()
+    td = torch.from_numpy(np.ascontiguousarray(d).astype(np.int64)).cuda()
+    k = (ts << 32) | td
+    k = k[ts != td]
+    return int(torch.unique(k).numel())
