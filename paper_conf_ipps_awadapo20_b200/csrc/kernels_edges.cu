@@ -69,169 +69,213 @@ __device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 stack_size) {
 //   inserts of one key always contend for the same slot.
 enum { ACT_NONE = 0, ACT_CAS_DEL = 1, ACT_CAS_INS = 2, ACT_EXTEND = 3 };
 
-template <int G, int OP>
-__global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) {
+// One pass of the round loop over the 32 ops of a warp (one per lane).  MAIN:
+// exactly one round; ops that still need work (a chain to walk, a lost CAS, a
+// chain extension) are returned as deferred and re-run from scratch later in a
+// dense backlog chunk, so a few slow ops no longer cost a whole extra round for
+// the other 31 lanes.  !MAIN: rounds until every op of the warp is done.
+template <int G, int OP, bool MAIN>
+__device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, const Group<G>& g,
+                                        const bool valid, const u64 opid, const u64 j,
+                                        const u32 stack_size, const bool reuse, u32& my_count,
+                                        u32& spare, bool& bad_range) {
   constexpr int W = Group<G>::W;
   constexpr u32 FULL = 0xFFFFFFFFu;
   constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
+  const bool lastl = g.last();
+  bool deferred = false;
+  // ---- 1. stage one op per lane
+  u32 u = 0, v = 0, w = 0;
+  if (valid) {
+    u64 i = opid;
+    const bool rev = opid >= a.n;  // undirected mirror op
+    if (rev) i = opid - a.n;
+    u = a.src[i];
+    v = a.dst[i];
+    if (OP == OP_INSERT && a.w) w = a.w[i];
+    if (rev) { const u32 x = u; u = v; v = x; }
+  }
+  bool pend = valid && u != v;  // self-loops are never stored (Alg1:L3)
+  if (OP == OP_QUERY && valid && ((u64)u >= a.nv || (u64)v >= a.nv)) {
+    pend = false;
+    bad_range = true;
+  }
+  const u32 row = (t.nranks == 1) ? u : u / t.nranks;
+  u32 head = 0;
+  if (pend) {
+    // base/nb never change during an edge phase; only deg is written (atomics)
+    const uint4 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
+    head = de.x + bucket_of(v, de.y);
+  }
+  u32 cur = head;
+  bool found = false;
+  u32 val = 0;
+  u32* ff = nullptr;               // insert: first free slot of the chain (pair address)
+  unsigned long long ffo = 0;      //         and its contents when scanned
+
+  // ---- 2. rounds
+  while (true) {
+    const u32 pm = __ballot_sync(FULL, pend);
+    if (pm == 0) break;
+    // a. current buckets of the group's pending ops
+    uint4 q[G];
+#pragma unroll
+    for (int r = 0; r < G; ++r) {
+      const u32 cr = __shfl_sync(FULL, cur, g.base + r);
+      const u32* p = t.pool + (u64)cr * W + 4 * g.gl;
+      if ((pm >> (g.base + r)) & 1u) q[r] = (OP == OP_QUERY) ? ld_nc_v4(p) : ld_relaxed_v4(p);
+      else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+    }
+    // b. decide
+    int act = ACT_NONE;
+#pragma unroll
+    for (int r = 0; r < G; ++r) {
+      const uint4 x = q[r];
+      const u32 srcl = g.base + r;
+      const bool pr = (pm >> srcl) & 1u;
+      const u32 vr = __shfl_sync(FULL, v, srcl);
+      const u32 cr = __shfl_sync(FULL, cur, srcl);
+      u32* bp = t.pool + (u64)cr * W + 4 * g.gl;
+      const bool m0 = pr && x.x == vr, m1 = pr && !lastl && x.z == vr;
+      const u32 hit = (__ballot_sync(FULL, m0 || m1) >> g.base) & GBITS;
+      const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
+      const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
+      const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
+      const bool end = em != 0 || next == kNil;  // EMPTY slots only exist at the tail
+      const u32 lh = hit ? __ffs(hit) - 1 : 0;
+      const bool mine = pr && g.gl == (u32)r;
+      if (OP == OP_QUERY) {
+        const u32 hv = __shfl_sync(FULL, m0 ? x.y : x.w, g.base + lh);
+        if (mine) {
+          if (hit) { found = true; val = hv; pend = false; }
+          else if (end) pend = false;
+          else cur = next;
+        }
+      } else if (OP == OP_DELETE) {
+        const u64 ka = __shfl_sync(FULL, (unsigned long long)(bp + (m0 ? 0 : 2)), g.base + lh);
+        if (mine) {
+          if (hit) { act = ACT_CAS_DEL; ff = reinterpret_cast<u32*>(ka); }
+          else if (end) pend = false;
+          else cur = next;
+        }
+      } else {  // insert
+        const u32 wr = __shfl_sync(FULL, w, srcl);
+        if (hit && g.gl == lh) st_relaxed_u32(bp + (m0 ? 1 : 3), wr);  // replace
+        const bool f0 = e0 || (reuse && x.x == kTomb);
+        const bool f1 = e1 || (reuse && !lastl && x.z == kTomb);
+        const u32 fm = (__ballot_sync(FULL, f0 || f1) >> g.base) & GBITS;
+        const u32 lf = fm ? __ffs(fm) - 1 : 0;
+        const unsigned long long cont = f0 ? pack_pair(x.x, x.y) : pack_pair(x.z, x.w);
+        const u64 sa = __shfl_sync(FULL, (unsigned long long)(bp + (f0 ? 0 : 2)), g.base + lf);
+        const unsigned long long so = __shfl_sync(FULL, cont, g.base + lf);
+        if (mine) {
+          if (hit) {
+            pend = false;
+          } else {
+            if (!ff && fm) { ff = reinterpret_cast<u32*>(sa); ffo = so; }
+            if (end) act = ff ? ACT_CAS_INS : ACT_EXTEND;
+            else cur = next;
+          }
+        }
+      }
+    }
+    // c. one atomic per lane, all in flight together
+    if (OP == OP_DELETE && act == ACT_CAS_DEL) {
+      if (atomicCAS(ff, v, kTomb) == v) {
+        atomicSub(&t.dir[row].deg, 1u);
+        ++my_count;
+      }
+      pend = false;  // a lost CAS means another op deleted the key (Q5)
+    }
+    if (OP == OP_INSERT && act == ACT_CAS_INS) {
+      const unsigned long long old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
+                                               (unsigned long long)pack_pair(v, w));
+      if (old == ffo) {
+        atomicAdd(&t.dir[row].deg, 1u);
+        ++my_count;
+        pend = false;
+      } else if ((u32)old == v) {  // a racing op installed the same key: replace
+        st_relaxed_u32(ff + 1, w);
+        pend = false;
+      } else {  // the slot went to another key: re-scan from the head
+        cur = head;
+        ff = nullptr;
+      }
+    }
+    if (OP == OP_INSERT && act == ACT_EXTEND) {
+      // chain full: link a new bucket at the tail (a8)
+      if (spare == kNil) spare = alloc_bucket(t, stack_size);
+      if (spare == kNil) {  // pool exhausted: the host grows it and re-runs this op
+        a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
+        pend = false;
+      } else {
+        st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
+        const u32 old = atomicCAS(t.pool + (u64)cur * W + Group<G>::NEXT, kNil, spare);
+        if (old == kNil) {
+          cur = spare;
+          spare = kNil;
+        } else {
+          cur = old;  // another op linked first (no earlier slot can free up); keep ours
+        }
+      }
+    }
+    if (MAIN) {
+      deferred = pend;
+      break;
+    }
+  }
+  if (OP == OP_QUERY && valid && !deferred) {
+    a.found[j] = found ? 1 : 0;
+    if (a.wout) a.wout[j] = found ? val : 0u;
+  }
+  return deferred;
+}
+
+template <int G, int OP>
+__global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) {
+  constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<G> g;
   if (OP != OP_QUERY) {
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
   }
   const u32 stack_size = (OP == OP_INSERT) ? ld_relaxed_u32(&t.ctl->stack_size) : 0u;
   const bool reuse = a.reuse_tombstones != 0;
-  const bool lastl = g.last();
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
   u32 my_count = 0;
   u32 spare = kNil;  // a fresh bucket this lane allocated but could not link
   bool bad_range = false;
-
+  // per-warp backlog of deferred op ids (shared memory)
+  __shared__ unsigned long long backlog[kEdgeBlock / 32][64];
+  unsigned long long* bl = backlog[threadIdx.x >> 5];
+  const u32 below = (1u << g.lane) - 1u;
+  u32 nbl = 0;  // warp-uniform
   for (u64 chunk = warp; chunk * 32 < a.n_ops; chunk += nwarps) {
-    // ---- 1. stage one op per lane
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
-    u64 opid = j;
-    u32 u = 0, v = 0, w = 0;
-    if (valid) {
-      if (a.idx) opid = a.idx[j];
-      u64 i = opid;
-      const bool rev = opid >= a.n;  // undirected mirror op
-      if (rev) i = opid - a.n;
-      u = a.src[i];
-      v = a.dst[i];
-      if (OP == OP_INSERT && a.w) w = a.w[i];
-      if (rev) { const u32 x = u; u = v; v = x; }
+    const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
+    const bool d = run_ops<G, OP, true>(t, a, g, valid, opid, j, stack_size, reuse, my_count,
+                                        spare, bad_range);
+    const u32 dm = __ballot_sync(FULL, d);
+    if (d) bl[nbl + __popc(dm & below)] = OP == OP_QUERY ? j : opid;
+    nbl += __popc(dm);
+    __syncwarp();
+    if (nbl >= 32) {
+      nbl -= 32;
+      const u64 op2 = bl[nbl + g.lane];
+      __syncwarp();
+      run_ops<G, OP, false>(t, a, g, true, op2, op2, stack_size, reuse, my_count, spare,
+                            bad_range);
     }
-    bool pend = valid && u != v;  // self-loops are never stored (Alg1:L3)
-    if (OP == OP_QUERY && valid && ((u64)u >= a.nv || (u64)v >= a.nv)) {
-      pend = false;
-      bad_range = true;
-    }
-    const u32 row = (t.nranks == 1) ? u : u / t.nranks;
-    u32 head = 0;
-    if (pend) {
-      // base/nb never change during an edge phase; only deg is written (atomics)
-      const uint4 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
-      head = de.x + bucket_of(v, de.y);
-    }
-    u32 cur = head;
-    bool found = false;
-    u32 val = 0;
-    u32* ff = nullptr;               // insert: first free slot of the chain (pair address)
-    unsigned long long ffo = 0;      //         and its contents when scanned
-
-    // ---- 2. rounds
-    while (true) {
-      const u32 pm = __ballot_sync(FULL, pend);
-      if (pm == 0) break;
-      // a. current buckets of the group's pending ops
-      uint4 q[G];
-#pragma unroll
-      for (int r = 0; r < G; ++r) {
-        const u32 cr = __shfl_sync(FULL, cur, g.base + r);
-        const u32* p = t.pool + (u64)cr * W + 4 * g.gl;
-        if ((pm >> (g.base + r)) & 1u) q[r] = (OP == OP_QUERY) ? ld_nc_v4(p) : ld_relaxed_v4(p);
-        else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
-      }
-      // b. decide
-      int act = ACT_NONE;
-#pragma unroll
-      for (int r = 0; r < G; ++r) {
-        const uint4 x = q[r];
-        const u32 srcl = g.base + r;
-        const bool pr = (pm >> srcl) & 1u;
-        const u32 vr = __shfl_sync(FULL, v, srcl);
-        const u32 cr = __shfl_sync(FULL, cur, srcl);
-        u32* bp = t.pool + (u64)cr * W + 4 * g.gl;
-        const bool m0 = pr && x.x == vr, m1 = pr && !lastl && x.z == vr;
-        const u32 hit = (__ballot_sync(FULL, m0 || m1) >> g.base) & GBITS;
-        const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
-        const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
-        const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
-        const bool end = em != 0 || next == kNil;  // EMPTY slots only exist at the tail
-        const u32 lh = hit ? __ffs(hit) - 1 : 0;
-        const bool mine = pr && g.gl == (u32)r;
-        if (OP == OP_QUERY) {
-          const u32 hv = __shfl_sync(FULL, m0 ? x.y : x.w, g.base + lh);
-          if (mine) {
-            if (hit) { found = true; val = hv; pend = false; }
-            else if (end) pend = false;
-            else cur = next;
-          }
-        } else if (OP == OP_DELETE) {
-          const u64 ka = __shfl_sync(FULL, (unsigned long long)(bp + (m0 ? 0 : 2)), g.base + lh);
-          if (mine) {
-            if (hit) { act = ACT_CAS_DEL; ff = reinterpret_cast<u32*>(ka); }
-            else if (end) pend = false;
-            else cur = next;
-          }
-        } else {  // insert
-          const u32 wr = __shfl_sync(FULL, w, srcl);
-          if (hit && g.gl == lh) st_relaxed_u32(bp + (m0 ? 1 : 3), wr);  // replace
-          const bool f0 = e0 || (reuse && x.x == kTomb);
-          const bool f1 = e1 || (reuse && !lastl && x.z == kTomb);
-          const u32 fm = (__ballot_sync(FULL, f0 || f1) >> g.base) & GBITS;
-          const u32 lf = fm ? __ffs(fm) - 1 : 0;
-          const unsigned long long cont = f0 ? pack_pair(x.x, x.y) : pack_pair(x.z, x.w);
-          const u64 sa = __shfl_sync(FULL, (unsigned long long)(bp + (f0 ? 0 : 2)), g.base + lf);
-          const unsigned long long so = __shfl_sync(FULL, cont, g.base + lf);
-          if (mine) {
-            if (hit) {
-              pend = false;
-            } else {
-              if (!ff && fm) { ff = reinterpret_cast<u32*>(sa); ffo = so; }
-              if (end) act = ff ? ACT_CAS_INS : ACT_EXTEND;
-              else cur = next;
-            }
-          }
-        }
-      }
-      // c. one atomic per lane, all in flight together
-      if (OP == OP_DELETE && act == ACT_CAS_DEL) {
-        if (atomicCAS(ff, v, kTomb) == v) {
-          atomicSub(&t.dir[row].deg, 1u);
-          ++my_count;
-        }
-        pend = false;  // a lost CAS means another op deleted the key (Q5)
-      }
-      if (OP == OP_INSERT && act == ACT_CAS_INS) {
-        const unsigned long long old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
-                                                 (unsigned long long)pack_pair(v, w));
-        if (old == ffo) {
-          atomicAdd(&t.dir[row].deg, 1u);
-          ++my_count;
-          pend = false;
-        } else if ((u32)old == v) {  // a racing op installed the same key: replace
-          st_relaxed_u32(ff + 1, w);
-          pend = false;
-        } else {  // the slot went to another key: re-scan from the head
-          cur = head;
-          ff = nullptr;
-        }
-      }
-      if (OP == OP_INSERT && act == ACT_EXTEND) {
-        // chain full: link a new bucket at the tail (a8)
-        if (spare == kNil) spare = alloc_bucket(t, stack_size);
-        if (spare == kNil) {  // pool exhausted: the host grows it and re-runs this op
-          a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
-          pend = false;
-        } else {
-          st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
-          const u32 old = atomicCAS(t.pool + (u64)cur * W + Group<G>::NEXT, kNil, spare);
-          if (old == kNil) {
-            cur = spare;
-            spare = kNil;
-          } else {
-            cur = old;  // another op linked first (no earlier slot can free up); keep ours
-          }
-        }
-      }
-    }
-    if (OP == OP_QUERY && valid) {
-      a.found[j] = found ? 1 : 0;
-      if (a.wout) a.wout[j] = found ? val : 0u;
-    }
+  }
+  while (nbl > 0) {  // drain the backlog
+    const u32 take = nbl < 32 ? nbl : 32;
+    nbl -= take;
+    const bool valid = g.lane < take;
+    const u64 op2 = valid ? bl[nbl + g.lane] : 0;
+    __syncwarp();
+    run_ops<G, OP, false>(t, a, g, valid, op2, op2, stack_size, reuse, my_count, spare,
+                          bad_range);
   }
   // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
   if (OP == OP_INSERT && spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
