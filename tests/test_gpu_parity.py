@@ -233,7 +233,8 @@ def test_heavy_intra_batch_duplicates():
 def test_host_buffers_match_device_buffers():
     from paper_conf_ipps_awadapo20_b200 import Graph
     nv = 5000
-    s, d, w = wl.uniform_edges(21, 0, 100_000, nv)
+    s, d, _ = wl.uniform_edges(21, 0, 100_000, nv)
+    w = (s.astype(np.uint64) * 2654435761 ^ d).astype(np.uint32)  # duplicate keys: equal weights (Q1)
     a, b = Graph(nv), Graph(nv)
     assert a.insert_edges(s, d, w, count=True) == b.insert_edges(cuda(s), cuda(d), cuda(w), count=True)
     qs, qd, _ = wl.uniform_edges(21, 1, 50_000, nv)
