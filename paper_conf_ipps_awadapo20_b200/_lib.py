@@ -10,7 +10,7 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libdg.so")
+LIB_PATH = os.environ.get("DG_LIB_PATH") or os.path.join(_HERE, "libdg.so")
 
 DG_OK = 0
 DG_ERR_INVALID_ARGUMENT = 1

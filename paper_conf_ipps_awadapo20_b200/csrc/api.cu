@@ -209,11 +209,11 @@ dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) 
   }
   const u64 missing = need - free_exact;
   static const bool no_upfront = std::getenv("DG_TEST_RETRY_PATH") != nullptr;
-  // Reserve the worst case (one new bucket per op) only when that is small next to
-  // the pool; otherwise launch in retry mode and grow by what actually failed (a
-  // bulk build allocates far fewer buckets than it has ops).
-  const u64 limit = std::min<u64>(std::min<u64>(4ull << 30, device_free_bytes() / 2),
-                                  std::max<u64>(256ull << 20, g->pool.mapped() / 4));
+  // Reserve the worst case (one new bucket per op) up front when it is bounded
+  // (<= 4 GB and half of free device memory): steady-state batches then never
+  // synchronise.  Larger batches (bulk builds) launch in retry mode and grow by what
+  // actually failed.
+  const u64 limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
   if (!no_upfront && missing * g->bucket_bytes <= limit) {
     const u64 want = (u64)g->cap + missing + std::max<u64>(missing / 4, 65536);
     dg_status st = grow_pool(g, want, s);

@@ -231,8 +231,11 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
   return deferred;
 }
 
+#ifndef DG_EDGE_MINB
+#define DG_EDGE_MINB 4
+#endif
 template <int G, int OP>
-__global__ void __launch_bounds__(kEdgeBlock, 4) k_edges(Tables t, EdgeBatch a) {
+__global__ void __launch_bounds__(kEdgeBlock, DG_EDGE_MINB) k_edges(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<G> g;
   if (OP != OP_QUERY) {
