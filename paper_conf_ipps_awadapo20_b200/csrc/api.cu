@@ -401,6 +401,9 @@ static void destroy_graph(dg_graph g) {
     if (b.p) cudaFree(b.p);
   for (auto& b : g->tc)
     if (b.p) cudaFree(b.p);
+  for (auto& cs : g->cstream)
+    if (cs) cudaStreamDestroy(cs);
+  for (cudaEvent_t e : g->pipe_ev) cudaEventDestroy(e);
   cudaGetLastError();
   delete g;
 }
@@ -621,6 +624,50 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
   return DG_OK;
 }
 
+// Host-buffer queries are pipelined in chunks over two internal copy streams: the
+// upload of chunk k+1 and the download of the answers of chunk k-1 overlap the probe
+// kernel of chunk k (PCIe is full duplex).  Queries never mutate, so unlike
+// inserts/deletes they need no batch-wide validation before the first kernel.
+static dg_status query_host_pipelined(dg_graph g, const u32* src, const u32* dst, u64 n,
+                                      uint8_t* found, u32* wout, u32 epoch, cudaStream_t s) {
+  constexpr u64 kChunk = 1ull << 22;
+  const u64 nch = (n + kChunk - 1) / kChunk;
+  DG_CK(ensure_buf(g->stage[0], n * 4));
+  DG_CK(ensure_buf(g->stage[1], n * 4));
+  DG_CK(ensure_buf(g->stage[3], n));
+  if (wout) DG_CK(ensure_buf(g->stage[4], n * 4));
+  for (auto& cs : g->cstream)
+    if (!cs) DG_CK(cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking));
+  while (g->pipe_ev.size() < 2 * nch + 1) {
+    cudaEvent_t e;
+    DG_CK(cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
+    g->pipe_ev.push_back(e);
+  }
+  u32* ds = reinterpret_cast<u32*>(g->stage[0].p);
+  u32* dd = reinterpret_cast<u32*>(g->stage[1].p);
+  uint8_t* df = reinterpret_cast<uint8_t*>(g->stage[3].p);
+  u32* dw = wout ? reinterpret_cast<u32*>(g->stage[4].p) : nullptr;
+  cudaStream_t up = g->cstream[0], down = g->cstream[1];
+  DG_CK(cudaEventRecord(g->pipe_ev[0], s));  // after earlier work on the caller's stream
+  DG_CK(cudaStreamWaitEvent(up, g->pipe_ev[0], 0));
+  for (u64 k = 0; k < nch; ++k) {
+    const u64 off = k * kChunk, cnt = std::min(kChunk, n - off);
+    DG_CK(cudaMemcpyAsync(ds + off, src + off, cnt * 4, cudaMemcpyHostToDevice, up));
+    DG_CK(cudaMemcpyAsync(dd + off, dst + off, cnt * 4, cudaMemcpyHostToDevice, up));
+    DG_CK(cudaEventRecord(g->pipe_ev[1 + 2 * k], up));
+    DG_CK(cudaStreamWaitEvent(s, g->pipe_ev[1 + 2 * k], 0));
+    DG_TRY(dg::local_query(g, ds + off, dd + off, cnt, df + off, dw ? dw + off : nullptr, epoch, s));
+    DG_CK(cudaEventRecord(g->pipe_ev[2 + 2 * k], s));
+    DG_CK(cudaStreamWaitEvent(down, g->pipe_ev[2 + 2 * k], 0));
+    DG_CK(cudaMemcpyAsync(found + off, df + off, cnt, cudaMemcpyDeviceToHost, down));
+    if (wout)
+      DG_CK(cudaMemcpyAsync(wout + off, dw + off, cnt * 4, cudaMemcpyDeviceToHost, down));
+  }
+  DG_CK(cudaStreamSynchronize(down));
+  DG_CK(cudaStreamSynchronize(s));
+  return DG_OK;
+}
+
 dg_status dg_query_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
                          uint8_t* found, uint32_t* weight_out, void* stream) {
   DG_TRY(check_handle(g));
@@ -628,6 +675,14 @@ dg_status dg_query_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, u
   if (n && (!src || !dst || !found)) return DG_ERR_INVALID_ARGUMENT;
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   const u32 epoch = ++g->epoch;
+  if (!g->router && n >= (1ull << 23) && !is_device_ptr(src) && !is_device_ptr(dst) &&
+      !is_device_ptr(found) && (!weight_out || !is_device_ptr(weight_out))) {
+    DG_TRY(query_host_pipelined(g, src, dst, n, found, weight_out, epoch, s));
+    if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+    g->snap_pending = false;
+    DG_TRY(read_ctl(g, s));
+    return status_of(g, epoch);
+  }
   bool host = false;
   const void *ds = nullptr, *dd = nullptr;
   void *df = nullptr, *dw = nullptr;

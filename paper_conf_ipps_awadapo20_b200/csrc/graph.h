@@ -59,6 +59,8 @@ struct dg_graph_s {
     size_t bytes = 0;
   } stage[8];
   Buf tc[6];  // triangle counting scratch (CSR, orientation)
+  cudaStream_t cstream[2] = {nullptr, nullptr};  // host-buffer pipeline: upload, download
+  std::vector<cudaEvent_t> pipe_ev;
 
   dg::Router* router = nullptr;
 

@@ -440,3 +440,29 @@ def test_tc_matches_oracle_rmat(bb):
     g.insert_edges(cuda(s2), cuda(d2))
     o.insert_edges(s2, d2)
     assert g.triangle_count() == o.triangle_count()
+
+
+def test_host_query_pipeline_large():
+    """Host-buffer queries above 2^23 take the chunked upload/probe/download pipeline;
+    answers must equal the device-buffer path and the oracle on a sample."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 200_000
+    s, d, _ = wl.uniform_edges(23, 0, 2_000_000, nv)
+    w = (s.astype(np.uint64) * 2654435761 ^ d).astype(np.uint32)
+    g = Graph(nv)
+    g.insert_edges(cuda(s), cuda(d), cuda(w))
+    n = (1 << 23) + 12345
+    qs, qd, _ = wl.uniform_edges(23, 1, n, nv, weights=False)
+    qs[: 1 << 20], qd[: 1 << 20] = s[: 1 << 20], d[: 1 << 20]
+    fh = np.empty(n, np.uint8)
+    wh = np.empty(n, np.uint32)
+    g.query_edges(qs, qd, found_out=fh, weight_out=wh)
+    fd, wd = g.query_edges(cuda(qs), cuda(qd))
+    assert np.array_equal(fh, fd.cpu().numpy()) and np.array_equal(wh, wd.cpu().numpy())
+    live = s[: 1 << 20] != d[: 1 << 20]  # self-loops are never stored (Alg1:L3)
+    assert fh[: 1 << 20][live].all() and not fh[: 1 << 20][~live].any()
+    o = Oracle(nv)
+    o.insert_edges(s, d, w)
+    idx = np.arange(0, n, 97)
+    st, rf, rw = o.query_edges(qs[idx], qd[idx])
+    assert np.array_equal(rf, fh[idx]) and np.array_equal(rw, wh[idx])
