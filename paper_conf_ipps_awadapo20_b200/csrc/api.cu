@@ -384,6 +384,7 @@ static void destroy_graph(dg_graph g) {
   prof_clear(g);
   if (g->router) dg::router_destroy(g->router);
   g->dir.release();
+  g->degv.release();
   g->pool.release();
   g->stack.release();
   if (g->ctl) cudaFree(g->ctl);
@@ -436,6 +437,9 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
     return st;
   }
   cudaError_t e = g->dir.ensure((row0 + count) * sizeof(dg::DirEntry), 0, s);
+  if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
+  DG_CK(e);
+  e = g->degv.ensure((row0 + count) * sizeof(u32), 0, s);
   if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
   DG_CK(e);
   g->rows = row0 + count;
@@ -495,7 +499,8 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (g->stack.reserve(g->device, total_mem / g->bucket_bytes * 4 + (2u << 20)) != cudaSuccess)
     return fail(DG_ERR_CUDA);
   const u64 max_rows = (kMaxVertices + g->nranks - 1) / g->nranks + 1;
-  if (g->dir.reserve(g->device, max_rows * sizeof(dg::DirEntry)) != cudaSuccess)
+  if (g->dir.reserve(g->device, max_rows * sizeof(dg::DirEntry)) != cudaSuccess ||
+      g->degv.reserve(g->device, max_rows * sizeof(u32)) != cudaSuccess)
     return fail(DG_ERR_CUDA);
   if (cudaMalloc(&g->ctl, sizeof(dg::DevCtl)) != cudaSuccess) return fail(DG_ERR_CUDA);
   if (cudaMemsetAsync(g->ctl, 0, sizeof(dg::DevCtl), s) != cudaSuccess) return fail(DG_ERR_CUDA);
@@ -880,7 +885,7 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   out->live_pairs = h.live;
   out->tombstones = h.tombs;
   out->max_chain = h.max_chain;
-  out->pool_bytes = g->pool.mapped() + g->dir.mapped() + g->stack.mapped();
+  out->pool_bytes = g->pool.mapped() + g->dir.mapped() + g->degv.mapped() + g->stack.mapped();
   out->load_factor = h.linked_buckets ? (double)h.live / ((double)h.linked_buckets * g->BC) : 0.0;
   out->utilization =
       h.linked_buckets ? (double)h.live * 8.0 / ((double)h.linked_buckets * g->bucket_bytes) : 0.0;

@@ -1,8 +1,10 @@
 // dg_common.cuh — device-side layout and primitives shared by the kernels.
 //
 // Data layout in HBM:
-//   directory  : DirEntry[local_rows], 16 B per row {base bucket, #buckets, degree, flags}
-//                (the paper's vertex dictionary)
+//   directory  : DirEntry[local_rows], 8 B per row {base bucket, #base buckets} and
+//   degree     : u32[local_rows], the exact neighbour count (the paper's vertex
+//                dictionary holds both; split so the
+//                read-mostly 8-B entries and the 4-B counters stay L2-resident)
 //   pool       : bucket array; bucket b occupies words [b*W, (b+1)*W), W = bucket_bytes/4.
 //                words 2i, 2i+1 = (key, value) of pair i, i < BC = W/2 - 1
 //                word W-2 = next bucket index of the chain (NIL = 0xFFFFFFFF)
@@ -25,11 +27,9 @@ constexpr u32 kTomb = 0xFFFFFFFEu;        // tombstone (deleted key)
 constexpr u32 kNil = 0xFFFFFFFFu;         // end of chain / no bucket
 constexpr u64 kEmptyPair = 0xFFFFFFFFFFFFFFFFull;
 
-struct __align__(16) DirEntry {
+struct __align__(8) DirEntry {
   u32 base;    // first base bucket
   u32 nb;      // number of base buckets
-  u32 deg;     // exact number of stored neighbours
-  u32 flags;   // reserved
 };
 
 struct DevCtl {
@@ -47,6 +47,7 @@ struct DevCtl {
 
 struct Tables {
   DirEntry* dir;
+  u32* deg;          // exact degree per local row
   u32* pool;
   u32* stack;
   DevCtl* ctl;
@@ -82,13 +83,14 @@ __device__ __forceinline__ uint4 ld_nc_v4(const u32* p) {
   asm volatile("ld.global.nc.v2.u64 {%0,%1}, [%2];" : "=l"(a), "=l"(b) : "l"(p));
   return make_uint4((u32)a, (u32)(a >> 32), (u32)b, (u32)(b >> 32));
 }
-__device__ __forceinline__ uint4 ld_nc_dir(const DirEntry* p) {
-  return ld_nc_v4(reinterpret_cast<const u32*>(p));
+__device__ __forceinline__ uint2 ld_nc_dir(const DirEntry* p) {
+  uint2 r;
+  asm volatile("ld.global.nc.v2.u32 {%0,%1}, [%2];" : "=r"(r.x), "=r"(r.y) : "l"(p));
+  return r;
 }
-__device__ __forceinline__ uint4 ld_dir(const DirEntry* p) {
-  uint4 r;
-  asm volatile("ld.global.v4.u32 {%0,%1,%2,%3}, [%4];"
-               : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w) : "l"(p));
+__device__ __forceinline__ uint2 ld_dir(const DirEntry* p) {
+  uint2 r;
+  asm volatile("ld.global.v2.u32 {%0,%1}, [%2];" : "=r"(r.x), "=r"(r.y) : "l"(p));
   return r;
 }
 __device__ __forceinline__ u32 ld_relaxed_u32(const u32* p) {

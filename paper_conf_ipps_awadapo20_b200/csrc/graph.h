@@ -30,7 +30,7 @@ struct dg_graph_s {
   uint64_t nv = 0;        // global vertex capacity
   uint64_t rows = 0;      // local rows
 
-  dg::VmmArray dir, pool, stack;
+  dg::VmmArray dir, degv, pool, stack;
   uint32_t cap = 0;       // buckets mapped in the pool
   uint64_t bump_ub = 0;   // host upper bound of the device bump cursor
 
@@ -72,6 +72,7 @@ struct dg_graph_s {
   dg::Tables tables() const {
     dg::Tables t;
     t.dir = reinterpret_cast<dg::DirEntry*>(dir.ptr());
+    t.deg = reinterpret_cast<uint32_t*>(degv.ptr());
     t.pool = reinterpret_cast<uint32_t*>(pool.ptr());
     t.stack = reinterpret_cast<uint32_t*>(stack.ptr());
     t.ctl = ctl;

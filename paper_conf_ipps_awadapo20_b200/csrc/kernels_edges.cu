@@ -104,7 +104,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
   u32 head = 0;
   if (pend) {
     // base/nb never change during an edge phase; only deg is written (atomics)
-    const uint4 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
+    const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
     head = de.x + bucket_of(v, de.y);
   }
   u32 cur = head;
@@ -182,7 +182,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
     // c. one atomic per lane, all in flight together
     if (OP == OP_DELETE && act == ACT_CAS_DEL) {
       if (atomicCAS(ff, v, kTomb) == v) {
-        atomicSub(&t.dir[row].deg, 1u);
+        atomicSub(&t.deg[row], 1u);
         ++my_count;
       }
       pend = false;  // a lost CAS means another op deleted the key (Q5)
@@ -191,7 +191,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
       const unsigned long long old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
                                                (unsigned long long)pack_pair(v, w));
       if (old == ffo) {
-        atomicAdd(&t.dir[row].deg, 1u);
+        atomicAdd(&t.deg[row], 1u);
         ++my_count;
         pend = false;
       } else if ((u32)old == v) {  // a racing op installed the same key: replace

@@ -69,9 +69,8 @@ __global__ void k_init_rows(Tables t, u64 row0, u64 count, const u64* off, const
     DirEntry e;
     e.base = base;
     e.nb = n;
-    e.deg = 0;
-    e.flags = 0;
     t.dir[row0 + r] = e;
+    t.deg[row0 + r] = 0;
     for (u32 k = 0; k < n; ++k) t.pool[(u64)(base + k) * W + Group<G>::OWNER] = (u32)(row0 + r);
   }
 }
@@ -130,30 +129,30 @@ cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s) {
 }
 
 // ------------------------------------------------------------------ degrees ----
-__global__ void k_degrees(const DirEntry* dir, u64 rows, u32* out) {
+__global__ void k_degrees(const u32* deg, u64 rows, u32* out) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < rows; r += stride)
-    out[r] = dir[r].deg;
+    out[r] = deg[r];
 }
 
 cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s) {
   if (t.rows == 0) return cudaSuccess;
   u64 blocks = (t.rows + 255) / 256;
   if (blocks > 65535) blocks = 65535;
-  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.dir, t.rows, out); note_kernel(1);
+  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.deg, t.rows, out); note_kernel(1);
   return cudaGetLastError();
 }
 
 // ------------------------------------------------------------ export (a12) ----
 struct DegAt {
-  const DirEntry* dir;
+  const u32* deg;
   u64 rows;
-  __host__ __device__ u64 operator()(u64 i) const { return i < rows ? (u64)dir[i].deg : 0ull; }
+  __host__ __device__ u64 operator()(u64 i) const { return i < rows ? (u64)deg[i] : 0ull; }
 };
 
 cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
                                   cudaStream_t s) {
-  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0), DegAt{t.dir, t.rows});
+  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0), DegAt{t.deg, t.rows});
   size_t need = 0;
   cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, ro, (int64_t)(t.rows + 1), s);
   if (e != cudaSuccess) return e;
@@ -332,7 +331,7 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
       u32 dec = 0;
       if (h0 && atomicCAS(bp, x.x, kTomb) == x.x) ++dec;
       if (h1 && atomicCAS(bp + 2, x.z, kTomb) == x.z) ++dec;
-      if (dec) atomicSub(&t.dir[owner].deg, dec);
+      if (dec) atomicSub(&t.deg[owner], dec);
     }
   }
 }
@@ -436,7 +435,7 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
         else lm1 &= ~(1u << l);
         const DirEntry dv = t.dir[v];
         if (purge_delete<G>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
-          atomicSub(&t.dir[v].deg, 1u);
+          atomicSub(&t.deg[v], 1u);
       }
       b = g.shfl(q.z, G - 1);
     }
@@ -487,7 +486,7 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
       base_bucket = false;
       b = next;
     }
-    if (j == 0 && g.gl == 0) t.dir[row].deg = 0;
+    if (j == 0 && g.gl == 0) t.deg[row] = 0;
   }
 }
 

@@ -25,7 +25,7 @@ __device__ __forceinline__ bool rank_less(u32 du, u32 u, u32 dv, u32 v) {
 }
 
 __global__ void __launch_bounds__(256) k_tc_orient_count(const u64* ro, const u32* dst,
-                                                         const DirEntry* dir, u64 rows, u32 part,
+                                                         const u32* deg, u64 rows, u32 part,
                                                          u32 nparts, u64* ocnt) {
   const u32 lane = threadIdx.x & 31;
   const u64 wid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
@@ -33,10 +33,10 @@ __global__ void __launch_bounds__(256) k_tc_orient_count(const u64* ro, const u3
   for (u64 u = wid; u < rows; u += nw) {
     u32 c = 0;
     if (u % nparts == part) {
-      const u32 du = dir[u].deg;
+      const u32 du = deg[u];
       for (u64 k = ro[u] + lane; k < ro[u + 1]; k += 32) {
         const u32 v = dst[k];
-        c += rank_less(du, (u32)u, __ldg(&dir[v].deg), v) ? 1u : 0u;
+        c += rank_less(du, (u32)u, __ldg(&deg[v]), v) ? 1u : 0u;
       }
       c = __reduce_add_sync(0xFFFFFFFFu, c);
     }
@@ -46,7 +46,7 @@ __global__ void __launch_bounds__(256) k_tc_orient_count(const u64* ro, const u3
 }
 
 __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32* dst,
-                                                        const DirEntry* dir, u64 rows, u32 part,
+                                                        const u32* deg, u64 rows, u32 part,
                                                         u32 nparts, const u64* oro, u32* oadj,
                                                         u32* oend) {
   const u32 lane = threadIdx.x & 31;
@@ -54,7 +54,7 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
   const u64 nw = ((u64)gridDim.x * blockDim.x) >> 5;
   for (u64 u = wid; u < rows; u += nw) {
     if (u % nparts != part) continue;
-    const u32 du = dir[u].deg;
+    const u32 du = deg[u];
     u64 pos = oro[u];
     const u32 end = (u32)oro[u + 1];
     for (u64 k0 = ro[u]; k0 < ro[u + 1]; k0 += 32) {
@@ -63,7 +63,7 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
       u32 v = 0;
       if (k < ro[u + 1]) {
         v = dst[k];
-        keep = rank_less(du, (u32)u, __ldg(&dir[v].deg), v);
+        keep = rank_less(du, (u32)u, __ldg(&deg[v]), v);
       }
       const u32 m = __ballot_sync(0xFFFFFFFFu, keep);
       if (keep) {
@@ -86,7 +86,7 @@ __global__ void __launch_bounds__(256) k_tc_wedges(Tables t, const u32* __restri
   for (u64 e = (u64)blockIdx.x * blockDim.x + threadIdx.x; e < n_units; e += stride) {
     const u32 v = oadj[e];
     const u32 end = oend[e];
-    const uint4 dv = ld_nc_dir(t.dir + v);
+    const uint2 dv = ld_nc_dir(t.dir + v);
     for (u32 k = (u32)e + 1; k < end; ++k) {
       const u32 w = __ldg(oadj + k);
       u32 b = dv.x + bucket_of(w, dv.y);
@@ -121,7 +121,7 @@ __global__ void __launch_bounds__(256) k_tc_wedges(Tables t, const u32* __restri
 
 cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* dst, u32 part,
                                    u32 nparts, u64* ocnt, int sms, cudaStream_t s) {
-  k_tc_orient_count<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.dir, t.rows, part, nparts, ocnt);
+  k_tc_orient_count<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, ocnt);
   note_kernel(1);
   return cudaGetLastError();
 }
@@ -129,7 +129,7 @@ cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* ds
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
                                   u32 nparts, const u64* oro, u32* oadj, u32* oend, int sms,
                                   cudaStream_t s) {
-  k_tc_orient_fill<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.dir, t.rows, part, nparts, oro, oadj,
+  k_tc_orient_fill<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, oro, oadj,
                                                      oend);
   note_kernel(1);
   return cudaGetLastError();
