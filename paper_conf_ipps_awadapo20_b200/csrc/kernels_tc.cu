@@ -76,46 +76,89 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
   }
 }
 
+// Wedge probes, organised like the edge-query kernel: a group of G lanes owns one
+// oriented entry e = (u, i) at a time (32/G entries per warp, consecutive entries
+// of a row have similar candidate counts); per step every lane takes one candidate
+// w = N+(u)[j] and the group loads the G candidates' buckets of A_v together (one
+// 16-B load per lane per candidate), then decides all G with group ballots.  Warp
+// loops are warp-uniform so every intrinsic uses the full mask.  The rare probes
+// whose key may sit further down a chain are walked by their own lane.
 template <int G>
-__global__ void __launch_bounds__(256) k_tc_wedges(Tables t, const u32* __restrict__ oadj,
-                                                   const u32* __restrict__ oend, u64 n_units,
-                                                   unsigned long long* count) {
+__global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __restrict__ oadj,
+                                                      const u32* __restrict__ oend, u64 n_units,
+                                                      unsigned long long* count) {
   constexpr int W = Group<G>::W;
+  constexpr u32 FULL = 0xFFFFFFFFu;
+  constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
+  constexpr int PER_WARP = 32 / G;
+  const Group<G> g;
+  const bool lastl = g.last();
   u32 hits = 0;
-  const u64 stride = (u64)gridDim.x * blockDim.x;
-  for (u64 e = (u64)blockIdx.x * blockDim.x + threadIdx.x; e < n_units; e += stride) {
-    const u32 v = oadj[e];
-    const u32 end = oend[e];
-    const uint2 dv = ld_nc_dir(t.dir + v);
-    for (u32 k = (u32)e + 1; k < end; ++k) {
-      const u32 w = __ldg(oadj + k);
-      u32 b = dv.x + bucket_of(w, dv.y);
-      while (true) {  // edgeExist(v, w): walk the chain of w's bucket in A_v
-        const uint4* bp = reinterpret_cast<const uint4*>(t.pool + (u64)b * W);
-        bool found = false, ended = false;
-        u32 next = kNil;
+  const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+  const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
+  for (u64 e0 = warp * PER_WARP; e0 < n_units; e0 += nwarps * PER_WARP) {
+    const u64 e = e0 + g.lane / G;                // this group's entry
+    const bool ev = e < n_units;
+    const u32 v = ev ? __ldg(oadj + e) : 0u;
+    const u32 ncand = ev ? __ldg(oend + e) - (u32)e - 1u : 0u;
+    const uint2 dv = ev ? ld_nc_dir(t.dir + v) : make_uint2(0, 1);
+    const u32 maxc = __reduce_max_sync(FULL, ncand);
+    for (u32 k0 = 0; k0 < maxc; k0 += G) {
+      const bool act = k0 + g.gl < ncand;
+      const u32 w = act ? __ldg(oadj + e + 1 + k0 + g.gl) : kEmpty;
+      const u32 head = dv.x + bucket_of(w, dv.y);
+      const u32 amask = __ballot_sync(FULL, act);
+      uint4 q[G];
 #pragma unroll
-        for (int c = 0; c < G; ++c) {
-          const uint4 q = __ldg(bp + c);
-          found |= q.x == w;
-          ended |= q.x == kEmpty;
-          if (c < G - 1) {
-            found |= q.z == w;
-            ended |= q.z == kEmpty;
-          } else {
-            next = q.z;
+      for (int r = 0; r < G; ++r) {
+        const u32 hr = __shfl_sync(FULL, head, g.base + r);
+        if ((amask >> (g.base + r)) & 1u) q[r] = ld_nc_v4(t.pool + (u64)hr * W + 4 * g.gl);
+        else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+      }
+      bool walk = false;
+      u32 nxt = kNil;
+#pragma unroll
+      for (int r = 0; r < G; ++r) {
+        const uint4 x = q[r];
+        const u32 wr = __shfl_sync(FULL, w, g.base + r);
+        const bool pr = (amask >> (g.base + r)) & 1u;
+        const bool m = pr && (x.x == wr || (!lastl && x.z == wr));
+        const u32 hit = (__ballot_sync(FULL, m) >> g.base) & GBITS;
+        const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
+        const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
+        const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
+        if (pr && g.gl == (u32)r) {
+          if (hit) ++hits;
+          else if (!em && next != kNil) { walk = true; nxt = next; }
+        }
+      }
+      // rare: the key may sit further down the chain (edgeExist)
+      if (walk) {
+        u32 b = nxt;
+        while (b != kNil) {
+          const uint4* bp = reinterpret_cast<const uint4*>(t.pool + (u64)b * W);
+          bool found = false, ended = false;
+          u32 nb2 = kNil;
+#pragma unroll
+          for (int c = 0; c < G; ++c) {
+            const uint4 y = __ldg(bp + c);
+            found |= y.x == w;
+            ended |= y.x == kEmpty;
+            if (c < G - 1) {
+              found |= y.z == w;
+              ended |= y.z == kEmpty;
+            } else {
+              nb2 = y.z;
+            }
           }
+          if (found) { ++hits; break; }
+          if (ended) break;
+          b = nb2;
         }
-        if (found) {
-          ++hits;
-          break;
-        }
-        if (ended || next == kNil) break;
-        b = next;
       }
     }
   }
-  const u32 tot = __reduce_add_sync(0xFFFFFFFFu, hits);
+  const u32 tot = __reduce_add_sync(FULL, hits);
   if ((threadIdx.x & 31) == 0 && tot) atomicAdd(count, (unsigned long long)tot);
 }
 
@@ -138,8 +181,8 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
 cudaError_t launch_tc_wedges(int G, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s) {
   if (n_units == 0) return cudaSuccess;
-  u64 blocks = (n_units + 255) / 256;
-  if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  u64 blocks = (n_units * G + 255) / 256;
+  if (blocks > (u64)sms * 4) blocks = (u64)sms * 4;
   switch (G) {
     case 2: k_tc_wedges<2><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); break;
     case 4: k_tc_wedges<4><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); break;

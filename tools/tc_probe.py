@@ -1,0 +1,21 @@
+"""TC timing at R-MAT scale s (symmetrised): python tools/tc_probe.py [scale] [bucket_bytes]"""
+import os, sys, time
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import numpy as np, torch
+import workloads as wl
+from paper_conf_ipps_awadapo20_b200 import Graph
+scale = int(sys.argv[1]) if len(sys.argv) > 1 else 22
+bb = int(sys.argv[2]) if len(sys.argv) > 2 else 128
+nv = 1 << scale
+s, d = wl.rmat_edges(5, 0, 16 * nv, scale, wl.GRAPH500)
+dev = torch.device("cuda", 0)
+deg = torch.bincount(torch.from_numpy(np.concatenate([s, d]).astype(np.int64)).to(dev), minlength=nv).to(torch.int32)
+g = Graph(nv, deg, directed=False, bucket_bytes=bb)
+g.insert_edges(torch.from_numpy(s).to(dev), torch.from_numpy(d).to(dev))
+g.profile_enable(True)
+for r in range(2):
+    torch.cuda.synchronize(); t0 = time.perf_counter()
+    c = g.triangle_count()
+    t1 = time.perf_counter()
+    p = g.profile_read()
+    print(f"scale {scale} S={bb}: triangles {c}  total {1e3*(t1-t0):.1f} ms  wedge kernel {p['kernel_ms']['tc']:.1f} ms (cumulative)")
