@@ -269,6 +269,11 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_fixup_alloc(t, s));
+  if (g->hot_steps && !g->in_rehash) {  // chain-length metric, read before the next batch
+    DG_CK(cudaMemcpyAsync(g->h_hot, &g->ctl->hot_count, 8, cudaMemcpyDeviceToHost, s));
+    DG_CK(cudaEventRecord(g->hot_event, s));
+    g->hot_pending = true;
+  }
   if (!retry_mode) {
     note_launch(g, need, s);
     return DG_OK;
@@ -328,6 +333,74 @@ dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t
   prof_mark(g, PROF_QUERY, s);
   DG_CK(dg::launch_query(g->G, g->tables(), a, g->sms, s));
   prof_mark(g, PROF_QUERY, s);
+  return DG_OK;
+}
+
+// Re-size the rows flagged by the insert kernel for long chains:
+// export their pairs, release all their buckets, give each a fresh base range sized
+// for twice its degree, and insert the pairs again.  Runs before an insert batch
+// (phase-concurrent: no other batch in flight on the handle).
+dg_status rehash_hot(dg_graph g, cudaStream_t s) {
+  const u32 n = std::min<u32>(*g->h_hot, g->hot_cap);
+  if (n == 0) return DG_OK;
+  g->in_rehash = true;
+  struct Guard {
+    dg_graph g;
+    ~Guard() { g->in_rehash = false; }
+  } guard{g};
+  const u64 m = (u64)n + 1;
+  DG_CK(ensure_buf(g->rh[0], 7 * m * 8));
+  u64* nbnew = reinterpret_cast<u64*>(g->rh[0].p);
+  u64* nbold = nbnew + m;
+  u64* degs = nbold + m;
+  u64* nboff = degs + m;
+  u64* obo = nboff + m;
+  u64* doff = obo + m;
+  u64* cursor = doff + m;
+  dg::Tables t = g->tables();
+  DG_CK(dg::launch_hot_sizes(t, n, g->lf_milli, g->BC, nbnew, nbold, degs, s));
+  DG_CK(dg::scan_exclusive_u64(nbnew, nboff, m, &g->scan_temp, &g->scan_bytes, s));
+  DG_CK(dg::scan_exclusive_u64(nbold, obo, m, &g->scan_temp, &g->scan_bytes, s));
+  DG_CK(dg::scan_exclusive_u64(degs, doff, m, &g->scan_temp, &g->scan_bytes, s));
+  u64 tot[3] = {0, 0, 0};
+  DG_CK(cudaMemcpyAsync(&tot[0], nboff + n, 8, cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaMemcpyAsync(&tot[1], doff + n, 8, cudaMemcpyDeviceToHost, s));
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  g->snap_pending = false;
+  DG_TRY(read_ctl(g, s));
+  const u64 total_new = tot[0], total_deg = tot[1];
+  if (std::getenv("DG_DEBUG"))
+    std::fprintf(stderr, "dg: re-sizing %u rows (%llu pairs, %llu new base buckets)\n", n,
+                 (unsigned long long)total_deg, (unsigned long long)total_new);
+  const u64 bump0 = g->hctl->bump;
+  if (bump0 + total_new + 1 >= 0xFFFFFFFEull) {  // no room: forget the flags
+    DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
+    DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
+    return DG_OK;
+  }
+  DG_TRY(grow_pool(g, bump0 + total_new + g->cap / 8 + 65536, s));
+  t = g->tables();
+  DG_CK(ensure_buf(g->rh[1], total_deg * 4 + 4));
+  DG_CK(ensure_buf(g->rh[2], total_deg * 4 + 4));
+  DG_CK(ensure_buf(g->rh[3], total_deg * 4 + 4));
+  u32* osrc = reinterpret_cast<u32*>(g->rh[1].p);
+  u32* odst = reinterpret_cast<u32*>(g->rh[2].p);
+  u32* ow = reinterpret_cast<u32*>(g->rh[3].p);
+  DG_CK(cudaMemcpyAsync(cursor, doff, n * 8, cudaMemcpyDeviceToDevice, s));
+  DG_CK(dg::launch_hot_export(g->G, t, n, obo, reinterpret_cast<unsigned long long*>(cursor), osrc,
+                              odst, ow, g->rank, g->sms, s));
+  DG_CK(dg::launch_hot_release(g->G, t, n, obo, g->sms, s));
+  DG_CK(dg::launch_hot_install(t, n, nbnew, nboff, (u32)bump0, g->W, s));
+  const u32 newbump = (u32)(bump0 + total_new);
+  DG_CK(cudaMemcpyAsync(&g->ctl->bump, &newbump, 4, cudaMemcpyHostToDevice, s));
+  DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
+  DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));  // hot_count, hot_pairs
+  DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
+  DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, 4, s));
+  g->bump_ub = std::max<u64>(g->bump_ub, newbump);
+  // the pairs go back through the ordinary insert kernel (all keys distinct)
+  DG_TRY(local_insert(g, osrc, odst, ow, total_deg, false, ++g->epoch, s));
+  DG_CK(cudaStreamSynchronize(s));
   return DG_OK;
 }
 
@@ -402,6 +475,12 @@ static void destroy_graph(dg_graph g) {
     if (b.p) cudaFree(b.p);
   for (auto& b : g->tc)
     if (b.p) cudaFree(b.p);
+  for (auto& b : g->rh)
+    if (b.p) cudaFree(b.p);
+  if (g->hot_flags) cudaFree(g->hot_flags);
+  if (g->hot_list) cudaFree(g->hot_list);
+  if (g->h_hot) cudaFreeHost(g->h_hot);
+  if (g->hot_event) cudaEventDestroy(g->hot_event);
   for (auto& cs : g->cstream)
     if (cs) cudaStreamDestroy(cs);
   for (cudaEvent_t e : g->pipe_ev) cudaEventDestroy(e);
@@ -443,6 +522,18 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
   if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
   DG_CK(e);
   g->rows = row0 + count;
+  {  // re-sizing flags: one bit per row (transient: a growth simply clears them)
+    const u64 words = (g->rows + 31) / 32 + 1;
+    if (words > g->hot_words) {
+      if (g->hot_flags) cudaFree(g->hot_flags);
+      g->hot_flags = nullptr;
+      g->hot_words = 0;
+      DG_CK(cudaMalloc(&g->hot_flags, words * 4));
+      g->hot_words = words;
+      DG_CK(cudaMemsetAsync(g->hot_flags, 0, words * 4, s));
+      DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
+    }
+  }
   DG_CK(dg::launch_init_rows(g->G, g->tables(), row0, count, off, nb, (u32)base0, s));
   const u32 newbump = (u32)(base0 + total);
   DG_CK(cudaMemcpyAsync(&g->ctl->bump, &newbump, 4, cudaMemcpyHostToDevice, s));
@@ -511,6 +602,12 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (cudaMalloc(&g->ret_list, dg::max_groups(g->G, g->sms) * 4 + 64) != cudaSuccess)
     return fail(DG_ERR_CUDA);
   if (cudaMalloc(&g->small_dev, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (const char* hs = std::getenv("DG_HOT_STEPS")) g->hot_steps = (u32)std::atoi(hs);
+  if (cudaMalloc(&g->hot_list, (size_t)g->hot_cap * 4) != cudaSuccess) return fail(DG_ERR_CUDA);
+  if (cudaMallocHost(&g->h_hot, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
+  *g->h_hot = 0;
+  if (cudaEventCreateWithFlags(&g->hot_event, cudaEventDisableTiming) != cudaSuccess)
+    return fail(DG_ERR_CUDA);
   if (cudaMalloc(&g->stats_dev, sizeof(dg::StatsOut)) != cudaSuccess) return fail(DG_ERR_CUDA);
 
   if (g->nranks > 1) {
@@ -574,6 +671,17 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   if (n && (!src || !dst)) return DG_ERR_INVALID_ARGUMENT;
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   if (n_added) *n_added = 0;
+  // re-size tables whose chains grew too long in earlier batches
+  if (g->hot_steps && g->hot_pending) {
+    const cudaError_t q = cudaEventQuery(g->hot_event);
+    if (q == cudaSuccess) {
+      g->hot_pending = false;
+      // worth a re-sizing pass: enough pairs to move, or the flag list filling up
+      if (g->h_hot[1] >= 2048 || g->h_hot[0] >= g->hot_cap / 2) DG_TRY(dg::rehash_hot(g, s));
+    } else if (q != cudaErrorNotReady) {
+      DG_CK(q);
+    }
+  }
   const u32 epoch = ++g->epoch;
   bool host = false;
   const void *ds = nullptr, *dd = nullptr, *dw = nullptr;

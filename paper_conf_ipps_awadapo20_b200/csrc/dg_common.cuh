@@ -42,7 +42,8 @@ struct DevCtl {
   u32 queue;         // work-queue cursor (vertex purge, Alg2:L3-6)
   u32 dedup_count;   // distinct vertices in the current vertex-deletion batch
   u64 count;         // n_added / n_removed / TC accumulator of the current batch
-  u64 aux;
+  u32 hot_count;     // rows flagged for re-sizing (long chains), see k_edges / rehash
+  u32 hot_pairs;     // sum of their degrees when flagged (saturating): work to re-size
 };
 
 struct Tables {
@@ -55,6 +56,10 @@ struct Tables {
   u64 rows;          // local rows
   u32 cap;           // buckets mapped in the pool
   u32 nranks;        // row = global id / nranks at nranks > 1
+  u32* hot_flags;    // bit per local row: flagged for re-sizing (nullable = off)
+  u32* hot_list;     // flagged rows
+  u32 hot_cap;       // capacity of hot_list
+  u32 hot_steps;     // chain buckets an insert may walk before flagging its row
 };
 
 // ------------------------------------------------------------------ hashing ----

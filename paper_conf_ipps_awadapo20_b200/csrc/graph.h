@@ -59,6 +59,17 @@ struct dg_graph_s {
     size_t bytes = 0;
   } stage[8];
   Buf tc[6];  // triangle counting scratch (CSR, orientation)
+  Buf rh[4];  // re-sizing scratch
+  // per-vertex re-sizing of long chains
+  uint32_t* hot_flags = nullptr;
+  uint64_t hot_words = 0;
+  uint32_t* hot_list = nullptr;
+  uint32_t hot_cap = 65536;
+  uint32_t hot_steps = 4;      // 0 = off
+  uint32_t* h_hot = nullptr;   // pinned copy of ctl->hot_count
+  cudaEvent_t hot_event = nullptr;
+  bool hot_pending = false;
+  bool in_rehash = false;
   cudaStream_t cstream[2] = {nullptr, nullptr};  // host-buffer pipeline: upload, download
   std::vector<cudaEvent_t> pipe_ev;
 
@@ -80,6 +91,10 @@ struct dg_graph_s {
     t.rows = rows;
     t.cap = cap;
     t.nranks = nranks;
+    t.hot_flags = hot_steps ? hot_flags : nullptr;
+    t.hot_list = hot_list;
+    t.hot_cap = hot_cap;
+    t.hot_steps = hot_steps;
     return t;
   }
 };
@@ -96,6 +111,7 @@ void prof_mark(dg_graph g, int k, cudaStream_t s);
 
 // internal entry points shared by api.cu and router.cu
 dg_status grow_pool(dg_graph g, uint64_t min_buckets, cudaStream_t s);
+dg_status rehash_hot(dg_graph g, cudaStream_t s);
 dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
                        uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s);
 dg_status local_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,

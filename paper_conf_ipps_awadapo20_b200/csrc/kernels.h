@@ -88,4 +88,15 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
 cudaError_t launch_tc_wedges(int G, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s);
 
+// per-vertex re-sizing of long-chained tables (kernels_rehash.cu)
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
+                             u64* degs, cudaStream_t s);
+cudaError_t launch_hot_export(int G, const Tables& t, u32 n, const u64* obo,
+                              unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
+                              int sms, cudaStream_t s);
+cudaError_t launch_hot_release(int G, const Tables& t, u32 n, const u64* obo, int sms,
+                               cudaStream_t s);
+cudaError_t launch_hot_install(const Tables& t, u32 n, const u64* nbnew, const u64* nboff,
+                               u32 base0, u32 words, cudaStream_t s);
+
 }  // namespace dg

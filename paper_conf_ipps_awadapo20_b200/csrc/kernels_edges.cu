@@ -102,14 +102,17 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
   }
   const u32 row = (t.nranks == 1) ? u : u / t.nranks;
   u32 head = 0;
+  u32 nbase = 0;
   if (pend) {
     // base/nb never change during an edge phase; only deg is written (atomics)
     const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
     head = de.x + bucket_of(v, de.y);
+    nbase = de.y;
   }
   u32 cur = head;
   bool found = false;
   u32 val = 0;
+  u32 steps = 0;                   // insert: chain buckets walked
   u32* ff = nullptr;               // insert: first free slot of the chain (pair address)
   unsigned long long ffo = 0;      //         and its contents when scanned
 
@@ -173,8 +176,25 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a, con
             pend = false;
           } else {
             if (!ff && fm) { ff = reinterpret_cast<u32*>(sa); ffo = so; }
-            if (end) act = ff ? ACT_CAS_INS : ACT_EXTEND;
-            else cur = next;
+            if (end) {
+              act = ff ? ACT_CAS_INS : ACT_EXTEND;
+            } else {
+              cur = next;
+              // a long chain in an over-full table (more keys than base slots):
+              // flag the row for re-sizing before the next batch (per-vertex chain
+              // metric + rehash)
+              if (++steps == t.hot_steps && t.hot_flags) {
+                const u32 dr = ld_relaxed_u32(t.deg + row);
+                if (dr > nbase * Group<G>::BC) {
+                  const u32 bit = 1u << (row & 31);
+                  if (!(atomicOr(&t.hot_flags[row >> 5], bit) & bit)) {
+                    const u32 k = atomicAdd(&t.ctl->hot_count, 1u);
+                    if (k < t.hot_cap) t.hot_list[k] = row;
+                    atomicAdd(&t.ctl->hot_pairs, dr);
+                  }
+                }
+              }
+            }
           }
         }
       }

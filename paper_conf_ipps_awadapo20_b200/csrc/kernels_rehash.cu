@@ -1,0 +1,177 @@
+// kernels_rehash.cu — per-vertex table re-sizing (P:L309-313:
+// "maintain low-cost metrics per vertex to determine the chain-length and
+// periodically perform rehashing if it exceeds a given threshold").
+//
+// An insert that walks more than `hot_steps` chained buckets flags its row
+// (k_edges).  Before the next insert batch the host re-sizes the flagged rows:
+//   k_hot_sizes    : new #base buckets = max(nb+1, ceil(2*deg / (lf*Bc))), old nb, deg
+//   k_hot_export   : live pairs of the flagged tables -> (src, dst, w) lists
+//   k_hot_release  : every bucket of the old tables (base and chained) reset to
+//                    EMPTY and pushed on the free stack
+//   k_hot_install  : new directory entries over a fresh consecutive base range
+// and the exported pairs are inserted again with the ordinary insert kernel.  The
+// logical graph is unchanged (same keys, same values, exact degrees); only chain
+// lengths (and any tombstones of those rows) go away.
+#include "dg_common.cuh"
+#include "kernels.h"
+
+namespace dg {
+
+__global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
+                            u64* degs) {
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k <= n; k += stride) {
+    if (k == n) {
+      nbnew[k] = nbold[k] = degs[k] = 0;
+      continue;
+    }
+    const u32 row = t.hot_list[k];
+    const DirEntry de = t.dir[row];
+    const u64 d = t.deg[row];
+    const u64 den = (u64)lf_milli * bc;
+    u64 want = (2 * d * 1000 + den - 1) / den;  // room to double before chaining again
+    if (want < (u64)de.nb + 1) want = (u64)de.nb + 1;
+    nbnew[k] = want;
+    nbold[k] = de.nb;
+    degs[k] = d;
+  }
+}
+
+// largest k < cnt with off[k] <= x
+__device__ __forceinline__ u32 seg_of(const u64* off, u32 cnt, u64 x) {
+  u32 lo = 0, hi = cnt;
+  while (hi - lo > 1) {
+    const u32 mid = (lo + hi) >> 1;
+    if (off[mid] <= x) lo = mid;
+    else hi = mid;
+  }
+  return lo;
+}
+
+// one group per (flagged row, old base bucket): walk the chain, append live pairs
+template <int G>
+__global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* obo,
+                                                    unsigned long long* cursor, u32* osrc,
+                                                    u32* odst, u32* ow, u32 rank) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  const u64 total = obo[n];
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  const u32 below = (1u << g.gl) - 1u;
+  for (u64 x = gid; x < total; x += ng) {
+    const u32 k = seg_of(obo, n, x);
+    const u32 row = t.hot_list[k];
+    const u32 gid_u = row * t.nranks + rank;  // global source id
+    u32 b = t.dir[row].base + (u32)(x - obo[k]);
+    while (b != kNil) {
+      const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
+      const bool l0 = q.x < kTomb, l1 = !g.last() && q.z < kTomb;
+      const u32 m0 = g.ballot(l0), m1 = g.ballot(l1);
+      const u32 cnt = __popc(m0) + __popc(m1);
+      unsigned long long pos = 0;
+      if (g.gl == 0 && cnt) pos = atomicAdd(cursor + k, (unsigned long long)cnt);
+      pos = g.shfl(pos, 0);
+      const u64 before = __popc(m0 & below) + __popc(m1 & below);
+      if (l0) {
+        osrc[pos + before] = gid_u;
+        odst[pos + before] = q.x;
+        ow[pos + before] = q.y;
+      }
+      if (l1) {
+        const u64 at = pos + before + (l0 ? 1 : 0);
+        osrc[at] = gid_u;
+        odst[at] = q.z;
+        ow[at] = q.w;
+      }
+      b = g.shfl(q.z, G - 1);
+    }
+  }
+}
+
+// every bucket of the old tables -> EMPTY, onto the free stack (base ones too: the
+// row moves to a new base range)
+template <int G>
+__global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64* obo) {
+  constexpr int W = Group<G>::W;
+  const Group<G> g;
+  const u64 total = obo[n];
+  const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  for (u64 x = gid; x < total; x += ng) {
+    const u32 k = seg_of(obo, n, x);
+    const u32 row = t.hot_list[k];
+    u32 b = t.dir[row].base + (u32)(x - obo[k]);
+    while (b != kNil) {
+      u32* bp = t.pool + (u64)b * W + 4 * g.gl;
+      const uint4 q = ld_relaxed_v4(bp);
+      const u32 next = g.shfl(q.z, G - 1);
+      st_v4(bp, empty4);
+      if (g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
+      b = next;
+    }
+  }
+}
+
+__global__ void k_hot_install(Tables t, u32 n, const u64* nbnew, const u64* nboff, u32 base0,
+                              u32 words) {
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k < n; k += stride) {
+    const u32 row = t.hot_list[k];
+    const u32 base = base0 + (u32)nboff[k];
+    const u32 nb = (u32)nbnew[k];
+    DirEntry e;
+    e.base = base;
+    e.nb = nb;
+    t.dir[row] = e;
+    t.deg[row] = 0;
+    for (u32 j = 0; j < nb; ++j) t.pool[(u64)(base + j) * words + words - 1] = row;
+    atomicAnd(&t.hot_flags[row >> 5], ~(1u << (row & 31)));
+  }
+}
+
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
+                             u64* degs, cudaStream_t s) {
+  const unsigned blocks = (n + 256) / 256;
+  k_hot_sizes<<<blocks, 256, 0, s>>>(t, n, lf_milli, bc, nbnew, nbold, degs);
+  note_kernel(1);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_hot_export(int G, const Tables& t, u32 n, const u64* obo,
+                              unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
+                              int sms, cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (G) {
+    case 2: k_hot_export<2><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
+    case 4: k_hot_export<4><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
+    case 8: k_hot_export<8><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
+    default: return cudaErrorInvalidValue;
+  }
+  note_kernel(1);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_hot_release(int G, const Tables& t, u32 n, const u64* obo, int sms,
+                               cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (G) {
+    case 2: k_hot_release<2><<<blocks, 256, 0, s>>>(t, n, obo); break;
+    case 4: k_hot_release<4><<<blocks, 256, 0, s>>>(t, n, obo); break;
+    case 8: k_hot_release<8><<<blocks, 256, 0, s>>>(t, n, obo); break;
+    default: return cudaErrorInvalidValue;
+  }
+  note_kernel(1);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_hot_install(const Tables& t, u32 n, const u64* nbnew, const u64* nboff,
+                               u32 base0, u32 words, cudaStream_t s) {
+  const unsigned blocks = (n + 255) / 256;
+  k_hot_install<<<blocks, 256, 0, s>>>(t, n, nbnew, nboff, base0, words);
+  note_kernel(1);
+  return cudaGetLastError();
+}
+
+}  // namespace dg

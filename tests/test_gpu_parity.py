@@ -131,7 +131,12 @@ def test_churn_tombstone_policy(reuse):
     from paper_conf_ipps_awadapo20_b200 import Graph
     nv = 50_000
     s0, d0, w0 = wl.uniform_edges(13, 0, 400_000, nv)
-    g = Graph(nv, wl.out_degrees(s0, nv), reuse_tombstones=reuse)
+    if not reuse:
+        os.environ["DG_HOT_STEPS"] = "0"  # pure append-only policy: no re-sizing compaction
+    try:
+        g = Graph(nv, wl.out_degrees(s0, nv), reuse_tombstones=reuse)
+    finally:
+        os.environ.pop("DG_HOT_STEPS", None)
     o = Oracle(nv)
     g.insert_edges(cuda(s0), cuda(d0), cuda(w0))
     o.insert_edges(s0, d0, w0)
@@ -201,7 +206,11 @@ def test_freed_buckets_are_reused():
     from paper_conf_ipps_awadapo20_b200 import Graph
     s = np.zeros(3000, np.uint32)
     d = (np.arange(3000) + 4).astype(np.uint32)
-    g2 = Graph(3100, bucket_bytes=32)  # 3 pairs per bucket, one base bucket per vertex
+    os.environ["DG_HOT_STEPS"] = "0"  # keep the long chain (no re-sizing) for this check
+    try:
+        g2 = Graph(3100, bucket_bytes=32)  # 3 pairs per bucket, one base bucket per vertex
+    finally:
+        del os.environ["DG_HOT_STEPS"]
     g2.insert_edges(cuda(s), cuda(d))
     st1 = g2.stats()
     assert st1["overflow_buckets"] == 999 and st1["live_pairs"] == 3000
@@ -466,3 +475,31 @@ def test_host_query_pipeline_large():
     idx = np.arange(0, n, 97)
     st, rf, rw = o.query_edges(qs[idx], qd[idx])
     assert np.array_equal(rf, fh[idx]) and np.array_equal(rw, wh[idx])
+
+
+@pytest.mark.parametrize("bb", [32, 128])
+def test_rehash_long_chains_without_hints(bb):
+    """Per-vertex re-sizing: an R-MAT graph built
+    incrementally with one bucket per vertex grows hub chains; flagged tables are
+    re-sized before the next batch.  Results stay identical to the oracle and the
+    chains end short."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    scale = 16
+    nv = 1 << scale
+    g = Graph(nv, bucket_bytes=bb)
+    o = Oracle(nv)
+    for b in range(8):
+        s, d = wl.rmat_edges(7, b, 150_000, scale, wl.GRAPH500)
+        w = wl.weights(7, b, s.size)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+        check_against_oracle(g, o, f"batch {b}")
+        if b == 0:
+            first_chain = g.stats()["max_chain"]
+    ds, dd = wl.rmat_edges(7, 0, 50_000, scale, wl.GRAPH500)
+    assert g.delete_edges(cuda(ds), cuda(dd), count=True) == o.delete_edges(ds, dd)[1]
+    e = torch.empty(0, dtype=torch.uint32, device="cuda")
+    g.insert_edges(e, e)  # the re-sizing check runs at the start of an insert batch
+    check_against_oracle(g, o, "after re-sizing")
+    st = g.stats()
+    assert first_chain > 20 and st["max_chain"] <= 8, (first_chain, st["max_chain"])
+    assert st["live_pairs"] == o.num_edges() and st["tombstones"] < 50_000
