@@ -85,6 +85,7 @@ def run_mixed(args, cfg):
         pg.barrier()
     a0, a1 = ev(), ev()
     g = Graph(nv, hints, bucket_bytes=S, load_factor=args.load_factor, rank=rank, nranks=world,
+              set_variant=args.variant == "set",
               nccl_unique_id=uid)
     BS, BD, BW = cu(bs), cu(bd), cu(bw)
     torch.cuda.synchronize()
@@ -226,7 +227,10 @@ def run_tc(args, cfg):
     gen_s = time.perf_counter() - t0
     cu = lambda a: torch.from_numpy(np.ascontiguousarray(a)).to(dev)  # noqa: E731
     ev = lambda: torch.cuda.Event(enable_timing=True)  # noqa: E731
-    g = Graph(nv, hints, bucket_bytes=S, load_factor=args.load_factor, directed=False)
+    # the paper counts triangles on the set variant (keys only)
+    variant = args.variant or "set"
+    g = Graph(nv, hints, bucket_bytes=S, load_factor=args.load_factor, directed=False,
+              set_variant=variant == "set")
     a0, a1 = ev(), ev()
     BS, BD = cu(bs), cu(bd)
     torch.cuda.synchronize()
@@ -284,7 +288,7 @@ def run_tc(args, cfg):
     value = edge_ops / (total_ms * 1e3)
     peak, peak_src = load_peaks()
     bytes_per_probe = S + 4  # one bucket of A_v + the streamed candidate id
-    roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16}>", "unit": "GB/s",
+    roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16},{variant}>", "unit": "GB/s",
                 "achieved": wedge_ops / world * bytes_per_probe / (wk / nl * 1e-3) / 1e9,
                 "peak": peak, "peak_source": peak_src, "traffic": None,
                 "algorithmic_bytes_per_launch": wedge_ops / world * bytes_per_probe,
@@ -301,7 +305,7 @@ def run_tc(args, cfg):
                                f"symmetrised; step = insert {IB:,} new undirected edges + TC "
                                f"(edge ops counted: 2 directed inserts per edge + 1 edgeExist "
                                f"per wedge)",
-                   "bucket_bytes": S, "load_factor": args.load_factor,
+                   "bucket_bytes": S, "load_factor": args.load_factor, "variant": variant,
                    "l2": "flushed (256 MiB write) before every step",
                    "parallelism": f"replicas x{world}, wedges split by u mod {world}"
                    if world > 1 else "single GPU"},

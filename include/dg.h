@@ -103,6 +103,12 @@ typedef struct dg_config {
  * router over a 1-rank NCCL communicator (exercises partition / exchange / answer
  * return on one GPU). */
 #define DG_FLAG_FORCE_ROUTER 2u
+/* Set variant: the per-vertex tables hold keys only, twice as many
+ * per bucket (30 per 128 B, 14 per 64 B, 6 per 32 B), for unweighted graphs and
+ * triangle counting.  Weights are not stored: dg_insert_edges ignores
+ * `weight`, dg_query_edges reports weight 0 for every hit, dg_export_adjacency
+ * writes weight 0.  Membership results are those of the map variant. */
+#define DG_FLAG_SET 4u
 
 /* Memory / structure statistics (Fig. 2b/c quantities). */
 typedef struct dg_stats {

@@ -22,6 +22,7 @@ DG_ERR_BAD_STATE = 6
 DG_ERR_UNSUPPORTED = 7
 DG_FLAG_NO_TOMBSTONE_REUSE = 1
 DG_FLAG_FORCE_ROUTER = 2
+DG_FLAG_SET = 4
 
 VP = ctypes.c_void_p
 U64 = ctypes.c_uint64

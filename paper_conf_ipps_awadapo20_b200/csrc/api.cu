@@ -266,7 +266,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   a.epoch = epoch;
   a.nv = g->nv;
   prof_mark(g, PROF_INSERT, s);
-  DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
+  DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_fixup_alloc(t, s));
   if (g->hot_steps && !g->in_rehash) {  // chain-length metric, read before the next batch
@@ -294,7 +294,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
     a.idx = g->retry[cur];
     a.n_ops = failed;
     a.retry_out = g->retry[cur ^ 1];
-    DG_CK(dg::launch_insert(g->G, t, a, g->sms, s));
+    DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
     DG_CK(dg::launch_fixup_alloc(t, s));
     cur ^= 1;
   }
@@ -313,7 +313,7 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
   a.epoch = epoch;
   a.nv = g->nv;
   prof_mark(g, PROF_DELETE, s);
-  DG_CK(dg::launch_delete(g->G, g->tables(), a, g->sms, s));
+  DG_CK(dg::launch_delete(g->lay, g->tables(), a, g->sms, s));
   prof_mark(g, PROF_DELETE, s);
   return DG_OK;
 }
@@ -331,7 +331,7 @@ dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t
   a.found = found;
   a.wout = wout;
   prof_mark(g, PROF_QUERY, s);
-  DG_CK(dg::launch_query(g->G, g->tables(), a, g->sms, s));
+  DG_CK(dg::launch_query(g->lay, g->tables(), a, g->sms, s));
   prof_mark(g, PROF_QUERY, s);
   return DG_OK;
 }
@@ -387,7 +387,7 @@ dg_status rehash_hot(dg_graph g, cudaStream_t s) {
   u32* odst = reinterpret_cast<u32*>(g->rh[2].p);
   u32* ow = reinterpret_cast<u32*>(g->rh[3].p);
   DG_CK(cudaMemcpyAsync(cursor, doff, n * 8, cudaMemcpyDeviceToDevice, s));
-  DG_CK(dg::launch_hot_export(g->G, t, n, obo, reinterpret_cast<unsigned long long*>(cursor), osrc,
+  DG_CK(dg::launch_hot_export(g->lay, t, n, obo, reinterpret_cast<unsigned long long*>(cursor), osrc,
                               odst, ow, g->rank, g->sms, s));
   DG_CK(dg::launch_hot_release(g->G, t, n, obo, g->sms, s));
   DG_CK(dg::launch_hot_install(t, n, nbnew, nboff, (u32)bump0, g->W, s));
@@ -555,7 +555,8 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
-  if (cfg->flags & ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER)) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->flags & ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER | DG_FLAG_SET))
+    return DG_ERR_INVALID_ARGUMENT;
 
   dg_graph g = new (std::nothrow) dg_graph_s();
   if (!g) return DG_ERR_OUT_OF_MEMORY;
@@ -577,7 +578,9 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   g->bucket_bytes = cfg->bucket_bytes;
   g->G = (int)(cfg->bucket_bytes / 16);
   g->W = cfg->bucket_bytes / 4;
-  g->BC = cfg->bucket_bytes / 8 - 1;
+  g->set = (cfg->flags & DG_FLAG_SET) != 0;
+  g->BC = g->set ? cfg->bucket_bytes / 4 - 2 : cfg->bucket_bytes / 8 - 1;  // Q15
+  g->lay = DG_LAY(g->G, g->set ? 1 : 0);
   g->lf_milli = std::max<u32>(1, (u32)std::lround((double)cfg->load_factor * 1000.0));
   g->nranks = (u32)cfg->nranks;
   g->rank = (u32)cfg->rank;
@@ -909,10 +912,10 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
   dg::prof_mark(g, dg::PROF_VDEL, s);
   if (!g->directed && g->nranks == 1 && !force_sweep) {
     // undirected: Alg. 2 — delete u from the tables of its neighbours
-    DG_CK(dg::launch_vdel_neighbors(g->G, t, g->dedup, boff, epoch, g->sms, s));
+    DG_CK(dg::launch_vdel_neighbors(g->lay, t, g->dedup, boff, epoch, g->sms, s));
   } else {
     // directed: follow-up sweep over all tables
-    DG_CK(dg::launch_vdel_sweep(g->G, t, g->bitmap, epoch, g->sms, s));
+    DG_CK(dg::launch_vdel_sweep(g->lay, t, g->bitmap, epoch, g->sms, s));
   }
   DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, boff, epoch, g->sms, s));
   dg::prof_mark(g, dg::PROF_VDEL, s);
@@ -948,7 +951,7 @@ dg_status dg_export_adjacency(dg_graph g, uint64_t* row_offsets, uint32_t* dst, 
     void *dd = nullptr, *dw = nullptr;
     DG_TRY(stage_out(g, 4, dst, m * 4, &dd, &host));
     DG_TRY(stage_out(g, 7, weight, weight ? m * 4 : 0, &dw, &host));
-    DG_CK(dg::launch_export_fill(g->G, t, (const u64*)dro, (u32*)dd, (u32*)dw, g->sms, s));
+    DG_CK(dg::launch_export_fill(g->lay, t, (const u64*)dro, (u32*)dd, (u32*)dw, g->sms, s));
     DG_TRY(finish_out(g, dst, dd, m * 4, s));
     DG_TRY(finish_out(g, weight, dw, weight ? m * 4 : 0, s));
   }
@@ -978,7 +981,7 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   dg::StatsOut h{};
   auto* d = reinterpret_cast<dg::StatsOut*>(g->stats_dev);
-  DG_CK(dg::launch_stats(g->G, g->tables(), d, g->sms, s));
+  DG_CK(dg::launch_stats(g->lay, g->tables(), d, g->sms, s));
   DG_CK(cudaMemcpyAsync(&h, d, sizeof(h), cudaMemcpyDeviceToHost, s));
   if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   g->snap_pending = false;
@@ -1031,7 +1034,7 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   if (m >= 0xFFFFFFFFull) return DG_ERR_UNSUPPORTED;
   DG_CK(ensure_buf(g->tc[1], m * 4 + 4));
   u32* dst = reinterpret_cast<u32*>(g->tc[1].p);
-  DG_CK(dg::launch_export_fill(g->G, t, ro, dst, nullptr, g->sms, s));
+  DG_CK(dg::launch_export_fill(g->lay, t, ro, dst, nullptr, g->sms, s));
   // (2) orientation by rank = (degree, id)
   DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8));
   DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8));
@@ -1050,7 +1053,7 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   // (3) one edgeExist per wedge
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);
-  DG_CK(dg::launch_tc_wedges(g->G, t, oadj, oend, mo,
+  DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, mo,
                              reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
   dg::prof_mark(g, dg::PROF_TC, s);
   DG_TRY(read_ctl(g, s));

@@ -7,6 +7,7 @@
 //                read-mostly 8-B entries and the 4-B counters stay L2-resident)
 //   pool       : bucket array; bucket b occupies words [b*W, (b+1)*W), W = bucket_bytes/4.
 //                words 2i, 2i+1 = (key, value) of pair i, i < BC = W/2 - 1
+//                (set variant: word i = key i, i < BC = W - 2; see Lay below)
 //                word W-2 = next bucket index of the chain (NIL = 0xFFFFFFFF)
 //                word W-1 = owner row of the bucket (for the streaming purge sweep)
 //                Base buckets of a row are consecutive (Fig. 1 caption P:L357-363);
@@ -110,6 +111,9 @@ __device__ __forceinline__ void st_v4(u32* p, uint4 v) {
   asm volatile("st.global.v4.u32 [%0], {%1,%2,%3,%4};" ::"l"(p), "r"(v.x), "r"(v.y), "r"(v.z),
                "r"(v.w) : "memory");
 }
+__device__ __forceinline__ void prefetch_l1(const void* p) {
+  asm volatile("prefetch.global.L1 [%0];" ::"l"(p));
+}
 __device__ __forceinline__ void prefetch_l2(const void* p) {
   asm volatile("prefetch.global.L2 [%0];" ::"l"(p));
 }
@@ -145,5 +149,38 @@ struct Group {
 };
 
 __device__ __forceinline__ u64 pack_pair(u32 key, u32 val) { return (u64)key | ((u64)val << 32); }
+
+__device__ __forceinline__ u32 u4c(const uint4& x, int i) {
+  return i == 0 ? x.x : i == 1 ? x.y : i == 2 ? x.z : x.w;
+}
+
+// ---------------------------------------------------------- slot layouts -------
+// A bucket is G 16-B units (W = 4G words); the last unit's words z, w hold the
+// next link and the owner row in both variants.
+//   map (S = 0): pair i = (key, value) in words 2i, 2i+1; BC = 2G-1
+//        pairs (15 per 128 B);
+//   set (S = 1): key i in word i, no values; BC = 4G-2 keys (30 per
+//        128 B).
+// Slot k of unit uu: key word 4uu + (S ? k : 2k); the last unit has half the slots.
+template <int G, int S>
+struct Lay {
+  static constexpr int W = 4 * G;
+  static constexpr int SPU = S ? 4 : 2;  // slots per 16-B unit
+  static constexpr int BC = S ? W - 2 : W / 2 - 1;
+  static constexpr int NEXT = W - 2;
+  static constexpr int OWNER = W - 1;
+  static __device__ __forceinline__ bool has(u32 uu, int k) {
+    return uu != (u32)(G - 1) || k < SPU / 2;
+  }
+  static __device__ __forceinline__ u32 key(const uint4& x, int k) { return u4c(x, S ? k : 2 * k); }
+  static __device__ __forceinline__ u32 val(const uint4& x, int k) {
+    return S ? 0u : u4c(x, 2 * k + 1);
+  }
+  static __device__ __forceinline__ u32 word(u32 uu, int k) { return 4 * uu + (S ? k : 2 * k); }
+};
+
+// layout code passed to the launchers: G | set << 5
+#define DG_LAY(G, S) ((G) | ((S) << 5))
+#define DG_FOR_LAYOUTS(X) X(2, 0) X(4, 0) X(8, 0) X(2, 1) X(4, 1) X(8, 1)
 
 }  // namespace dg

@@ -19,8 +19,10 @@ struct dg_graph_s {
   int device = 0;
   int sms = 148;
   int G = 8;              // lanes per bucket (bucket_bytes / 16)
+  bool set = false;       // set variant: keys only (DG_FLAG_SET)
+  int lay = DG_LAY(8, 0); // layout code for the launchers
   uint32_t W = 32;        // words per bucket
-  uint32_t BC = 15;       // pairs per bucket
+  uint32_t BC = 15;       // pairs (keys, set variant) per bucket
   uint32_t bucket_bytes = 128;
   uint32_t lf_milli = 700;
   uint32_t nranks = 1, rank = 0;

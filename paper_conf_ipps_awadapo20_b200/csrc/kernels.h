@@ -28,12 +28,14 @@ struct EdgeBatch {
   u32 reuse_tombstones;  // insert: install new keys in the first tombstone
 };
 
+// `lay` = DG_LAY(G, S): G 16-B units per bucket, S = 1 for the set variant
+// (keys only); launchers that take `G` are layout-independent.
 // edge ops (kernels_edges.cu)
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
                             int sms, cudaStream_t s);
-cudaError_t launch_insert(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
-cudaError_t launch_delete(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
-cudaError_t launch_query(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_delete(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
+cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
 cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s);
 u64 max_groups(int G, int sms);
 
@@ -58,23 +60,23 @@ cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s);
 cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s);
 cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
                                   cudaStream_t s);
-cudaError_t launch_export_fill(int G, const Tables& t, const u64* ro, u32* dst, u32* w,
+cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w,
                                int sms, cudaStream_t s);
 
 struct StatsOut {
   unsigned long long base_buckets, linked_buckets, live, tombs, max_chain;
 };
-cudaError_t launch_stats(int G, const Tables& t, StatsOut* out, int sms, cudaStream_t s);
+cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, int sms, cudaStream_t s);
 
 // vertex deletion (kernels_graph.cu)
 cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
                              DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s);
-cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epoch, int sms,
+cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, u32 epoch, int sms,
                               cudaStream_t s);
 // nbarr[k] = base buckets of the k-th distinct deleted vertex (0 past the count), k <= n_max
 cudaError_t launch_vdel_nb(const Tables& t, const u32* dedup, u64 n_max, u64* nbarr, int sms,
                            cudaStream_t s);
-cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, const u64* boff,
+cudaError_t launch_vdel_neighbors(int lay, const Tables& t, const u32* dedup, const u64* boff,
                                   u32 epoch, int sms, cudaStream_t s);
 cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
                               int sms, cudaStream_t s);
@@ -85,13 +87,13 @@ cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* ds
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
                                   u32 nparts, const u64* oro, u32* oadj, u32* oend, int sms,
                                   cudaStream_t s);
-cudaError_t launch_tc_wedges(int G, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
+cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s);
 
 // per-vertex re-sizing of long-chained tables (kernels_rehash.cu)
 cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
                              u64* degs, cudaStream_t s);
-cudaError_t launch_hot_export(int G, const Tables& t, u32 n, const u64* obo,
+cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
                               unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
                               int sms, cudaStream_t s);
 cudaError_t launch_hot_release(int G, const Tables& t, u32 n, const u64* obo, int sms,

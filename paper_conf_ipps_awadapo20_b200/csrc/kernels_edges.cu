@@ -89,13 +89,14 @@ struct Lanes {
   static constexpr int K = G / L;
 };
 
-template <int G, int OP, bool MAIN>
+template <int G, int S, int OP, bool MAIN>
 __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
                                         const Group<Lanes<G, OP>::L>& g, const bool valid,
                                         const u64 opid, const u64 j, const u32 stack_size,
                                         const bool reuse, u32& my_count, u32& spare,
                                         bool& bad_range) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   constexpr int L = Lanes<G, OP>::L;
   constexpr int K = Lanes<G, OP>::K;
   constexpr u32 FULL = 0xFFFFFFFFu;
@@ -159,25 +160,22 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       const u32 vr = __shfl_sync(FULL, v, srcl);
       const u32 cr = __shfl_sync(FULL, cur, srcl);
       bool lhit = false, lempty = false, lfree = false;
-      u32 hslot = 0, hval = 0, fslot = 0;
+      u32 hslot = 0, hval = 0, fslot = 0;   // key word indices in the bucket
       unsigned long long fcont = 0;
 #pragma unroll
       for (int c = 0; c < K; ++c) {
         const uint4 x = q[r][c];
         const u32 uu = K * g.gl + c;               // 16-B unit index in the bucket
-        const bool tail_unit = (uu == (u32)(G - 1));  // holds (next, owner) in z, w
-        if (pr && !lhit && x.x == vr) { lhit = true; hslot = 2 * uu; hval = x.y; }
-        const bool e0 = x.x == kEmpty;
-        lempty |= e0;
-        if (!lfree && (e0 || (reuse && x.x == kTomb))) {
-          lfree = true; fslot = 2 * uu; fcont = pack_pair(x.x, x.y);
-        }
-        if (!tail_unit) {
-          if (pr && !lhit && x.z == vr) { lhit = true; hslot = 2 * uu + 1; hval = x.w; }
-          const bool e1 = x.z == kEmpty;
-          lempty |= e1;
-          if (!lfree && (e1 || (reuse && x.z == kTomb))) {
-            lfree = true; fslot = 2 * uu + 1; fcont = pack_pair(x.z, x.w);
+#pragma unroll
+        for (int k = 0; k < LY::SPU; ++k) {
+          if (!LY::has(uu, k)) continue;           // (next, owner) words of the last unit
+          const u32 kk = LY::key(x, k);
+          if (pr && !lhit && kk == vr) { lhit = true; hslot = LY::word(uu, k); hval = LY::val(x, k); }
+          const bool e = kk == kEmpty;
+          lempty |= e;
+          if (!lfree && (e || (reuse && kk == kTomb))) {
+            lfree = true; fslot = LY::word(uu, k);
+            fcont = S ? (unsigned long long)kk : pack_pair(kk, LY::val(x, k));
           }
         }
       }
@@ -197,13 +195,13 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       } else if (OP == OP_DELETE) {
         const u32 hs = __shfl_sync(FULL, hslot, g.base + lh);
         if (mine) {
-          if (hit) { act = ACT_CAS_DEL; ff = t.pool + (u64)cur * W + 2 * hs; }
+          if (hit) { act = ACT_CAS_DEL; ff = t.pool + (u64)cur * W + hs; }
           else if (end) pend = false;
           else cur = next;
         }
       } else {  // insert
         const u32 wr = __shfl_sync(FULL, w, srcl);
-        if (lhit && g.gl == lh) st_relaxed_u32(t.pool + (u64)cr * W + 2 * hslot + 1, wr);  // replace
+        if (!S && lhit && g.gl == lh) st_relaxed_u32(t.pool + (u64)cr * W + hslot + 1, wr);  // replace
         const u32 fm = (__ballot_sync(FULL, lfree) >> g.base) & GBITS;
         const u32 lf = fm ? __ffs(fm) - 1 : 0;
         const u32 sslot = __shfl_sync(FULL, fslot, g.base + lf);
@@ -212,7 +210,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
           if (hit) {
             pend = false;
           } else {
-            if (!ff && fm) { ff = t.pool + (u64)cur * W + 2 * sslot; ffo = so; }
+            if (!ff && fm) { ff = t.pool + (u64)cur * W + sslot; ffo = so; }
             if (end) {
               act = ff ? ACT_CAS_INS : ACT_EXTEND;
             } else {
@@ -222,7 +220,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
               // metric + rehash)
               if (++steps == t.hot_steps && t.hot_flags) {
                 const u32 dr = ld_relaxed_u32(t.deg + row);
-                if (dr > nbase * Group<G>::BC) {
+                if (dr > nbase * LY::BC) {
                   const u32 bit = 1u << (row & 31);
                   if (!(atomicOr(&t.hot_flags[row >> 5], bit) & bit)) {
                     const u32 k = atomicAdd(&t.ctl->hot_count, 1u);
@@ -245,14 +243,16 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       pend = false;  // a lost CAS means another op deleted the key (Q5)
     }
     if (OP == OP_INSERT && act == ACT_CAS_INS) {
-      const unsigned long long old = atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
-                                               (unsigned long long)pack_pair(v, w));
-      if (old == ffo) {
+      // map: one 64-bit CAS installs (key, value); set: a 32-bit CAS installs the key
+      const u32 okey = S ? atomicCAS(ff, (u32)ffo, v)
+                         : (u32)atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
+                                          (unsigned long long)pack_pair(v, w));
+      if (okey == (u32)ffo) {
         atomicAdd(&t.deg[row], 1u);
         ++my_count;
         pend = false;
-      } else if ((u32)old == v) {  // a racing op installed the same key: replace
-        st_relaxed_u32(ff + 1, w);
+      } else if (okey == v) {  // a racing op installed the same key: replace
+        if (!S) st_relaxed_u32(ff + 1, w);
         pend = false;
       } else {  // the slot went to another key: re-scan from the head
         cur = head;
@@ -266,8 +266,8 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
         a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
         pend = false;
       } else {
-        st_relaxed_u32(t.pool + (u64)spare * W + Group<G>::OWNER, row);
-        const u32 old = atomicCAS(t.pool + (u64)cur * W + Group<G>::NEXT, kNil, spare);
+        st_relaxed_u32(t.pool + (u64)spare * W + LY::OWNER, row);
+        const u32 old = atomicCAS(t.pool + (u64)cur * W + LY::NEXT, kNil, spare);
         if (old == kNil) {
           cur = spare;
           spare = kNil;
@@ -291,7 +291,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
 #ifndef DG_EDGE_MINB
 #define DG_EDGE_MINB 4
 #endif
-template <int G, int OP>
+template <int G, int S, int OP>
 __global__ void __launch_bounds__(kEdgeBlock, DG_EDGE_MINB) k_edges(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<Lanes<G, OP>::L> g;
@@ -314,7 +314,7 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_EDGE_MINB) k_edges(Tables t, Ed
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
     const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
-    const bool d = run_ops<G, OP, true>(t, a, g, valid, opid, j, stack_size, reuse, my_count,
+    const bool d = run_ops<G, S, OP, true>(t, a, g, valid, opid, j, stack_size, reuse, my_count,
                                         spare, bad_range);
     const u32 dm = __ballot_sync(FULL, d);
     if (d) bl[nbl + __popc(dm & below)] = OP == OP_QUERY ? j : opid;
@@ -324,7 +324,7 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_EDGE_MINB) k_edges(Tables t, Ed
       nbl -= 32;
       const u64 op2 = bl[nbl + g.lane];
       __syncwarp();
-      run_ops<G, OP, false>(t, a, g, true, op2, op2, stack_size, reuse, my_count, spare,
+      run_ops<G, S, OP, false>(t, a, g, true, op2, op2, stack_size, reuse, my_count, spare,
                             bad_range);
     }
   }
@@ -334,7 +334,7 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_EDGE_MINB) k_edges(Tables t, Ed
     const bool valid = g.lane < take;
     const u64 op2 = valid ? bl[nbl + g.lane] : 0;
     __syncwarp();
-    run_ops<G, OP, false>(t, a, g, valid, op2, op2, stack_size, reuse, my_count, spare,
+    run_ops<G, S, OP, false>(t, a, g, valid, op2, op2, stack_size, reuse, my_count, spare,
                           bad_range);
   }
   // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
@@ -387,12 +387,12 @@ __global__ void k_fixup_alloc(Tables t) {
 }
 
 // ---------------------------------------------------------------- launchers ----
-template <int G, int OP>
+template <int G, int S, int OP>
 static int grid_for() {
   static int blocks_per_sm = -1;
   if (blocks_per_sm < 0) {
     int b = 0;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_edges<G, OP>, kEdgeBlock, 0) !=
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_edges<G, S, OP>, kEdgeBlock, 0) !=
             cudaSuccess || b <= 0)
       b = 1;
     blocks_per_sm = b;
@@ -400,36 +400,36 @@ static int grid_for() {
   return blocks_per_sm;
 }
 
-template <int G, int OP>
+template <int G, int S, int OP>
 static cudaError_t launch_g(const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
   if (a.n_ops == 0) return cudaSuccess;
   const u64 warps_needed = (a.n_ops + 31) / 32;
   const u64 per_block = kEdgeBlock / 32;
   u64 blocks = (warps_needed + per_block - 1) / per_block;
-  const u64 maxb = (u64)sms * grid_for<G, OP>();
+  const u64 maxb = (u64)sms * grid_for<G, S, OP>();
   if (blocks > maxb) blocks = maxb;
-  k_edges<G, OP><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
+  k_edges<G, S, OP><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
   return cudaGetLastError();
 }
 
 template <int OP>
-static cudaError_t launch_op(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
-  switch (G) {
-    case 2: return launch_g<2, OP>(t, a, sms, s);
-    case 4: return launch_g<4, OP>(t, a, sms, s);
-    case 8: return launch_g<8, OP>(t, a, sms, s);
+static cudaError_t launch_op(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
+  switch (lay) {
+#define DG_CASE(G, S) case DG_LAY(G, S): return launch_g<G, S, OP>(t, a, sms, s);
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
 }
 
-cudaError_t launch_insert(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
-  return launch_op<OP_INSERT>(G, t, a, sms, s);
+cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
+  return launch_op<OP_INSERT>(lay, t, a, sms, s);
 }
-cudaError_t launch_delete(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
-  return launch_op<OP_DELETE>(G, t, a, sms, s);
+cudaError_t launch_delete(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
+  return launch_op<OP_DELETE>(lay, t, a, sms, s);
 }
-cudaError_t launch_query(int G, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
-  return launch_op<OP_QUERY>(G, t, a, sms, s);
+cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
+  return launch_op<OP_QUERY>(lay, t, a, sms, s);
 }
 
 u64 max_groups(int G, int sms) {

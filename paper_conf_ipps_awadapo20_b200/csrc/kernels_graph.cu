@@ -169,10 +169,12 @@ cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t*
 }
 
 // One group per row walks every bucket chain of the row (the adjacency iterator,
-// P:L431-436) and writes the live pairs compactly at row_offsets[row].
-template <int G>
+// P:L431-436) and writes the live pairs compactly at row_offsets[row] (the set
+// variant stores no weights: w gets 0).
+template <int G, int S>
 __global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u32* dst, u32* w) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
@@ -184,43 +186,51 @@ __global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u3
       u32 b = de.base + k;
       while (b != kNil) {
         const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
-        const bool l0 = q.x < kTomb;
-        const bool l1 = !g.last() && q.z < kTomb;
-        const u32 m0 = g.ballot(l0), m1 = g.ballot(l1);
-        const u64 before = __popc(m0 & below) + __popc(m1 & below);
-        if (l0) {
-          dst[pos + before] = q.x;
-          if (w) w[pos + before] = q.y;
+        u32 before = 0, total = 0;
+#pragma unroll
+        for (int j = 0; j < LY::SPU; ++j) {
+          const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+          before += __popc(m & below);
+          total += __popc(m);
         }
-        if (l1) {
-          dst[pos + before + (l0 ? 1 : 0)] = q.z;
-          if (w) w[pos + before + (l0 ? 1 : 0)] = q.w;
+        u64 at = pos + before;
+#pragma unroll
+        for (int j = 0; j < LY::SPU; ++j) {
+          if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
+            dst[at] = LY::key(q, j);
+            if (w) w[at] = LY::val(q, j);
+            ++at;
+          }
         }
-        pos += __popc(m0) + __popc(m1);
+        pos += total;
         b = g.shfl(q.z, G - 1);
       }
     }
   }
 }
 
-cudaError_t launch_export_fill(int G, const Tables& t, const u64* ro, u32* dst, u32* w, int sms,
+cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w, int sms,
                                cudaStream_t s) {
   if (t.rows == 0) return cudaSuccess;
+  const int G = lay & 31;
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
-  switch (G) {
-    case 2: k_export_fill<2><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
-    case 4: k_export_fill<4><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
-    case 8: k_export_fill<8><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); note_kernel(1); break;
+  switch (lay) {
+#define DG_CASE(G_, S_) \
+  case DG_LAY(G_, S_): k_export_fill<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
+  note_kernel(1);
   return cudaGetLastError();
 }
 
 // --------------------------------------------------------------- statistics ----
-template <int G>
+template <int G, int S>
 __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
@@ -233,10 +243,12 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
       unsigned long long len = 0;
       while (b != kNil) {
         const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
-        const bool l0 = q.x < kTomb, l1 = !g.last() && q.z < kTomb;
-        const bool t0 = q.x == kTomb, t1 = !g.last() && q.z == kTomb;
-        live += __popc(g.ballot(l0)) + __popc(g.ballot(l1));
-        tombs += __popc(g.ballot(t0)) + __popc(g.ballot(t1));
+#pragma unroll
+        for (int j = 0; j < LY::SPU; ++j) {
+          const bool h = LY::has(g.gl, j);
+          live += __popc(g.ballot(h && LY::key(q, j) < kTomb));
+          tombs += __popc(g.ballot(h && LY::key(q, j) == kTomb));
+        }
         ++len;
         b = g.shfl(q.z, G - 1);
       }
@@ -253,17 +265,20 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
   }
 }
 
-cudaError_t launch_stats(int G, const Tables& t, StatsOut* out, int sms, cudaStream_t s) {
+cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, int sms, cudaStream_t s) {
   cudaError_t e = cudaMemsetAsync(out, 0, sizeof(StatsOut), s);
   if (e != cudaSuccess || t.rows == 0) return e;
+  const int G = lay & 31;
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
-  switch (G) {
-    case 2: k_stats<2><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
-    case 4: k_stats<4><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
-    case 8: k_stats<8><<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1); break;
+  switch (lay) {
+#define DG_CASE(G_, S_) \
+  case DG_LAY(G_, S_): k_stats<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
+  note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -301,10 +316,11 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // vertices in all hash tables"): one streaming pass over every allocated bucket
 // of the pool (coalesced, G lanes per bucket); every live key in D becomes a
 // tombstone and the owner row's degree drops by one.
-template <int G>
+template <int G, int S>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     u32 epoch) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   constexpr int U = 4;  // buckets in flight per group (memory-level parallelism)
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
@@ -322,50 +338,60 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const u64 b = b0 + (u64)k * ng;
-      u32* bp = t.pool + b * W + 4 * g.gl;
+      u32* bp = t.pool + b * W;
       const uint4 x = q[k];
       const u32 owner = g.shfl(x.w, G - 1);
-      const bool h0 = x.x < kTomb && ((__ldg(bitmap + (x.x >> 5)) >> (x.x & 31)) & 1u);
-      const bool h1 =
-          !g.last() && x.z < kTomb && ((__ldg(bitmap + (x.z >> 5)) >> (x.z & 31)) & 1u);
       u32 dec = 0;
-      if (h0 && atomicCAS(bp, x.x, kTomb) == x.x) ++dec;
-      if (h1 && atomicCAS(bp + 2, x.z, kTomb) == x.z) ++dec;
+#pragma unroll
+      for (int j = 0; j < LY::SPU; ++j) {
+        const u32 kk = LY::key(x, j);
+        if (LY::has(g.gl, j) && kk < kTomb && ((__ldg(bitmap + (kk >> 5)) >> (kk & 31)) & 1u) &&
+            atomicCAS(bp + LY::word(g.gl, j), kk, kTomb) == kk)
+          ++dec;
+      }
       if (dec) atomicSub(&t.deg[owner], dec);
     }
   }
 }
 
-cudaError_t launch_vdel_sweep(int G, const Tables& t, const u32* bitmap, u32 epoch, int sms,
+cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, u32 epoch, int sms,
                               cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
-  switch (G) {
-    case 2: k_vdel_sweep<2><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
-    case 4: k_vdel_sweep<4><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
-    case 8: k_vdel_sweep<8><<<blocks, 256, 0, s>>>(t, bitmap, epoch); note_kernel(1); break;
+  switch (lay) {
+#define DG_CASE(G_, S_) \
+  case DG_LAY(G_, S_): k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
+  note_kernel(1);
   return cudaGetLastError();
 }
 
 // probe used by the undirected purge: delete key v from the table starting at b
-template <int G>
+template <int G, int S>
 __device__ __forceinline__ int purge_delete(const Tables& t, const Group<G>& g, u32 b, u32 v) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   while (true) {
     u32* bp = t.pool + (u64)b * W;
     const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
-    const bool lastl = g.last();
-    const bool m0 = q.x == v, m1 = !lastl && q.z == v;
-    const u32 hit = g.ballot(m0 || m1);
+    bool m = false, e = false;
+    u32 wd = 0;
+#pragma unroll
+    for (int j = 0; j < LY::SPU; ++j) {
+      const bool h = LY::has(g.gl, j);
+      if (h && !m && LY::key(q, j) == v) { m = true; wd = LY::word(g.gl, j); }
+      e |= h && LY::key(q, j) == kEmpty;
+    }
+    const u32 hit = g.ballot(m);
     if (hit) {
       const u32 l = __ffs(hit) - 1;
       u32 old = 0;
-      if (g.gl == l) old = atomicCAS(bp + 4 * g.gl + (m0 ? 0 : 2), v, kTomb);
+      if (g.gl == l) old = atomicCAS(bp + wd, v, kTomb);
       return g.shfl(old, l) == v ? 1 : 0;
     }
-    const bool e0 = q.x == kEmpty, e1 = !lastl && q.z == kEmpty;
-    if (g.ballot(e0 || e1)) return 0;
+    if (g.ballot(e)) return 0;
     const u32 next = g.shfl(q.z, G - 1);
     if (next == kNil) return 0;
     b = next;
@@ -407,10 +433,11 @@ __device__ __forceinline__ u32 owner_of(const u64* boff, u32 cnt, u64 x) {
 // Undirected purge, Alg. 2: for every deleted vertex u,
 // iterate over A_u (L11-12) and delete u from A_v of every neighbour v (L13-17).
 // Valid only for graphs kept symmetric (directed = 0, single rank).
-template <int G>
+template <int G, int S>
 __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* dedup,
                                                         const u64* boff, u32 epoch) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
@@ -424,33 +451,34 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
     u32 b = t.dir[u].base + (u32)(x - boff[k]);
     while (b != kNil) {
       const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
-      u32 lm0 = g.ballot(q.x < kTomb);
-      u32 lm1 = g.ballot(!g.last() && q.z < kTomb);
-      while (lm0 | lm1) {
-        const u32 l = __ffs(lm0 | lm1) - 1;
-        const bool s0 = (lm0 >> l) & 1u;
-        const u32 x0 = g.shfl(q.x, l), x1 = g.shfl(q.z, l);
-        const u32 v = s0 ? x0 : x1;
-        if (s0) lm0 &= ~(1u << l);
-        else lm1 &= ~(1u << l);
-        const DirEntry dv = t.dir[v];
-        if (purge_delete<G>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
-          atomicSub(&t.deg[v], 1u);
+#pragma unroll
+      for (int j = 0; j < LY::SPU; ++j) {
+        u32 lm = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+        while (lm) {
+          const u32 l = __ffs(lm) - 1;
+          lm &= lm - 1;
+          const u32 v = g.shfl(LY::key(q, j), l);
+          const DirEntry dv = t.dir[v];
+          if (purge_delete<G, S>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
+            atomicSub(&t.deg[v], 1u);
+        }
       }
       b = g.shfl(q.z, G - 1);
     }
   }
 }
 
-cudaError_t launch_vdel_neighbors(int G, const Tables& t, const u32* dedup, const u64* boff,
+cudaError_t launch_vdel_neighbors(int lay, const Tables& t, const u32* dedup, const u64* boff,
                                   u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
-  switch (G) {
-    case 2: k_vdel_neighbors<2><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
-    case 4: k_vdel_neighbors<4><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
-    case 8: k_vdel_neighbors<8><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+  switch (lay) {
+#define DG_CASE(G_, S_) \
+  case DG_LAY(G_, S_): k_vdel_neighbors<G_, S_><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
+  note_kernel(1);
   return cudaGetLastError();
 }
 

@@ -49,11 +49,12 @@ __device__ __forceinline__ u32 seg_of(const u64* off, u32 cnt, u64 x) {
 }
 
 // one group per (flagged row, old base bucket): walk the chain, append live pairs
-template <int G>
+template <int G, int S>
 __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* obo,
                                                     unsigned long long* cursor, u32* osrc,
                                                     u32* odst, u32* ow, u32 rank) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   const Group<G> g;
   const u64 total = obo[n];
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
@@ -66,23 +67,24 @@ __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* 
     u32 b = t.dir[row].base + (u32)(x - obo[k]);
     while (b != kNil) {
       const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
-      const bool l0 = q.x < kTomb, l1 = !g.last() && q.z < kTomb;
-      const u32 m0 = g.ballot(l0), m1 = g.ballot(l1);
-      const u32 cnt = __popc(m0) + __popc(m1);
+      u32 before = 0, cnt = 0;
+#pragma unroll
+      for (int j = 0; j < LY::SPU; ++j) {
+        const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+        before += __popc(m & below);
+        cnt += __popc(m);
+      }
       unsigned long long pos = 0;
       if (g.gl == 0 && cnt) pos = atomicAdd(cursor + k, (unsigned long long)cnt);
-      pos = g.shfl(pos, 0);
-      const u64 before = __popc(m0 & below) + __popc(m1 & below);
-      if (l0) {
-        osrc[pos + before] = gid_u;
-        odst[pos + before] = q.x;
-        ow[pos + before] = q.y;
-      }
-      if (l1) {
-        const u64 at = pos + before + (l0 ? 1 : 0);
-        osrc[at] = gid_u;
-        odst[at] = q.z;
-        ow[at] = q.w;
+      u64 at = g.shfl(pos, 0) + before;
+#pragma unroll
+      for (int j = 0; j < LY::SPU; ++j) {
+        if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
+          osrc[at] = gid_u;
+          odst[at] = LY::key(q, j);
+          ow[at] = LY::val(q, j);
+          ++at;
+        }
       }
       b = g.shfl(q.z, G - 1);
     }
@@ -139,14 +141,17 @@ cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* 
   return cudaGetLastError();
 }
 
-cudaError_t launch_hot_export(int G, const Tables& t, u32 n, const u64* obo,
+cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
                               unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
                               int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
-  switch (G) {
-    case 2: k_hot_export<2><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
-    case 4: k_hot_export<4><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
-    case 8: k_hot_export<8><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); break;
+  switch (lay) {
+#define DG_CASE(G_, S_)                                                                    \
+  case DG_LAY(G_, S_):                                                                     \
+    k_hot_export<G_, S_><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); \
+    break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
   note_kernel(1);

@@ -83,11 +83,12 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
 // 16-B load per lane per candidate), then decides all G with group ballots.  Warp
 // loops are warp-uniform so every intrinsic uses the full mask.  The rare probes
 // whose key may sit further down a chain are walked by their own lane.
-template <int G>
+template <int G, int S>
 __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __restrict__ oadj,
                                                       const u32* __restrict__ oend, u64 n_units,
                                                       unsigned long long* count) {
-  constexpr int W = Group<G>::W;
+  typedef Lay<G, S> LY;
+  constexpr int W = LY::W;
   constexpr u32 FULL = 0xFFFFFFFFu;
   constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
   constexpr int PER_WARP = 32 / G;
@@ -122,10 +123,15 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
         const uint4 x = q[r];
         const u32 wr = __shfl_sync(FULL, w, g.base + r);
         const bool pr = (amask >> (g.base + r)) & 1u;
-        const bool m = pr && (x.x == wr || (!lastl && x.z == wr));
-        const u32 hit = (__ballot_sync(FULL, m) >> g.base) & GBITS;
-        const bool e0 = x.x == kEmpty, e1 = !lastl && x.z == kEmpty;
-        const u32 em = (__ballot_sync(FULL, e0 || e1) >> g.base) & GBITS;
+        bool m = false, e = false;
+#pragma unroll
+        for (int j = 0; j < LY::SPU; ++j) {
+          const bool h = !lastl || j < LY::SPU / 2;
+          m |= h && LY::key(x, j) == wr;
+          e |= h && LY::key(x, j) == kEmpty;
+        }
+        const u32 hit = (__ballot_sync(FULL, pr && m) >> g.base) & GBITS;
+        const u32 em = (__ballot_sync(FULL, e) >> g.base) & GBITS;
         const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
         if (pr && g.gl == (u32)r) {
           if (hit) ++hits;
@@ -142,14 +148,14 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
 #pragma unroll
           for (int c = 0; c < G; ++c) {
             const uint4 y = __ldg(bp + c);
-            found |= y.x == w;
-            ended |= y.x == kEmpty;
-            if (c < G - 1) {
-              found |= y.z == w;
-              ended |= y.z == kEmpty;
-            } else {
-              nb2 = y.z;
+#pragma unroll
+            for (int j = 0; j < LY::SPU; ++j) {
+              if (LY::has(c, j)) {
+                found |= LY::key(y, j) == w;
+                ended |= LY::key(y, j) == kEmpty;
+              }
             }
+            if (c == G - 1) nb2 = y.z;
           }
           if (found) { ++hits; break; }
           if (ended) break;
@@ -178,15 +184,19 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
   return cudaGetLastError();
 }
 
-cudaError_t launch_tc_wedges(int G, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
+cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s) {
   if (n_units == 0) return cudaSuccess;
+  const int G = lay & 31;
   u64 blocks = (n_units * G + 255) / 256;
   if (blocks > (u64)sms * 4) blocks = (u64)sms * 4;
-  switch (G) {
-    case 2: k_tc_wedges<2><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); break;
-    case 4: k_tc_wedges<4><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); break;
-    case 8: k_tc_wedges<8><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); break;
+  switch (lay) {
+#define DG_CASE(G_, S_)                                                                     \
+  case DG_LAY(G_, S_):                                                                      \
+    k_tc_wedges<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); \
+    break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
   note_kernel(1);

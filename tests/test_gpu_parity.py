@@ -35,7 +35,7 @@ def test_golden_scripts_on_gpu(name, bb):
     run_script(load(name), lambda n, directed: GpuAdapter(n, directed, bucket_bytes=bb))
 
 
-def _config1_stream(bb, hints, directed, seed=1, reuse=True):
+def _config1_stream(bb, hints, directed, seed=1, reuse=True, set_variant=False):
     """Config 1 (BASELINE.json configs[0]; SURVEY §8(d) cfg 1): |V| = 1,024;
     16 insert batches of 1,024 (5% forced intra-batch duplicates with distinct
     weights), queries, deletes, vertex deletions, re-insertion, growth and an
@@ -43,14 +43,19 @@ def _config1_stream(bb, hints, directed, seed=1, reuse=True):
     from paper_conf_ipps_awadapo20_b200 import DGError, DG_ERR_VERTEX_OUT_OF_RANGE, Graph
     nv = 1024
     hint = wl.out_degrees(wl.uniform_edges(seed, 0, 16 * 1024, nv)[0], nv) if hints else None
-    g = Graph(nv, hint, bucket_bytes=bb, directed=directed, reuse_tombstones=reuse)
+    g = Graph(nv, hint, bucket_bytes=bb, directed=directed, reuse_tombstones=reuse,
+              set_variant=set_variant)
     o = Oracle(nv, directed)
+
+    def ow(w):  # the set variant stores no weights: the oracle sees 0
+        return np.zeros_like(w) if set_variant else w
+
     stream = 1000
     for b in range(16):
         s, d, w = wl.uniform_edges(seed, stream + b, 1024, nv)
         k = 51  # 5%: repeat earlier keys of the same batch with distinct weights
         s[-k:], d[-k:] = s[:k], d[:k]
-        st, added = o.insert_edges(s, d, w)
+        st, added = o.insert_edges(s, d, ow(w))
         assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
         cand = check_against_oracle(g, o, f"insert batch {b}")
         # queries: half live (from the oracle's export), half uniform
@@ -78,7 +83,7 @@ def _config1_stream(bb, hints, directed, seed=1, reuse=True):
         s, d, w = wl.uniform_edges(seed, 9500 + b, 256, nv)
         s[:128] = ids[np.arange(128) % ids.size]
         d[128:] = ids[np.arange(128) % ids.size]
-        st, added = o.insert_edges(s, d, w)
+        st, added = o.insert_edges(s, d, ow(w))
         assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
         check_against_oracle(g, o, f"re-insert {b}")
     # growth: vertex insertion 1024..1279, then 1,024 edges over [0, 1280)
@@ -87,7 +92,7 @@ def _config1_stream(bb, hints, directed, seed=1, reuse=True):
     o.insert_vertices(new)
     assert g.num_vertices == 1280
     s, d, w = wl.uniform_edges(seed, 9900, 1024, 1280)
-    st, added = o.insert_edges(s, d, w)
+    st, added = o.insert_edges(s, d, ow(w))
     assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == added
     check_against_oracle(g, o, "after growth")
     # out-of-range batch: rejected, graph unchanged (Q7)
@@ -121,6 +126,36 @@ def test_config1_undirected(bb):
 def test_config1_append_only(bb):
     """The paper's default policy: tombstones are never reused."""
     _config1_stream(bb, False, True, seed=4, reuse=False)
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("directed", [True, False])
+def test_config1_set_variant(bb, directed):
+    """Set variant (keys only): the config-1 stream
+    against the oracle with weights read as 0."""
+    _config1_stream(bb, directed, directed, seed=11, set_variant=True)
+
+
+@pytest.mark.parametrize("bb", GEOMS)
+def test_set_variant_bucket_capacity(bb):
+    """A set bucket holds 30 keys per 128 B, W/4-2 in general: one vertex
+    without a hint (one bucket) takes exactly Bc neighbours before its
+    first overflow bucket; hinted tables get ceil(hint / (0.7 Bc)) base buckets."""
+    from oracle import initial_buckets
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    bc = bb // 4 - 2
+    nv = 4 * bc + 8
+    g = Graph(nv, set_variant=True, bucket_bytes=bb)
+    g.insert_edges(cuda(np.zeros(bc, np.uint32)), cuda(np.arange(1, bc + 1, dtype=np.uint32)))
+    st = g.stats()
+    assert st["overflow_buckets"] == 0 and st["live_pairs"] == bc
+    g.insert_edges(cuda([0]), cuda([bc + 1]))
+    assert g.stats()["overflow_buckets"] == 1
+    hints = np.arange(nv, dtype=np.uint32) * 3
+    h = Graph(nv, hints, set_variant=True, bucket_bytes=bb)
+    assert h.stats()["base_buckets"] == sum(initial_buckets(int(x), 700, bc) for x in hints)
+    g.close()
+    h.close()
 
 
 @pytest.mark.parametrize("reuse", [True, False])
@@ -412,30 +447,33 @@ def _golden_triangles():
     return out
 
 
+@pytest.mark.parametrize("set_variant", [False, True])
 @pytest.mark.parametrize("bb", GEOMS)
-def test_tc_golden_and_closed_forms(bb):
+def test_tc_golden_and_closed_forms(bb, set_variant):
     import math
     from paper_conf_ipps_awadapo20_b200 import Graph
     for name, n, want, edges in _golden_triangles():
-        g = Graph(n, directed=False, bucket_bytes=bb)
+        g = Graph(n, directed=False, bucket_bytes=bb, set_variant=set_variant)
         g.insert_edges(cuda([e[0] for e in edges]), cuda([e[1] for e in edges]))
         assert g.triangle_count() == want, name
     for n in (3, 10, 47):
         iu, ju = np.triu_indices(n, 1)
-        g = Graph(n, directed=False, bucket_bytes=bb)
+        g = Graph(n, directed=False, bucket_bytes=bb, set_variant=set_variant)
         g.insert_edges(cuda(iu), cuda(ju))
         assert g.triangle_count() == math.comb(n, 3)
 
 
+@pytest.mark.parametrize("set_variant", [False, True])
 @pytest.mark.parametrize("bb", GEOMS)
-def test_tc_matches_oracle_rmat(bb):
+def test_tc_matches_oracle_rmat(bb, set_variant):
     """Hash-intersection TC (GPU) vs the forward algorithm on sorted lists (oracle)
     on a symmetrised R-MAT graph; the part/nparts split sums to the total."""
     from paper_conf_ipps_awadapo20_b200 import Graph
     scale = 15
     nv = 1 << scale
     s, d = wl.rmat_edges(5, 0, 400_000, scale, wl.GRAPH500)
-    g = Graph(nv, wl.out_degrees(np.concatenate([s, d]), nv), directed=False, bucket_bytes=bb)
+    g = Graph(nv, wl.out_degrees(np.concatenate([s, d]), nv), directed=False, bucket_bytes=bb,
+              set_variant=set_variant)
     o = Oracle(nv, directed=False)
     g.insert_edges(cuda(s), cuda(d))
     o.insert_edges(s, d)
