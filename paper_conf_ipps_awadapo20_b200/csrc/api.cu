@@ -52,7 +52,9 @@ cudaError_t ensure_buf(dg_graph_s::Buf& b, size_t bytes) {
   if (b.p) cudaFree(b.p);
   b.p = nullptr;
   b.bytes = 0;
-  size_t want = std::max<size_t>(bytes, 1 << 20);
+  // geometric headroom: buffers that track a growing graph (TC scratch, export
+  // staging) are not re-allocated (cudaFree synchronises the device) every call
+  size_t want = std::max<size_t>(bytes + bytes / 4, 1 << 20);
   cudaError_t e = cudaMalloc(&b.p, want);
   if (e == cudaSuccess) b.bytes = want;
   return e;
