@@ -479,6 +479,7 @@ static void destroy_graph(dg_graph g) {
     if (b.p) cudaFree(b.p);
   for (auto& b : g->rh)
     if (b.p) cudaFree(b.p);
+  if (g->big.p) cudaFree(g->big.p);
   if (g->hot_flags) cudaFree(g->hot_flags);
   if (g->hot_list) cudaFree(g->hot_list);
   if (g->h_hot) cudaFreeHost(g->h_hot);
@@ -953,7 +954,9 @@ dg_status dg_export_adjacency(dg_graph g, uint64_t* row_offsets, uint32_t* dst, 
     void *dd = nullptr, *dw = nullptr;
     DG_TRY(stage_out(g, 4, dst, m * 4, &dd, &host));
     DG_TRY(stage_out(g, 7, weight, weight ? m * 4 : 0, &dw, &host));
-    DG_CK(dg::launch_export_fill(g->lay, t, (const u64*)dro, (u32*)dd, (u32*)dw, g->sms, s));
+    DG_CK(ensure_buf(g->big, (g->rows + 2) * 4));
+    DG_CK(dg::launch_export_fill(g->lay, t, (const u64*)dro, (u32*)dd, (u32*)dw, (u32*)g->big.p,
+                                 g->sms, s));
     DG_TRY(finish_out(g, dst, dd, m * 4, s));
     DG_TRY(finish_out(g, weight, dw, weight ? m * 4 : 0, s));
   }
@@ -983,7 +986,8 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   dg::StatsOut h{};
   auto* d = reinterpret_cast<dg::StatsOut*>(g->stats_dev);
-  DG_CK(dg::launch_stats(g->lay, g->tables(), d, g->sms, s));
+  DG_CK(ensure_buf(g->big, (g->rows + 2) * 4));
+  DG_CK(dg::launch_stats(g->lay, g->tables(), d, (u32*)g->big.p, g->sms, s));
   DG_CK(cudaMemcpyAsync(&h, d, sizeof(h), cudaMemcpyDeviceToHost, s));
   if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   g->snap_pending = false;
@@ -1036,13 +1040,15 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   if (m >= 0xFFFFFFFFull) return DG_ERR_UNSUPPORTED;
   DG_CK(ensure_buf(g->tc[1], m * 4 + 4));
   u32* dst = reinterpret_cast<u32*>(g->tc[1].p);
-  DG_CK(dg::launch_export_fill(g->lay, t, ro, dst, nullptr, g->sms, s));
+  DG_CK(ensure_buf(g->big, (rows + 2) * 4));
+  u32* big = reinterpret_cast<u32*>(g->big.p);
+  DG_CK(dg::launch_export_fill(g->lay, t, ro, dst, nullptr, big, g->sms, s));
   // (2) orientation by rank = (degree, id)
   DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8));
   DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8));
   u64* ocnt = reinterpret_cast<u64*>(g->tc[2].p);
   u64* oro = reinterpret_cast<u64*>(g->tc[3].p);
-  DG_CK(dg::launch_tc_orient_count(t, ro, dst, part, nparts, ocnt, g->sms, s));
+  DG_CK(dg::launch_tc_orient_count(t, ro, dst, part, nparts, ocnt, big, g->sms, s));
   DG_CK(dg::scan_exclusive_u64(ocnt, oro, rows + 1, &g->scan_temp, &g->scan_bytes, s));
   u64 mo = 0;
   DG_CK(cudaMemcpyAsync(&mo, oro + rows, 8, cudaMemcpyDeviceToHost, s));
@@ -1051,7 +1057,7 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   DG_CK(ensure_buf(g->tc[5], mo * 4 + 4));
   u32* oadj = reinterpret_cast<u32*>(g->tc[4].p);
   u32* oend = reinterpret_cast<u32*>(g->tc[5].p);
-  DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, g->sms, s));
+  DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, big, g->sms, s));
   // (3) one edgeExist per wedge
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);

@@ -62,6 +62,7 @@ struct dg_graph_s {
   } stage[8];
   Buf tc[6];  // triangle counting scratch (CSR, orientation)
   Buf rh[4];  // re-sizing scratch
+  Buf big;    // hub-row list (export, stats, TC orientation)
   // per-vertex re-sizing of long chains
   uint32_t* hot_flags = nullptr;
   uint64_t hot_words = 0;

@@ -8,6 +8,10 @@
 namespace dg {
 
 constexpr int kEdgeBlock = 256;
+// rows with more base buckets than this are walked by a whole block (export, stats)
+constexpr u32 kBigRowBuckets = 32;
+// rows with more neighbours than this are oriented by a whole block (TC)
+constexpr u32 kBigRowDegree = 1024;
 
 // process-wide count of kernels launched by the library (dg_profile.launches)
 void note_kernel(int n);
@@ -60,13 +64,14 @@ cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s);
 cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s);
 cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
                                   cudaStream_t s);
-cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w,
+// big: scratch u32[2 + rows] (hub-row list)
+cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w, u32* big,
                                int sms, cudaStream_t s);
 
 struct StatsOut {
   unsigned long long base_buckets, linked_buckets, live, tombs, max_chain;
 };
-cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, int sms, cudaStream_t s);
+cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s);
 
 // vertex deletion (kernels_graph.cu)
 cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
@@ -83,10 +88,10 @@ cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u6
 
 // triangle counting consumer (kernels_tc.cu)
 cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* dst, u32 part,
-                                   u32 nparts, u64* ocnt, int sms, cudaStream_t s);
+                                   u32 nparts, u64* ocnt, u32* big, int sms, cudaStream_t s);
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
-                                  u32 nparts, const u64* oro, u32* oadj, u32* oend, int sms,
-                                  cudaStream_t s);
+                                  u32 nparts, const u64* oro, u32* oadj, u32* oend,
+                                  const u32* big, int sms, cudaStream_t s);
 cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s);
 

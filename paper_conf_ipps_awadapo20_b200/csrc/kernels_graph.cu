@@ -170,67 +170,139 @@ cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t*
 
 // One group per row walks every bucket chain of the row (the adjacency iterator,
 // P:L431-436) and writes the live pairs compactly at row_offsets[row] (the set
-// variant stores no weights: w gets 0).
+// variant stores no weights: w gets 0).  Rows with more than kBigRowBuckets base
+// buckets (hubs) are listed in big[1..] (count in big[0]) and exported by
+// k_export_big, one block per row, so one group never walks a hub's thousands of
+// buckets alone.  The order of a row's entries is unspecified.
 template <int G, int S>
-__global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u32* dst, u32* w) {
+__device__ __forceinline__ u32 export_bucket(const Group<G>& g, const uint4& q, u32* dst, u32* w,
+                                             u64 pos) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
+  const u32 below = (1u << g.gl) - 1u;
+  u32 before = 0, total = 0;
+#pragma unroll
+  for (int j = 0; j < LY::SPU; ++j) {
+    const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+    before += __popc(m & below);
+    total += __popc(m);
+  }
+  u64 at = pos + before;
+#pragma unroll
+  for (int j = 0; j < LY::SPU; ++j) {
+    if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
+      dst[at] = LY::key(q, j);
+      if (w) w[at] = LY::val(q, j);
+      ++at;
+    }
+  }
+  return total;
+}
+
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u32* dst, u32* w,
+                                                     u32* big) {
+  constexpr int W = Lay<G, S>::W;
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
-  const u32 below = (1u << g.gl) - 1u;
   for (u64 row = gid; row < t.rows; row += ng) {
     const DirEntry de = t.dir[row];
+    if (de.nb > kBigRowBuckets) {
+      if (g.gl == 0) big[1 + atomicAdd(big, 1u)] = (u32)row;
+      continue;
+    }
     u64 pos = ro[row];
     for (u32 k = 0; k < de.nb; ++k) {
       u32 b = de.base + k;
       while (b != kNil) {
         const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
-        u32 before = 0, total = 0;
-#pragma unroll
-        for (int j = 0; j < LY::SPU; ++j) {
-          const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
-          before += __popc(m & below);
-          total += __popc(m);
-        }
-        u64 at = pos + before;
-#pragma unroll
-        for (int j = 0; j < LY::SPU; ++j) {
-          if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
-            dst[at] = LY::key(q, j);
-            if (w) w[at] = LY::val(q, j);
-            ++at;
-          }
-        }
-        pos += total;
+        pos += export_bucket<G, S>(g, q, dst, w, pos);
         b = g.shfl(q.z, G - 1);
       }
     }
   }
 }
 
-cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w, int sms,
-                               cudaStream_t s) {
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_export_big(Tables t, const u64* ro, u32* dst, u32* w,
+                                                    const u32* big) {
+  constexpr int W = Lay<G, S>::W;
+  __shared__ unsigned long long cursor;
+  const Group<G> g;
+  const u32 gib = threadIdx.x / G, ngb = blockDim.x / G;
+  const u32 nbig = big[0];
+  for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
+    const u32 row = big[1 + i];
+    const DirEntry de = t.dir[row];
+    __syncthreads();
+    if (threadIdx.x == 0) cursor = ro[row];
+    __syncthreads();
+    for (u32 k = gib; k < de.nb; k += ngb) {
+      u32 b = de.base + k;
+      while (b != kNil) {
+        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
+        u32 cnt = 0;
+#pragma unroll
+        for (int j = 0; j < Lay<G, S>::SPU; ++j)
+          cnt += __popc(g.ballot(Lay<G, S>::has(g.gl, j) && Lay<G, S>::key(q, j) < kTomb));
+        unsigned long long pos = 0;
+        if (g.gl == 0 && cnt) pos = atomicAdd(&cursor, (unsigned long long)cnt);
+        export_bucket<G, S>(g, q, dst, w, g.shfl(pos, 0));
+        b = g.shfl(q.z, G - 1);
+      }
+    }
+  }
+}
+
+cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst, u32* w, u32* big,
+                               int sms, cudaStream_t s) {
   if (t.rows == 0) return cudaSuccess;
   const int G = lay & 31;
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
+  cudaError_t e = cudaMemsetAsync(big, 0, 4, s);
+  if (e != cudaSuccess) return e;
   switch (lay) {
-#define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_export_fill<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w); break;
+#define DG_CASE(G_, S_)                                                                   \
+  case DG_LAY(G_, S_):                                                                    \
+    k_export_fill<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w, big);           \
+    k_export_big<G_, S_><<<(unsigned)sms * 2, 256, 0, s>>>(t, ro, dst, w, big); \
+    break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
+  note_kernel(2);
   return cudaGetLastError();
 }
 
 // --------------------------------------------------------------- statistics ----
+// one base-bucket chain: live / tombstone slots and its length
 template <int G, int S>
-__global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
+__device__ __forceinline__ void stats_chain(const Tables& t, const Group<G>& g, u32 b,
+                                            unsigned long long& live, unsigned long long& tombs,
+                                            unsigned long long& linked, unsigned long long& maxc) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
+  unsigned long long len = 0;
+  while (b != kNil) {
+    const uint4 q = ld_nc_v4(t.pool + (u64)b * LY::W + 4 * g.gl);
+#pragma unroll
+    for (int j = 0; j < LY::SPU; ++j) {
+      const bool h = LY::has(g.gl, j);
+      live += __popc(g.ballot(h && LY::key(q, j) < kTomb));
+      tombs += __popc(g.ballot(h && LY::key(q, j) == kTomb));
+    }
+    ++len;
+    b = g.shfl(q.z, G - 1);
+  }
+  linked += len;
+  if (len > maxc) maxc = len;
+}
+
+// group per row; hub rows (> kBigRowBuckets base buckets) are split over the
+// groups of one block by k_stats_big
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out, u32* big) {
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
@@ -238,23 +310,11 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
   for (u64 row = gid; row < t.rows; row += ng) {
     const DirEntry de = t.dir[row];
     nbase += de.nb;
-    for (u32 k = 0; k < de.nb; ++k) {
-      u32 b = de.base + k;
-      unsigned long long len = 0;
-      while (b != kNil) {
-        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
-#pragma unroll
-        for (int j = 0; j < LY::SPU; ++j) {
-          const bool h = LY::has(g.gl, j);
-          live += __popc(g.ballot(h && LY::key(q, j) < kTomb));
-          tombs += __popc(g.ballot(h && LY::key(q, j) == kTomb));
-        }
-        ++len;
-        b = g.shfl(q.z, G - 1);
-      }
-      linked += len;
-      if (len > maxc) maxc = len;
+    if (de.nb > kBigRowBuckets) {
+      if (g.gl == 0) big[1 + atomicAdd(big, 1u)] = (u32)row;
+      continue;
     }
+    for (u32 k = 0; k < de.nb; ++k) stats_chain<G, S>(t, g, de.base + k, live, tombs, linked, maxc);
   }
   if (g.gl == 0) {
     atomicAdd(&out->base_buckets, nbase);
@@ -265,20 +325,42 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out) {
   }
 }
 
-cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, int sms, cudaStream_t s) {
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_stats_big(Tables t, StatsOut* out, const u32* big) {
+  const Group<G> g;
+  const u32 gib = threadIdx.x / G, ngb = blockDim.x / G;
+  unsigned long long linked = 0, live = 0, tombs = 0, maxc = 0;
+  const u32 nbig = big[0];
+  for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
+    const DirEntry de = t.dir[big[1 + i]];
+    for (u32 k = gib; k < de.nb; k += ngb) stats_chain<G, S>(t, g, de.base + k, live, tombs, linked, maxc);
+  }
+  if (g.gl == 0 && (linked | live | tombs)) {
+    atomicAdd(&out->linked_buckets, linked);
+    atomicAdd(&out->live, live);
+    atomicAdd(&out->tombs, tombs);
+    atomicMax(&out->max_chain, maxc);
+  }
+}
+
+cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s) {
   cudaError_t e = cudaMemsetAsync(out, 0, sizeof(StatsOut), s);
+  if (e == cudaSuccess) e = cudaMemsetAsync(big, 0, 4, s);
   if (e != cudaSuccess || t.rows == 0) return e;
   const int G = lay & 31;
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   switch (lay) {
-#define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_stats<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, out); break;
+#define DG_CASE(G_, S_)                                                      \
+  case DG_LAY(G_, S_):                                                       \
+    k_stats<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, out, big);           \
+    k_stats_big<G_, S_><<<(unsigned)sms * 2, 256, 0, s>>>(t, out, big); \
+    break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
+  note_kernel(2);
   return cudaGetLastError();
 }
 

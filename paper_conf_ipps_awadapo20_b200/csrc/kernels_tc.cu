@@ -24,17 +24,24 @@ __device__ __forceinline__ bool rank_less(u32 du, u32 u, u32 dv, u32 v) {
   return du < dv || (du == dv && u < v);
 }
 
+// warp per row; rows with more than kBigRowDegree neighbours (hubs) are listed in
+// big[1..] (count big[0]) and oriented by the *_big kernels, one block per row.
 __global__ void __launch_bounds__(256) k_tc_orient_count(const u64* ro, const u32* dst,
                                                          const u32* deg, u64 rows, u32 part,
-                                                         u32 nparts, u64* ocnt) {
+                                                         u32 nparts, u64* ocnt, u32* big) {
   const u32 lane = threadIdx.x & 31;
   const u64 wid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nw = ((u64)gridDim.x * blockDim.x) >> 5;
   for (u64 u = wid; u < rows; u += nw) {
     u32 c = 0;
     if (u % nparts == part) {
+      const u64 r0 = ro[u], r1 = ro[u + 1];
+      if (r1 - r0 > kBigRowDegree) {
+        if (lane == 0) big[1 + atomicAdd(big, 1u)] = (u32)u;
+        continue;
+      }
       const u32 du = deg[u];
-      for (u64 k = ro[u] + lane; k < ro[u + 1]; k += 32) {
+      for (u64 k = r0 + lane; k < r1; k += 32) {
         const u32 v = dst[k];
         c += rank_less(du, (u32)u, __ldg(&deg[v]), v) ? 1u : 0u;
       }
@@ -43,6 +50,29 @@ __global__ void __launch_bounds__(256) k_tc_orient_count(const u64* ro, const u3
     if (lane == 0) ocnt[u] = c;
   }
   if (blockIdx.x == 0 && threadIdx.x == 0) ocnt[rows] = 0;
+}
+
+__global__ void __launch_bounds__(256) k_tc_orient_count_big(const u64* ro, const u32* dst,
+                                                             const u32* deg, u64* ocnt,
+                                                             const u32* big) {
+  __shared__ u32 total;
+  const u32 nbig = big[0];
+  for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
+    const u32 u = big[1 + i];
+    const u32 du = deg[u];
+    __syncthreads();
+    if (threadIdx.x == 0) total = 0;
+    __syncthreads();
+    u32 c = 0;
+    for (u64 k = ro[u] + threadIdx.x; k < ro[u + 1]; k += blockDim.x) {
+      const u32 v = dst[k];
+      c += rank_less(du, u, __ldg(&deg[v]), v) ? 1u : 0u;
+    }
+    c = __reduce_add_sync(0xFFFFFFFFu, c);
+    if ((threadIdx.x & 31) == 0 && c) atomicAdd(&total, c);
+    __syncthreads();
+    if (threadIdx.x == 0) ocnt[u] = total;
+  }
 }
 
 __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32* dst,
@@ -54,6 +84,7 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
   const u64 nw = ((u64)gridDim.x * blockDim.x) >> 5;
   for (u64 u = wid; u < rows; u += nw) {
     if (u % nparts != part) continue;
+    if (ro[u + 1] - ro[u] > kBigRowDegree) continue;  // k_tc_orient_fill_big
     const u32 du = deg[u];
     u64 pos = oro[u];
     const u32 end = (u32)oro[u + 1];
@@ -72,6 +103,42 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill(const u64* ro, const u32
         oend[at] = end;
       }
       pos += __popc(m);
+    }
+  }
+}
+
+// hub rows: warps of one block take 32-entry pieces; positions from a block cursor
+// (the order of N+(u) is immaterial: every pair i < j is probed once)
+__global__ void __launch_bounds__(256) k_tc_orient_fill_big(const u64* ro, const u32* dst,
+                                                            const u32* deg, const u64* oro,
+                                                            u32* oadj, u32* oend, const u32* big) {
+  __shared__ unsigned long long cursor;
+  const u32 lane = threadIdx.x & 31;
+  const u32 nbig = big[0];
+  for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
+    const u32 u = big[1 + i];
+    const u32 du = deg[u];
+    const u32 end = (u32)oro[u + 1];
+    __syncthreads();
+    if (threadIdx.x == 0) cursor = oro[u];
+    __syncthreads();
+    for (u64 k0 = ro[u] + (threadIdx.x & ~31u); k0 < ro[u + 1]; k0 += blockDim.x) {
+      const u64 k = k0 + lane;
+      bool keep = false;
+      u32 v = 0;
+      if (k < ro[u + 1]) {
+        v = dst[k];
+        keep = rank_less(du, u, __ldg(&deg[v]), v);
+      }
+      const u32 m = __ballot_sync(0xFFFFFFFFu, keep);
+      unsigned long long pos = 0;
+      if (lane == 0 && m) pos = atomicAdd(&cursor, (unsigned long long)__popc(m));
+      pos = __shfl_sync(0xFFFFFFFFu, pos, 0);
+      if (keep) {
+        const u64 at = pos + __popc(m & ((1u << lane) - 1u));
+        oadj[at] = v;
+        oend[at] = end;
+      }
     }
   }
 }
@@ -169,18 +236,24 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
 }
 
 cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* dst, u32 part,
-                                   u32 nparts, u64* ocnt, int sms, cudaStream_t s) {
-  k_tc_orient_count<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, ocnt);
-  note_kernel(1);
+                                   u32 nparts, u64* ocnt, u32* big, int sms, cudaStream_t s) {
+  cudaError_t e = cudaMemsetAsync(big, 0, 4, s);
+  if (e != cudaSuccess) return e;
+  k_tc_orient_count<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, ocnt,
+                                                      big);
+  k_tc_orient_count_big<<<(unsigned)sms * 2, 256, 0, s>>>(ro, dst, t.deg, ocnt, big);
+  note_kernel(2);
   return cudaGetLastError();
 }
 
+// big: the hub-row list left by launch_tc_orient_count
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
-                                  u32 nparts, const u64* oro, u32* oadj, u32* oend, int sms,
-                                  cudaStream_t s) {
+                                  u32 nparts, const u64* oro, u32* oadj, u32* oend,
+                                  const u32* big, int sms, cudaStream_t s) {
   k_tc_orient_fill<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, oro, oadj,
                                                      oend);
-  note_kernel(1);
+  k_tc_orient_fill_big<<<(unsigned)sms * 2, 256, 0, s>>>(ro, dst, t.deg, oro, oadj, oend, big);
+  note_kernel(2);
   return cudaGetLastError();
 }
 

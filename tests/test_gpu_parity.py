@@ -541,3 +541,28 @@ def test_rehash_long_chains_without_hints(bb):
     st = g.stats()
     assert first_chain > 20 and st["max_chain"] <= 8, (first_chain, st["max_chain"])
     assert st["live_pairs"] == o.num_edges() and st["tombstones"] < 50_000
+
+
+@pytest.mark.parametrize("set_variant", [False, True])
+@pytest.mark.parametrize("hints", [False, True])
+def test_hub_rows_export_stats_tc(hints, set_variant):
+    """Hub rows (more than 32 base buckets / 1,024 neighbours) are exported, counted
+    and oriented by the block-per-row kernels: a wheel W_n (hub 0 joined to the cycle
+    1..n) has exactly n triangles for n >= 4 and 4n directed entries."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    n = 6000
+    rim = np.arange(1, n + 1, dtype=np.uint32)
+    s = np.concatenate([np.zeros(n, np.uint32), rim])
+    d = np.concatenate([rim, np.roll(rim, -1)])
+    nv = n + 1
+    h = wl.out_degrees(np.concatenate([s, d]), nv) if hints else None
+    g = Graph(nv, h, directed=False, set_variant=set_variant)
+    o = Oracle(nv, directed=False)
+    g.insert_edges(cuda(s), cuda(d))
+    o.insert_edges(s, d)
+    check_against_oracle(g, o, "wheel")
+    st = g.stats()
+    assert st["live_pairs"] == 4 * n
+    assert g.triangle_count() == n == o.triangle_count()
+    assert sum(g.triangle_count(p, 2) for p in range(2)) == n
+    g.close()
