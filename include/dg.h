@@ -25,9 +25,14 @@
  *    (stream-ordered: the call enqueues work on `stream` and returns; the
  *    caller keeps the memory alive until that work completes) or HOST memory
  *    (pageable or pinned: the call stages it through library-owned device
- *    buffers and returns after every host output has been written, i.e. it is
- *    synchronous).  The caller owns all batch and result buffers; the library
- *    owns all table memory.
+ *    buffers and returns after every host output has been written and every
+ *    host input has been copied, so host buffers may be reused on return).  A
+ *    single-GPU dg_insert_edges / dg_delete_edges with host inputs and no count
+ *    requested returns once its batch is uploaded and validated (the status is
+ *    the call's return value) and leaves the mutation kernel running on
+ *    `stream`, where later calls are ordered behind it; the upload of the next
+ *    call overlaps it.  The caller owns all batch and result buffers; the
+ *    library owns all table memory.
  *  - `stream` is a cudaStream_t (NULL = legacy default stream).
  *  - Phase-concurrent model: calls on one handle must be
  *    serialised by the caller (one host thread, one stream at a time); a batch

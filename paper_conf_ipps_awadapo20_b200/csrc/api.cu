@@ -94,6 +94,56 @@ dg_status finish_out(dg_graph g, void* host, const void* dev, size_t bytes, cuda
   return DG_OK;
 }
 
+dg_status ensure_copy_streams(dg_graph g) {
+  for (auto& cs : g->cstream)
+    if (!cs) DG_CK(cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking));
+  return DG_OK;
+}
+
+// Asynchronous host input (insert / delete / query with host buffers): the bytes are
+// copied on the internal upload stream into staging slot `slot` (8..15) once the
+// kernels that read the slot's previous contents are done; `s` waits for the copy.
+// The call can then return as soon as the copy has landed, while its kernels run
+// behind the next call's upload (PCIe and HBM overlap across calls).
+dg_status upload_async(dg_graph g, int slot, const void* p, size_t bytes, cudaStream_t s,
+                       const void** out) {
+  if (!p || bytes == 0) {
+    *out = p;
+    return DG_OK;
+  }
+  DG_TRY(ensure_copy_streams(g));
+  if (!g->slot_ev[slot]) DG_CK(cudaEventCreateWithFlags(&g->slot_ev[slot], cudaEventDisableTiming));
+  DG_CK(ensure_buf(g->stage[slot], bytes));
+  cudaStream_t up = g->cstream[0];
+  DG_CK(cudaStreamWaitEvent(up, g->slot_ev[slot], 0));
+  DG_CK(cudaMemcpyAsync(g->stage[slot].p, p, bytes, cudaMemcpyHostToDevice, up));
+  DG_CK(cudaEventRecord(g->slot_ev[slot], up));
+  DG_CK(cudaStreamWaitEvent(s, g->slot_ev[slot], 0));
+  *out = g->stage[slot].p;
+  return DG_OK;
+}
+
+// after the kernels reading slots [a, b) were enqueued on s
+dg_status release_slots(dg_graph g, int a, int b, cudaStream_t s) {
+  for (int k = a; k < b; ++k)
+    if (g->slot_ev[k]) DG_CK(cudaEventRecord(g->slot_ev[k], s));
+  return DG_OK;
+}
+
+// snapshot the validation verdict (Q7) after k_validate on s, before the mutation
+dg_status note_validation(dg_graph g, cudaStream_t s) {
+  if (!g->val_event) DG_CK(cudaEventCreateWithFlags(&g->val_event, cudaEventDisableTiming));
+  if (!g->h_fail) DG_CK(cudaMallocHost(&g->h_fail, 64));
+  DG_CK(cudaMemcpyAsync(g->h_fail, &g->ctl->fail_epoch, 4, cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaEventRecord(g->val_event, s));
+  return DG_OK;
+}
+
+dg_status validation_status(dg_graph g, u32 epoch) {
+  DG_CK(cudaEventSynchronize(g->val_event));
+  return *g->h_fail >= epoch && *g->h_fail != 0 ? DG_ERR_VERTEX_OUT_OF_RANGE : DG_OK;
+}
+
 dg_status read_ctl(dg_graph g, cudaStream_t s) {
   DG_CK(cudaMemcpyAsync(g->hctl, g->ctl, sizeof(dg::DevCtl), cudaMemcpyDeviceToHost, s));
   DG_CK(cudaStreamSynchronize(s));
@@ -486,6 +536,10 @@ static void destroy_graph(dg_graph g) {
   if (g->hot_event) cudaEventDestroy(g->hot_event);
   for (auto& cs : g->cstream)
     if (cs) cudaStreamDestroy(cs);
+  for (cudaEvent_t e : g->slot_ev)
+    if (e) cudaEventDestroy(e);
+  if (g->val_event) cudaEventDestroy(g->val_event);
+  if (g->h_fail) cudaFreeHost(g->h_fail);
   for (cudaEvent_t e : g->pipe_ev) cudaEventDestroy(e);
   cudaGetLastError();
   delete g;
@@ -691,6 +745,20 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   const u32 epoch = ++g->epoch;
   bool host = false;
   const void *ds = nullptr, *dd = nullptr, *dw = nullptr;
+  if (!g->router && !n_added && n && !is_device_ptr(src) && !is_device_ptr(dst) &&
+      (!weight || !is_device_ptr(weight))) {
+    // host inputs, no count requested: return once the batch is uploaded and
+    // validated; the insert kernel runs behind the caller's next upload
+    DG_TRY(upload_async(g, 8, src, n * 4, s, &ds));
+    DG_TRY(upload_async(g, 9, dst, n * 4, s, &dd));
+    DG_TRY(upload_async(g, 10, weight, weight ? n * 4 : 0, s, &dw));
+    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    DG_TRY(note_validation(g, s));
+    DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
+                            epoch, s));
+    DG_TRY(release_slots(g, 8, 11, s));
+    return validation_status(g, epoch);
+  }
   DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
   DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
   DG_TRY(stage_in(g, 2, weight, weight ? n * 4 : 0, s, &dw, &host));
@@ -723,6 +791,16 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
   const u32 epoch = ++g->epoch;
   bool host = false;
   const void *ds = nullptr, *dd = nullptr;
+  if (!g->router && !n_removed && n && !is_device_ptr(src) && !is_device_ptr(dst)) {
+    // host inputs, no count requested: as in dg_insert_edges
+    DG_TRY(upload_async(g, 11, src, n * 4, s, &ds));
+    DG_TRY(upload_async(g, 12, dst, n * 4, s, &dd));
+    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    DG_TRY(note_validation(g, s));
+    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s));
+    DG_TRY(release_slots(g, 11, 13, s));
+    return validation_status(g, epoch);
+  }
   DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
   DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
   if (g->router) {
@@ -751,24 +829,23 @@ static dg_status query_host_pipelined(dg_graph g, const u32* src, const u32* dst
                                       uint8_t* found, u32* wout, u32 epoch, cudaStream_t s) {
   constexpr u64 kChunk = 1ull << 22;
   const u64 nch = (n + kChunk - 1) / kChunk;
-  DG_CK(ensure_buf(g->stage[0], n * 4));
-  DG_CK(ensure_buf(g->stage[1], n * 4));
+  DG_CK(ensure_buf(g->stage[13], n * 4));
+  DG_CK(ensure_buf(g->stage[14], n * 4));
   DG_CK(ensure_buf(g->stage[3], n));
   if (wout) DG_CK(ensure_buf(g->stage[4], n * 4));
-  for (auto& cs : g->cstream)
-    if (!cs) DG_CK(cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking));
+  DG_TRY(ensure_copy_streams(g));
   while (g->pipe_ev.size() < 2 * nch + 1) {
     cudaEvent_t e;
     DG_CK(cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
     g->pipe_ev.push_back(e);
   }
-  u32* ds = reinterpret_cast<u32*>(g->stage[0].p);
-  u32* dd = reinterpret_cast<u32*>(g->stage[1].p);
+  u32* ds = reinterpret_cast<u32*>(g->stage[13].p);
+  u32* dd = reinterpret_cast<u32*>(g->stage[14].p);
   uint8_t* df = reinterpret_cast<uint8_t*>(g->stage[3].p);
   u32* dw = wout ? reinterpret_cast<u32*>(g->stage[4].p) : nullptr;
   cudaStream_t up = g->cstream[0], down = g->cstream[1];
-  DG_CK(cudaEventRecord(g->pipe_ev[0], s));  // after earlier work on the caller's stream
-  DG_CK(cudaStreamWaitEvent(up, g->pipe_ev[0], 0));
+  // slots 13/14 belong to this pipeline alone (it completes before returning), so the
+  // uploads need not wait for earlier kernels on s: they overlap them
   for (u64 k = 0; k < nch; ++k) {
     const u64 off = k * kChunk, cnt = std::min(kChunk, n - off);
     DG_CK(cudaMemcpyAsync(ds + off, src + off, cnt * 4, cudaMemcpyHostToDevice, up));

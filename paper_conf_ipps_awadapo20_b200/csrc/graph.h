@@ -59,7 +59,12 @@ struct dg_graph_s {
   struct Buf {
     void* p = nullptr;
     size_t bytes = 0;
-  } stage[8];
+  } stage[16];
+  // asynchronous host inputs (slots 8..15): event recorded after the last kernel
+  // that read each slot; the next upload into the slot waits for it
+  cudaEvent_t slot_ev[16] = {};
+  cudaEvent_t val_event = nullptr;  // batch validated (status readable)
+  uint32_t* h_fail = nullptr;       // pinned copy of ctl->fail_epoch
   Buf tc[6];  // triangle counting scratch (CSR, orientation)
   Buf rh[4];  // re-sizing scratch
   Buf big;    // hub-row list (export, stats, TC orientation)

@@ -566,3 +566,46 @@ def test_hub_rows_export_stats_tc(hints, set_variant):
     assert g.triangle_count() == n == o.triangle_count()
     assert sum(g.triangle_count(p, 2) for p in range(2)) == n
     g.close()
+
+
+def test_async_host_batches():
+    """Host-buffer inserts/deletes without a count return once the batch is uploaded
+    and validated; the kernels run behind the next call.  The caller may overwrite
+    its host arrays on return (reused here for every batch), later calls see every
+    earlier batch (stream order), and a rejected batch still reports its status."""
+    from paper_conf_ipps_awadapo20_b200 import DGError, DG_ERR_VERTEX_OUT_OF_RANGE, Graph
+    nv = 50_000
+    g = Graph(nv)
+    o = Oracle(nv)
+    n = 300_000
+    hs = torch.empty(n, dtype=torch.int32).pin_memory()
+    hd = torch.empty(n, dtype=torch.int32).pin_memory()
+    hw = torch.empty(n, dtype=torch.int32).pin_memory()
+    hf = torch.empty(n, dtype=torch.uint8).pin_memory()
+    hq = torch.empty(n, dtype=torch.int32).pin_memory()
+    for b in range(6):
+        s, d, w = wl.uniform_edges(41, b, n, nv)
+        hs.numpy().view(np.uint32)[:] = s
+        hd.numpy().view(np.uint32)[:] = d
+        hw.numpy().view(np.uint32)[:] = w
+        if b % 3 == 2:  # delete the previous batch's first half
+            g.delete_edges(hs[: n // 2], hd[: n // 2])
+            o.delete_edges(s[: n // 2], d[: n // 2])
+        else:
+            g.insert_edges(hs, hd, hw)
+            o.insert_edges(s, d, w)
+        hs.fill_(0)  # overwritten right away: the library must hold its own copy
+        hd.fill_(0)
+        qs, qd, _ = wl.uniform_edges(41, 100 + b, n, nv)
+        qs[: n // 2], qd[: n // 2] = s[: n // 2], d[: n // 2]
+        hq.numpy().view(np.uint32)[:] = qd
+        f, qw = g.query_edges(qs, hq, found_out=hf, weight_out=np.empty(n, np.uint32))
+        _, rf, rw = o.query_edges(qs, qd)
+        assert np.array_equal(hf.numpy(), rf), b
+    s, d, w = wl.uniform_edges(41, 99, 1000, nv)
+    s[7] = nv
+    with pytest.raises(DGError) as e:
+        g.insert_edges(s, d, w)
+    assert e.value.status == DG_ERR_VERTEX_OUT_OF_RANGE
+    check_against_oracle(g, o, "async host batches")
+    g.close()

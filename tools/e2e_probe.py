@@ -18,6 +18,6 @@ for rep in range(3):
     hq.copy_(dst, non_blocking=True); torch.cuda.synchronize(); t2 = time.perf_counter()
     g.insert_edges(hs, hd, hw); t3 = time.perf_counter()
     g.query_edges(hs, hd, found_out=hf, weight_out=hq); t4 = time.perf_counter()
-    g.delete_edges(hs, hd); t5 = time.perf_counter()
+    g.delete_edges(hs, hd); t5 = time.perf_counter(); torch.cuda.synchronize(); t6 = time.perf_counter()
     print(f"H2D 64MB {1e3*(t1-t0):.2f} ms ({64/(t1-t0)/1e3:.1f} GB/s)  D2H 64MB {1e3*(t2-t1):.2f} ms  "
-          f"insert {1e3*(t3-t2):.2f}  query {1e3*(t4-t3):.2f}  delete {1e3*(t5-t4):.2f} ms")
+          f"insert {1e3*(t3-t2):.2f}  query {1e3*(t4-t3):.2f}  delete {1e3*(t5-t4):.2f} ms  (+{1e3*(t6-t5):.2f} kernel tail)  step {1e3*(t6-t2):.2f} ms")
