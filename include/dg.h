@@ -129,6 +129,8 @@ typedef struct dg_stats {
   uint64_t pool_bytes;        /* bytes of table memory mapped (pool + directory + stack) */
   double load_factor;         /* live_pairs / ((base+overflow) * pairs per bucket) (Q14) */
   double utilization;         /* live_pairs * 8 B / (linked buckets * bucket_bytes) (Fig. 2c) */
+  uint64_t exchange;          /* batch routing: 0 = none (single GPU), 1 = NCCL all-to-all,
+                                 2 = fused partition + peer stores into NVLink-mapped windows */
 } dg_stats;
 
 /* Fills defaults: load_factor 0.7, bucket_bytes 128, directed 1, pool_bytes 0,

@@ -59,6 +59,7 @@ class dg_stats(ctypes.Structure):
         ("pool_bytes", ctypes.c_uint64),
         ("load_factor", ctypes.c_double),
         ("utilization", ctypes.c_double),
+        ("exchange", ctypes.c_uint64),
     ]
 
 

@@ -680,6 +680,10 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
     if (st == DG_OK) st = dg::router_create(g, id, &g->router);
     if (st != DG_OK) return fail(st);
   }
+  if (g->router) {  // peer receive windows for the fused exchange (collective)
+    dg_status st = dg::router_setup_fused(g, s);
+    if (st != DG_OK) return fail(st);
+  }
 
   // hints: indexed by global vertex id
   const void* hints = nullptr;
@@ -1071,6 +1075,7 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   DG_TRY(read_ctl(g, s));
   std::memset(out, 0, sizeof(*out));
   out->local_rows = g->rows;
+  out->exchange = !g->router ? 0 : dg::router_fused(g->router) ? 2 : 1;
   out->base_buckets = h.base_buckets;
   out->overflow_buckets = h.linked_buckets - h.base_buckets;
   out->free_buckets = g->hctl->stack_size;

@@ -16,6 +16,11 @@ struct Router;
 dg_status router_unique_id(void* out128);
 dg_status router_create(dg_graph g, const void* unique_id, Router** out);
 void router_destroy(Router* r);
+// collective, after g->router is set: map every peer's receive window (CUDA IPC over
+// NVLink) for the fused exchange; falls back to the NCCL exchange if any rank cannot
+// (or DG_ROUTER=nccl).  router_fused() tells which path is active.
+dg_status router_setup_fused(dg_graph g, cudaStream_t s);
+bool router_fused(const Router* r);
 
 // collective edge ops: each rank passes its slice; validation is agreed on by all
 dg_status router_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,

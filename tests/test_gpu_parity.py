@@ -390,14 +390,21 @@ print("OK", g.stats()["pool_buckets"])
 
 
 @pytest.mark.parametrize("directed", [True, False])
-def test_routed_single_gpu(directed):
-    """The multi-GPU batch router (partition -> NCCL exchange -> local probe ->
-    answers back in caller order) on a 1-rank communicator: results identical to
-    the oracle."""
+@pytest.mark.parametrize("exchange", ["fused", "nccl"])
+def test_routed_single_gpu(directed, exchange, monkeypatch):
+    """The multi-GPU batch router (partition -> exchange -> local probe -> answers
+    back in caller order) on a 1-rank communicator: results identical to the oracle,
+    through the fused partition + window stores (default) and the NCCL exchange.
+    One batch outgrows the initial receive window (collective window re-setup)."""
     from paper_conf_ipps_awadapo20_b200 import Graph, DGError, DG_ERR_VERTEX_OUT_OF_RANGE
+    if exchange == "nccl":
+        monkeypatch.setenv("DG_ROUTER", "nccl")
     nv = 30_000
     g = Graph(nv, directed=directed, force_router=True)
+    assert g.stats()["exchange"] == (2 if exchange == "fused" else 1)
     o = Oracle(nv, directed)
+    s, d, w = wl.uniform_edges(17, 1000, 1_300_000, nv)  # > the 2^20-op initial window
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
     for b in range(3):
         s, d, w = wl.uniform_edges(17, b, 200_003, nv)
         s[-500:], d[-500:] = s[:500], d[:500]
