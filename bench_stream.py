@@ -246,9 +246,11 @@ def run_tc(args, cfg):
     wedges = 0
     tri = []
     clock = None
+    # warm-up steps count triangles on the bulk-built graph only; the timed steps are
+    # the paper's dynamic iterations (insert 2^22, then TC)
     for step in range(args.warmup + args.steps):
         timed = step >= args.warmup
-        s1, d1 = wl.rmat_edges(seed, 1 + step, IB, scale, abc)
+        s1, d1 = wl.rmat_edges(seed, 1 + max(0, step - args.warmup), IB if timed else 0, scale, abc)
         S1, D1 = cu(s1), cu(d1)
         if timed and step == args.warmup:
             torch.cuda.synchronize()

@@ -222,6 +222,16 @@ DG_API dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream);
  * (synchronises): DG_ERR_VERTEX_OUT_OF_RANGE if any was rejected, else DG_OK. */
 DG_API dg_status dg_batch_status(dg_graph g, void* stream);
 
+/* Tombstone flush ("Tombstones can later be completely flushed out of
+ * the data structure, if required"): every table holding a tombstone is rebuilt
+ * compactly — its live pairs are re-inserted into a fresh base range sized by the
+ * initial-bucket rule for its current degree and all of its old
+ * buckets go to the free stack.  The logical graph is unchanged.  Rows are found
+ * by one streaming pass over the allocated buckets per round of up to 65,536 rows.
+ * *rows_rebuilt (host, nullable) receives the number of rebuilt tables.  Local to
+ * this rank (not collective); synchronises `stream`. */
+DG_API dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* stream);
+
 /* Triangle count of a symmetric graph (undirected mode, directed = 0) by per-vertex
  * hash intersection (§VI-C): orient every edge from lower to higher rank,
  * rank(x) = (degree, id); for every vertex u and every pair v, w of its

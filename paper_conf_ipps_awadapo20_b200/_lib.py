@@ -90,6 +90,7 @@ SIGNATURES = [
     ("dg_get_stats", ctypes.c_int, [VP, ctypes.POINTER(dg_stats), VP]),
     ("dg_batch_status", ctypes.c_int, [VP, VP]),
     ("dg_triangle_count", ctypes.c_int, [VP, U32, U32, P_U64, VP]),
+    ("dg_flush_tombstones", ctypes.c_int, [VP, P_U64, VP]),
     ("dg_profile_enable", ctypes.c_int, [VP, ctypes.c_int]),
     ("dg_profile_read", ctypes.c_int, [VP, ctypes.POINTER(dg_profile), VP]),
 ]

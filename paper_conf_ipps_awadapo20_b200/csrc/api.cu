@@ -393,7 +393,12 @@ dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t
 // for twice its degree, and insert the pairs again.  Runs before an insert batch
 // (phase-concurrent: no other batch in flight on the handle).
 dg_status rehash_hot(dg_graph g, cudaStream_t s) {
-  const u32 n = std::min<u32>(*g->h_hot, g->hot_cap);
+  return rehash_rows(g, std::min<u32>(*g->h_hot, g->hot_cap), false, s);
+}
+
+// Re-build the n rows of hot_list (flush = false: long chains, sized to double;
+// true: tombstone flush, sized by the initial rule for their live keys).
+dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
   if (n == 0) return DG_OK;
   g->in_rehash = true;
   struct Guard {
@@ -410,7 +415,7 @@ dg_status rehash_hot(dg_graph g, cudaStream_t s) {
   u64* doff = obo + m;
   u64* cursor = doff + m;
   dg::Tables t = g->tables();
-  DG_CK(dg::launch_hot_sizes(t, n, g->lf_milli, g->BC, nbnew, nbold, degs, s));
+  DG_CK(dg::launch_hot_sizes(t, n, g->lf_milli, g->BC, flush ? 1u : 0u, nbnew, nbold, degs, s));
   DG_CK(dg::scan_exclusive_u64(nbnew, nboff, m, &g->scan_temp, &g->scan_bytes, s));
   DG_CK(dg::scan_exclusive_u64(nbold, obo, m, &g->scan_temp, &g->scan_bytes, s));
   DG_CK(dg::scan_exclusive_u64(degs, doff, m, &g->scan_temp, &g->scan_bytes, s));
@@ -428,7 +433,7 @@ dg_status rehash_hot(dg_graph g, cudaStream_t s) {
   if (bump0 + total_new + 1 >= 0xFFFFFFFEull) {  // no room: forget the flags
     DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
     DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
-    return DG_OK;
+    return flush ? DG_ERR_OUT_OF_MEMORY : DG_OK;
   }
   DG_TRY(grow_pool(g, bump0 + total_new + g->cap / 8 + 65536, s));
   t = g->tables();
@@ -1101,6 +1106,30 @@ dg_status dg_batch_status(dg_graph g, void* stream) {
   if (g->hctl->fail_epoch > g->checked_epoch) st = DG_ERR_VERTEX_OUT_OF_RANGE;
   g->checked_epoch = g->epoch;
   return st;
+}
+
+dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* stream) {
+  DG_TRY(check_handle(g));
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  if (rows_rebuilt) *rows_rebuilt = 0;
+  if (g->hot_pending) DG_CK(cudaEventSynchronize(g->hot_event));
+  g->hot_pending = false;  // rows flagged by earlier inserts are rebuilt below too
+  u64 total = 0;
+  for (int pass = 0; pass < 100000; ++pass) {
+    dg::Tables t = g->tables();
+    t.hot_flags = g->hot_flags;
+    DG_CK(dg::launch_tomb_sweep(g->lay, t, g->sms, s));
+    if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+    g->snap_pending = false;
+    DG_TRY(read_ctl(g, s));
+    const u32 found = g->hctl->hot_count;
+    if (found == 0) break;
+    const u32 n = std::min<u32>(found, g->hot_cap);
+    DG_TRY(dg::rehash_rows(g, n, true, s));
+    total += n;
+  }
+  if (rows_rebuilt) *rows_rebuilt = total;
+  return DG_OK;
 }
 
 dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t* count,

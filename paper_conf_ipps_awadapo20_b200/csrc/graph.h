@@ -120,6 +120,7 @@ void prof_mark(dg_graph g, int k, cudaStream_t s);
 // internal entry points shared by api.cu and router.cu
 dg_status grow_pool(dg_graph g, uint64_t min_buckets, cudaStream_t s);
 dg_status rehash_hot(dg_graph g, cudaStream_t s);
+dg_status rehash_rows(dg_graph g, uint32_t n, bool flush, cudaStream_t s);
 dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
                        uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s);
 dg_status local_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,

@@ -96,8 +96,12 @@ cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u3
                              unsigned long long* count, int sms, cudaStream_t s);
 
 // per-vertex re-sizing of long-chained tables (kernels_rehash.cu)
-cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
-                             u64* degs, cudaStream_t s);
+// flush = 0: re-size for long chains (room to double); 1: tombstone flush (the
+// initial-size rule for the live keys)
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
+                             u64* nbold, u64* degs, cudaStream_t s);
+// rows holding a tombstone -> hot flags / hot list (tombstone flush)
+cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s);
 cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
                               unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
                               int sms, cudaStream_t s);

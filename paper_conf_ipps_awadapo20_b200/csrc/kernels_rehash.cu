@@ -17,8 +17,8 @@
 
 namespace dg {
 
-__global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
-                            u64* degs) {
+__global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
+                            u64* nbold, u64* degs) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k <= n; k += stride) {
     if (k == n) {
@@ -29,8 +29,13 @@ __global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u
     const DirEntry de = t.dir[row];
     const u64 d = t.deg[row];
     const u64 den = (u64)lf_milli * bc;
-    u64 want = (2 * d * 1000 + den - 1) / den;  // room to double before chaining again
-    if (want < (u64)de.nb + 1) want = (u64)de.nb + 1;
+    u64 want;
+    if (flush) {  // tombstone flush: the initial-size rule for the live keys
+      want = d ? (d * 1000 + den - 1) / den : 1;
+    } else {      // re-size: room to double before chaining again
+      want = (2 * d * 1000 + den - 1) / den;
+      if (want < (u64)de.nb + 1) want = (u64)de.nb + 1;
+    }
     nbnew[k] = want;
     nbold[k] = de.nb;
     degs[k] = d;
@@ -133,10 +138,50 @@ __global__ void k_hot_install(Tables t, u32 n, const u64* nbnew, const u64* nbof
   }
 }
 
-cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u64* nbnew, u64* nbold,
-                             u64* degs, cudaStream_t s) {
+// Tombstone flush ("Tombstones can later be completely flushed out of
+// the data structure"): one streaming pass over every allocated bucket; a bucket
+// holding a tombstone flags its owner row (bucket word W-1) for a compacting
+// re-build (the rows are then re-sized with flush = 1).
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_tomb_sweep(Tables t) {
+  typedef Lay<G, S> LY;
+  const Group<G> g;
+  const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
+  const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
+  const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
+  for (u64 b = gid; b < nbk; b += ng) {
+    const uint4 x = *reinterpret_cast<const uint4*>(t.pool + b * LY::W + 4 * g.gl);
+    bool tomb = false;
+#pragma unroll
+    for (int j = 0; j < LY::SPU; ++j) tomb |= LY::has(g.gl, j) && LY::key(x, j) == kTomb;
+    const u32 owner = g.shfl(x.w, G - 1);
+    if (g.ballot(tomb) && g.gl == 0) {
+      const u32 bit = 1u << (owner & 31);
+      if (!(atomicOr(&t.hot_flags[owner >> 5], bit) & bit)) {
+        const u32 k = atomicAdd(&t.ctl->hot_count, 1u);
+        if (k < t.hot_cap) t.hot_list[k] = owner;
+      }
+    }
+  }
+}
+
+cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s) {
+  const unsigned blocks = (unsigned)sms * 8;
+  switch (lay) {
+#define DG_CASE(G_, S_) \
+  case DG_LAY(G_, S_): k_tomb_sweep<G_, S_><<<blocks, 256, 0, s>>>(t); break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
+    default: return cudaErrorInvalidValue;
+  }
+  note_kernel(1);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
+                             u64* nbold, u64* degs, cudaStream_t s) {
   const unsigned blocks = (n + 256) / 256;
-  k_hot_sizes<<<blocks, 256, 0, s>>>(t, n, lf_milli, bc, nbnew, nbold, degs);
+  k_hot_sizes<<<blocks, 256, 0, s>>>(t, n, lf_milli, bc, flush, nbnew, nbold, degs);
   note_kernel(1);
   return cudaGetLastError();
 }

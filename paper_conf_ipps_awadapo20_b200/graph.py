@@ -266,6 +266,14 @@ class Graph:
                 "kernel_launches": dict(zip(self.PROFILE_KINDS, list(p.kernel_launches))),
                 "kernel_ms": dict(zip(self.PROFILE_KINDS, list(p.kernel_ms)))}
 
+    def flush_tombstones(self, stream=None) -> int:
+        """Rebuild every table holding tombstones compactly; returns the
+        number of tables rebuilt.  The logical graph is unchanged."""
+        n = ctypes.c_uint64(0)
+        check(lib.dg_flush_tombstones(self._h, ctypes.byref(n), _stream(stream)),
+              "dg_flush_tombstones")
+        return n.value
+
     def triangle_count(self, part: int = 0, nparts: int = 1, stream=None) -> int:
         """Triangles by hash intersection (§VI-C); part/nparts split the work by u mod nparts."""
         c = ctypes.c_uint64()

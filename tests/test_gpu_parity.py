@@ -616,3 +616,36 @@ def test_async_host_batches():
     assert e.value.status == DG_ERR_VERTEX_OUT_OF_RANGE
     check_against_oracle(g, o, "async host batches")
     g.close()
+
+
+@pytest.mark.parametrize("set_variant", [False, True])
+@pytest.mark.parametrize("reuse", [False, True])
+def test_flush_tombstones(reuse, set_variant):
+    """Tombstone flush: after insert/delete churn the
+    tables hold tombstones; flushing rebuilds every such table compactly (several
+    rounds: > 65,536 rows carry tombstones), the logical graph is unchanged, no
+    tombstone is left and the freed buckets serve later inserts."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 200_000
+    g = Graph(nv, reuse_tombstones=reuse, set_variant=set_variant, bucket_bytes=64)
+    o = Oracle(nv)
+
+    def ow(w):
+        return np.zeros_like(w) if set_variant else w
+    for b in range(4):
+        s, d, w = wl.uniform_edges(61, b, 600_000, nv)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, ow(w))[1]
+        assert g.delete_edges(cuda(s[::2]), cuda(d[::2]), count=True) == o.delete_edges(s[::2], d[::2])[1]
+    before = g.stats()
+    assert before["tombstones"] > 100_000
+    rebuilt = g.flush_tombstones()
+    assert rebuilt > 65_536
+    after = g.stats()
+    assert after["tombstones"] == 0 and after["live_pairs"] == o.num_edges()
+    assert after["overflow_buckets"] < before["overflow_buckets"]
+    check_against_oracle(g, o, "after flush")
+    assert g.flush_tombstones() == 0
+    s, d, w = wl.uniform_edges(61, 99, 300_000, nv)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, ow(w))[1]
+    check_against_oracle(g, o, "inserts after flush")
+    g.close()
