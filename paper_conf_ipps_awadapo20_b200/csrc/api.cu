@@ -155,8 +155,9 @@ dg_status status_of(dg_graph g, u32 epoch) {
                                                                    : DG_OK;
 }
 
+// the |V|-bit deleted-vertex bitmap followed by its coarse filter (kVdelFilterBits)
 dg_status ensure_bitmap(dg_graph g, u64 nv) {
-  const u64 words = (nv + 31) / 32 + 1;
+  const u64 words = (nv + 31) / 32 + 1 + dg::kVdelFilterBits / 32;
   if (words > g->bitmap_words) {
     if (g->bitmap) cudaFree(g->bitmap);
     g->bitmap = nullptr;
@@ -986,11 +987,15 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
   if (all_n == 0) return DG_OK;
   DG_TRY(ensure_bitmap(g, g->nv));
   DG_TRY(ensure_dedup(g, all_n));
-  DG_CK(cudaMemsetAsync(g->bitmap, 0, ((g->nv + 31) / 32 + 1) * 4, s));
+  const u64 bwords = (g->nv + 31) / 32 + 1;
+  u32* filter = g->bitmap + bwords;
+  u32 fshift = 0;
+  while (((g->nv - 1) >> fshift) >= dg::kVdelFilterBits) ++fshift;
+  DG_CK(cudaMemsetAsync(g->bitmap, 0, (bwords + dg::kVdelFilterBits / 32) * 4, s));
   DG_CK(cudaMemsetAsync(&g->ctl->queue, 0, 2 * sizeof(u32), s));  // queue, dedup_count
   const dg::Tables t = g->tables();
-  DG_CK(dg::launch_vdel_mark(all_ids, all_n, g->nv, epoch, g->bitmap, g->dedup, g->ctl, g->nranks,
-                             g->rank, g->sms, s));
+  DG_CK(dg::launch_vdel_mark(all_ids, all_n, g->nv, epoch, g->bitmap, filter, fshift, g->dedup,
+                             g->ctl, g->nranks, g->rank, g->sms, s));
   static const bool force_sweep = std::getenv("DG_FORCE_SWEEP") != nullptr;
   // base-bucket offsets of the distinct deleted vertices (flattened purge work)
   DG_CK(ensure_buf(g->stage[7], (all_n + 1) * 8 * 2));
@@ -1004,7 +1009,7 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
     DG_CK(dg::launch_vdel_neighbors(g->lay, t, g->dedup, boff, epoch, g->sms, s));
   } else {
     // directed: follow-up sweep over all tables
-    DG_CK(dg::launch_vdel_sweep(g->lay, t, g->bitmap, epoch, g->sms, s));
+    DG_CK(dg::launch_vdel_sweep(g->lay, t, g->bitmap, filter, fshift, epoch, g->sms, s));
   }
   DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, boff, epoch, g->sms, s));
   dg::prof_mark(g, dg::PROF_VDEL, s);

@@ -74,10 +74,14 @@ struct StatsOut {
 cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s);
 
 // vertex deletion (kernels_graph.cu)
-cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
-                             DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s);
-cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, u32 epoch, int sms,
-                              cudaStream_t s);
+// coarse filter of the deleted-vertex bitmap (bit = id >> fshift), kept in shared
+// memory by the purge sweep
+constexpr u32 kVdelFilterBits = 1u << 17;
+cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* filter,
+                             u32 fshift, u32* dedup, DevCtl* ctl, u32 nranks, u32 rank, int sms,
+                             cudaStream_t s);
+cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const u32* filter,
+                              u32 fshift, u32 epoch, int sms, cudaStream_t s);
 // nbarr[k] = base buckets of the k-th distinct deleted vertex (0 past the count), k <= n_max
 cudaError_t launch_vdel_nb(const Tables& t, const u32* dedup, u64 n_max, u64* nbarr, int sms,
                            cudaStream_t s);

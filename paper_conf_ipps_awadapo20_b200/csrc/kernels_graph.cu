@@ -368,8 +368,11 @@ cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int 
 // Mark the batch in a |V|-bit bitmap D (all ranks mark every deleted ID, since
 // incoming edges may live on any shard), validate it (Q7/Q11), and list each
 // distinct ID owned by this rank once (duplicates are idempotent).
-__global__ void k_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
-                            DevCtl* ctl, u32 nranks, u32 rank) {
+// The coarse filter (kVdelFilterBits bits, bit = id >> fshift) is the bitmap at a
+// coarser grain: the purge sweep keeps it in shared memory and reads the fine bitmap
+// only for keys whose coarse bit is set.
+__global__ void k_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* filter,
+                            u32 fshift, u32* dedup, DevCtl* ctl, u32 nranks, u32 rank) {
   bool bad = false;
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
@@ -380,17 +383,23 @@ __global__ void k_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitma
     }
     const u32 bit = 1u << (id & 31);
     const u32 old = atomicOr(&bitmap[id >> 5], bit);
-    if (!(old & bit) && id % nranks == rank) dedup[atomicAdd(&ctl->dedup_count, 1u)] = id;
+    if (!(old & bit)) {
+      const u32 c = id >> fshift;
+      atomicOr(&filter[c >> 5], 1u << (c & 31));
+      if (id % nranks == rank) dedup[atomicAdd(&ctl->dedup_count, 1u)] = id;
+    }
   }
   if (__any_sync(0xFFFFFFFFu, bad) && (threadIdx.x & 31) == 0) atomicMax(&ctl->fail_epoch, epoch);
 }
 
-cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* dedup,
-                             DevCtl* ctl, u32 nranks, u32 rank, int sms, cudaStream_t s) {
+cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitmap, u32* filter,
+                             u32 fshift, u32* dedup, DevCtl* ctl, u32 nranks, u32 rank, int sms,
+                             cudaStream_t s) {
   if (n == 0) return cudaSuccess;
   u64 blocks = (n + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
-  k_vdel_mark<<<(unsigned)blocks, 256, 0, s>>>(ids, n, nv, epoch, bitmap, dedup, ctl, nranks, rank); note_kernel(1);
+  k_vdel_mark<<<(unsigned)blocks, 256, 0, s>>>(ids, n, nv, epoch, bitmap, filter, fshift, dedup,
+                                               ctl, nranks, rank); note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -400,12 +409,16 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // tombstone and the owner row's degree drops by one.
 template <int G, int S>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
+                                                    const u32* __restrict__ filter, u32 fshift,
                                                     u32 epoch) {
   typedef Lay<G, S> LY;
   constexpr int W = LY::W;
   constexpr int U = 4;  // buckets in flight per group (memory-level parallelism)
+  __shared__ u32 sf[kVdelFilterBits / 32];
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
+  for (u32 i = threadIdx.x; i < kVdelFilterBits / 32; i += blockDim.x) sf[i] = filter[i];
+  __syncthreads();
   const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
@@ -427,7 +440,9 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 #pragma unroll
       for (int j = 0; j < LY::SPU; ++j) {
         const u32 kk = LY::key(x, j);
-        if (LY::has(g.gl, j) && kk < kTomb && ((__ldg(bitmap + (kk >> 5)) >> (kk & 31)) & 1u) &&
+        if (!LY::has(g.gl, j) || kk >= kTomb) continue;
+        const u32 c = kk >> fshift;
+        if (((sf[c >> 5] >> (c & 31)) & 1u) && ((__ldg(bitmap + (kk >> 5)) >> (kk & 31)) & 1u) &&
             atomicCAS(bp + LY::word(g.gl, j), kk, kTomb) == kk)
           ++dec;
       }
@@ -436,12 +451,14 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
   }
 }
 
-cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, u32 epoch, int sms,
-                              cudaStream_t s) {
+cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const u32* filter,
+                              u32 fshift, u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (lay) {
-#define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, epoch); break;
+#define DG_CASE(G_, S_)                                                                  \
+  case DG_LAY(G_, S_):                                                                   \
+    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch); \
+    break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
