@@ -45,6 +45,7 @@ struct DevCtl {
   u64 count;         // n_added / n_removed / TC accumulator of the current batch
   u32 hot_count;     // rows flagged for re-sizing (long chains), see k_edges / rehash
   u32 hot_pairs;     // sum of their degrees when flagged (saturating): work to re-size
+  u32 route_timeout; // a fused-exchange wait gave up on a peer (router.cu)
 };
 
 struct Tables {

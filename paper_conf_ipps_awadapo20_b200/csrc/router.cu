@@ -242,9 +242,29 @@ __global__ void k_route_scatter_fused(const u32* src, const u32* dst, const u32*
   signal_peers(done, tb->arrive, P);
 }
 
-__global__ void k_route_wait(const unsigned long long* ctr, unsigned long long expected) {
-  if (threadIdx.x == 0)
-    while (ld_acquire_sys(ctr) < expected) __nanosleep(64);
+// Spins until every rank has signalled.  A peer that never arrives (a rank that
+// died or skipped the collective) must not hang the device: after kWaitTimeoutNs the
+// kernel raises ctl->route_timeout and returns; the host turns it into DG_ERR_NCCL at
+// the next batch and the handle goes bad.
+constexpr unsigned long long kWaitTimeoutNs = 30ull * 1000 * 1000 * 1000;
+
+__device__ __forceinline__ unsigned long long globaltimer_ns() {
+  unsigned long long t;
+  asm volatile("mov.u64 %0, %globaltimer;" : "=l"(t));
+  return t;
+}
+
+__global__ void k_route_wait(const unsigned long long* ctr, unsigned long long expected,
+                             DevCtl* ctl) {
+  if (threadIdx.x != 0) return;
+  const unsigned long long t0 = globaltimer_ns();
+  while (ld_acquire_sys(ctr) < expected) {
+    __nanosleep(64);
+    if (globaltimer_ns() - t0 > kWaitTimeoutNs) {
+      atomicExch(&ctl->route_timeout, 1u);
+      return;
+    }
+  }
 }
 
 // query answers back to the askers' answer windows (a11), in send order
@@ -357,7 +377,12 @@ dg_status route_partition(dg_graph g, const u32* src, const u32* dst, const u32*
   RT_CK(cudaGetLastError());
   RT_NC(N.AllGather(meta_mine, r.meta_all.p, P + 1, ncclUint64, r.comm, s));
   RT_CK(cudaMemcpyAsync(r.h_meta, r.meta_all.p, (size_t)P * (P + 1) * 8, cudaMemcpyDeviceToHost, s));
+  RT_CK(cudaMemcpyAsync(r.h_scalar + 1, &g->ctl->route_timeout, 4, cudaMemcpyDeviceToHost, s));
   RT_CK(cudaStreamSynchronize(s));
+  if (reinterpret_cast<const u32*>(r.h_scalar + 1)[0]) {  // a peer never arrived (k_route_wait)
+    g->bad = true;
+    return DG_ERR_NCCL;
+  }
   bool bad = false;
   r.scnt.assign(P, 0);
   r.rcnt.assign(P, 0);
@@ -532,7 +557,7 @@ dg_status route_fused_scatter(dg_graph g, const u32* src, const u32* dst, const 
       src, dst, w, n, n_ops, P, as<u64>(r.offs), as<RouteTable>(r.table), with_w,
       keep_pos ? as<u64>(r.pos) : nullptr, &mine.hdr->done);
   r.arrive_expected += P;
-  k_route_wait<<<1, 32, 0, s>>>(&mine.hdr->arrive, r.arrive_expected);
+  k_route_wait<<<1, 32, 0, s>>>(&mine.hdr->arrive, r.arrive_expected, g->ctl);
   note_kernel(2);
   RT_CK(cudaGetLastError());
   return DG_OK;
@@ -680,7 +705,7 @@ dg_status router_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_
     k_route_return<<<(unsigned)g->sms * 4, 256, 0, s>>>(as<uint8_t>(r.rfound), as<u32>(r.rwt), r.P,
                                                         as<RouteTable>(r.table), &x.hdr->done_ret);
     r.ans_expected += r.P;
-    k_route_wait<<<1, 32, 0, s>>>(&x.hdr->ans_arrive, r.ans_expected);
+    k_route_wait<<<1, 32, 0, s>>>(&x.hdr->ans_arrive, r.ans_expected, g->ctl);
     note_kernel(2);
     if (n) {
       u64 blocks = std::min<u64>((n + 255) / 256, (u64)g->sms * 8);
