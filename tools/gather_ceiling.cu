@@ -2,7 +2,11 @@
 // random S-byte reads (S = 32/64/128, one S-byte block per group of S/16 lanes
 // with 16-B lane loads) over a buffer >= 4x L2, enough loads in flight to
 // saturate.  This is the achievable bandwidth for hash probes, reported beside the
-// STREAM-copy peak of MEASURED_PEAKS.json.  Build/run:
+// STREAM-copy peak of MEASURED_PEAKS.json.  The read-modify-write modes add, per
+// gathered block, what an insert / delete adds per op: an 8-B store into the block
+// (M = 1: dirties one sector that is written back) or a 64-bit CAS on it (M = 2),
+// plus a fire-and-forget atomic on an L2-resident counter array (M = 3, the degree
+// update) — the achievable op rate for the mutating probe kernels.  Build/run:
 //   nvcc -gencode arch=compute_100a,code=sm_100a -O3 -o /tmp/gc tools/gather_ceiling.cu && /tmp/gc
 #include <cstdio>
 #include <cstdint>
@@ -13,9 +17,9 @@ __device__ __forceinline__ uint64_t mix(uint64_t x) {
   return x ^ (x >> 33);
 }
 
-template <int G, int U>
-__global__ void gather(const uint4* __restrict__ buf, uint64_t nblocks, uint64_t iters,
-                       unsigned long long* sink) {
+template <int G, int U, int M>
+__global__ void gather(uint4* __restrict__ buf, uint64_t nblocks, uint64_t iters,
+                       unsigned long long* sink, uint32_t* cnt, uint32_t ncnt) {
   const uint32_t lane = threadIdx.x & 31, gl = lane & (G - 1);
   const uint64_t gid = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) / G;
   uint32_t acc = 0;
@@ -24,34 +28,52 @@ __global__ void gather(const uint4* __restrict__ buf, uint64_t nblocks, uint64_t
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const uint64_t b = ((mix(gid * 1315423911ULL + it * U + k) & 0xFFFFFFFFull) * nblocks) >> 32;
-      q[k] = __ldg(buf + b * G + gl);
+      q[k] = M == 0 ? __ldg(buf + b * G + gl) : buf[b * G + gl];
     }
 #pragma unroll
     for (int k = 0; k < U; ++k) acc += q[k].x ^ q[k].w;
+    if (M > 0) {
+      // the lane that owns op k (k-th lane of the group) mutates its block
+#pragma unroll
+      for (int k = 0; k < U; ++k) {
+        if (gl != (uint32_t)(k % G)) continue;
+        const uint64_t h = mix(gid * 1315423911ULL + it * U + k);
+        const uint64_t b = ((h & 0xFFFFFFFFull) * nblocks) >> 32;
+        unsigned long long* p = reinterpret_cast<unsigned long long*>(buf + b * G) + ((h >> 40) & (2 * G - 1));
+        if (M == 1) {
+          *p = (unsigned long long)(acc + k);
+        } else {
+          acc += (uint32_t)atomicCAS(p, (unsigned long long)q[k].x, (unsigned long long)(acc + k));
+          if (M == 3) atomicAdd(cnt + ((h >> 8) % ncnt), 1u);
+        }
+      }
+    }
   }
   if (acc == 0x12345678u) atomicAdd(sink, 1ull);
 }
 
-template <int G, int U>
-double run(const uint4* buf, uint64_t bytes, int sms) {
+template <int G, int U, int M = 0>
+double run(uint4* buf, uint64_t bytes, int sms, uint32_t* cnt = nullptr, uint32_t ncnt = 1,
+           double* gops = nullptr, int bps = 8) {
   const uint64_t nblocks = bytes / (16 * G);
-  const int blocks = sms * 8, threads = 256;
+  const int blocks = sms * bps, threads = 256;
   const uint64_t groups = (uint64_t)blocks * threads / G;
   const uint64_t iters = 64;
   unsigned long long* sink;
   cudaMalloc(&sink, 8);
-  gather<G, U><<<blocks, threads>>>(buf, nblocks, 4, sink);
+  gather<G, U, M><<<blocks, threads>>>(buf, nblocks, 4, sink, cnt, ncnt);
   cudaEvent_t a, b;
   cudaEventCreate(&a);
   cudaEventCreate(&b);
   cudaEventRecord(a);
-  gather<G, U><<<blocks, threads>>>(buf, nblocks, iters, sink);
+  gather<G, U, M><<<blocks, threads>>>(buf, nblocks, iters, sink, cnt, ncnt);
   cudaEventRecord(b);
   cudaEventSynchronize(b);
   float ms = 0;
   cudaEventElapsedTime(&ms, a, b);
   cudaFree(sink);
   const double moved = (double)groups * iters * U * 16 * G;
+  if (gops) *gops = (double)groups * iters * U / (ms * 1e-3) / 1e9;
   return moved / (ms * 1e-3) / 1e9;
 }
 
@@ -69,7 +91,28 @@ int main() {
   printf("\"S64_U4\": %.1f, ", run<4, 4>(buf, bytes, p.multiProcessorCount));
   printf("\"S128_U2\": %.1f, ", run<8, 2>(buf, bytes, p.multiProcessorCount));
   printf("\"S128_U4\": %.1f, ", run<8, 4>(buf, bytes, p.multiProcessorCount));
-  printf("\"S128_U8\": %.1f}}\n", run<8, 8>(buf, bytes, p.multiProcessorCount));
+  printf("\"S128_U8\": %.1f}, ", run<8, 8>(buf, bytes, p.multiProcessorCount));
+  // read-modify-write modes (128-B blocks): G ops/s
+  uint32_t* cnt;
+  const uint32_t ncnt = 4847571;  // one counter per cfg2 row (19 MB, L2-resident)
+  cudaMalloc(&cnt, 4ull * ncnt);
+  cudaMemset(cnt, 0, 4ull * ncnt);
+  // best over in-flight depth U and resident blocks per SM
+  const int sm = p.multiProcessorCount;
+  double best[4] = {0, 0, 0, 0};
+  for (int bps : {4, 8, 16}) {
+    double g;
+#define DG_TRY(U_)                                                       \
+    run<8, U_, 0>(buf, bytes, sm, cnt, ncnt, &g, bps); best[0] = g > best[0] ? g : best[0]; \
+    run<8, U_, 1>(buf, bytes, sm, cnt, ncnt, &g, bps); best[1] = g > best[1] ? g : best[1]; \
+    run<8, U_, 2>(buf, bytes, sm, cnt, ncnt, &g, bps); best[2] = g > best[2] ? g : best[2]; \
+    run<8, U_, 3>(buf, bytes, sm, cnt, ncnt, &g, bps); best[3] = g > best[3] ? g : best[3];
+    DG_TRY(2) DG_TRY(4) DG_TRY(8)
+#undef DG_TRY
+  }
+  printf("\"G_ops_s_S128\": {\"read\": %.2f, \"read_store8\": %.2f, \"read_cas8\": %.2f, "
+         "\"read_cas8_counter\": %.2f}}\n", best[0], best[1], best[2], best[3]);
+  cudaFree(cnt);
   cudaFree(buf);
   return 0;
 }
