@@ -169,7 +169,7 @@ def run_mixed(args, cfg):
     peak, peak_src = load_peaks()
     # dominant kernel: the streaming purge sweep reads every allocated bucket once
     st_ = g.stats()
-    sweep_bytes = st_["bump_buckets"] * S
+    sweep_bytes = st_["bump_bytes"]
     vms = prof["kernel_ms"]["vertex_purge"]
     vl = max(1, prof["kernel_launches"]["vertex_purge"])
     kms = prof["kernel_ms"]
@@ -182,7 +182,7 @@ def run_mixed(args, cfg):
         roofline["algorithmic_bytes_per_launch"] = sweep_bytes
         roofline["note"] = "purge sweep + clear: model bytes = allocated buckets x bucket bytes"
     else:
-        mb = model_bytes(S)
+        mb = model_bytes(S or st_["table_bytes"] / max(1, st_["base_buckets"] + st_["overflow_buckets"]))
         per = {"insert": mb["insert_new"], "query": mb["query"], "delete": mb["delete_hit"]}
         nb = cnt_[dom] / world * per.get(dom, mb["query"])
         roofline["achieved"] = nb / (kms[dom] * 1e-3) / 1e9
@@ -289,8 +289,12 @@ def run_tc(args, cfg):
     total_ms = t_ins + t_tc
     value = edge_ops / (total_ms * 1e3)
     peak, peak_src = load_peaks()
-    bytes_per_probe = S + 4  # one bucket of A_v + the streamed candidate id
-    roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16},{variant}>", "unit": "GB/s",
+    # one bucket of A_v + the streamed candidate id; adaptive layout: the
+    # mean bytes of a linked bucket
+    Sb = S or st_["table_bytes"] / max(1, st_["base_buckets"] + st_["overflow_buckets"])
+    bytes_per_probe = Sb + 4
+    roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16 if S else 'adaptive'},{variant}>",
+                "unit": "GB/s",
                 "achieved": wedge_ops / world * bytes_per_probe / (wk / nl * 1e-3) / 1e9,
                 "peak": peak, "peak_source": peak_src, "traffic": None,
                 "algorithmic_bytes_per_launch": wedge_ops / world * bytes_per_probe,

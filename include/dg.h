@@ -114,6 +114,17 @@ typedef struct dg_config {
  * `weight`, dg_query_edges reports weight 0 for every hit, dg_export_adjacency
  * writes weight 0.  Membership results are those of the map variant. */
 #define DG_FLAG_SET 4u
+/* Degree-adaptive bucket sizes (the paper's future work,
+ * "hash tables with varying slab sizes may better suit load balancing in
+ * scale-free graphs").  Each vertex's table uses one of three bucket sizes, chosen
+ * from its degree hint: the smallest bucket that holds the hint at the load factor
+ * (32 B = 3 pairs for hints <= lf*3, 64 B = 7 pairs for hints <= lf*7), else 128-B
+ * buckets (15 pairs) sized by the usual rule.  A vertex without a hint starts with
+ * one 32-B bucket; the per-vertex re-sizing (long chains) picks the size class again
+ * for twice the degree, so growing vertices move up to larger buckets.  Each size
+ * class has its own bucket pool and free stack.  `bucket_bytes` is ignored.  Results
+ * are those of every other layout. */
+#define DG_FLAG_ADAPTIVE 8u
 
 /* Memory / structure statistics (Fig. 2b/c quantities). */
 typedef struct dg_stats {
@@ -127,10 +138,14 @@ typedef struct dg_stats {
   uint64_t tombstones;        /* deleted-key slots not yet reclaimed */
   uint64_t max_chain;         /* longest bucket chain (in buckets) */
   uint64_t pool_bytes;        /* bytes of table memory mapped (pool + directory + stack) */
-  double load_factor;         /* live_pairs / ((base+overflow) * pairs per bucket) (Q14) */
-  double utilization;         /* live_pairs * 8 B / (linked buckets * bucket_bytes) (Fig. 2c) */
+  double load_factor;         /* live_pairs / key slots of the linked (base+overflow)
+                                 buckets (Q14) */
+  double utilization;         /* live_pairs * 8 B / table_bytes (Fig. 2c) */
   uint64_t exchange;          /* batch routing: 0 = none (single GPU), 1 = NCCL all-to-all,
                                  2 = fused partition + peer stores into NVLink-mapped windows */
+  uint64_t table_bytes;       /* bytes of the linked (base+overflow) buckets */
+  uint64_t bump_bytes;        /* bytes of all buckets ever handed out (what the streaming
+                                 purge / tombstone sweeps read) */
 } dg_stats;
 
 /* Fills defaults: load_factor 0.7, bucket_bytes 128, directed 1, pool_bytes 0,

@@ -23,6 +23,7 @@ DG_ERR_UNSUPPORTED = 7
 DG_FLAG_NO_TOMBSTONE_REUSE = 1
 DG_FLAG_FORCE_ROUTER = 2
 DG_FLAG_SET = 4
+DG_FLAG_ADAPTIVE = 8
 
 VP = ctypes.c_void_p
 U64 = ctypes.c_uint64
@@ -60,6 +61,8 @@ class dg_stats(ctypes.Structure):
         ("load_factor", ctypes.c_double),
         ("utilization", ctypes.c_double),
         ("exchange", ctypes.c_uint64),
+        ("table_bytes", ctypes.c_uint64),
+        ("bump_bytes", ctypes.c_uint64),
     ]
 
 

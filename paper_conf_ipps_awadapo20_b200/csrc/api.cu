@@ -180,6 +180,21 @@ dg_status ensure_dedup(dg_graph g, u64 n) {
   return DG_OK;
 }
 
+// spare-bucket return list of an insert launch: one entry per resident thread, plus
+// (adaptive layout) one per op — a lane hands back its spare when the next chain it
+// extends has another size class, which happens at most once per lost link race
+dg_status ensure_ret(dg_graph g, u64 n_ops) {
+  const u64 want = dg::max_groups(g->G, g->sms) + (g->adaptive ? n_ops : 0) + 16;
+  if (want > g->ret_cap) {
+    if (g->ret_list) DG_CK(cudaFree(g->ret_list));
+    g->ret_list = nullptr;
+    g->ret_cap = 0;
+    DG_CK(cudaMalloc(&g->ret_list, want * 4));
+    g->ret_cap = want;
+  }
+  return DG_OK;
+}
+
 dg_status ensure_retry(dg_graph g, int k, u64 n) {
   if (n > g->retry_cap[k]) {
     if (g->retry[k]) cudaFree(g->retry[k]);
@@ -216,26 +231,32 @@ void prof_mark(dg_graph g, int k, cudaStream_t s) {
   g->prof_ev[k].push_back(e);
 }
 
-// Map more pool memory so that at least min_buckets buckets exist; new buckets
-// are all-EMPTY (0xFF bytes: EMPTY keys/values, NIL next, NIL owner).
-dg_status grow_pool(dg_graph g, u64 min_buckets, cudaStream_t s) {
-  const u64 max_buckets = std::min<u64>(0xFFFFFFFEull, g->pool.reserved() / g->bucket_bytes);
+// Map more memory in the pool of size class c so that at least min_buckets buckets
+// exist; new buckets are all-EMPTY (0xFF bytes: EMPTY keys/values, NIL next, NIL
+// owner).  Bucket indices stay below 2^30 (the id's class bits, dg_common.cuh).
+dg_status grow_pool(dg_graph g, int c, u64 min_buckets, cudaStream_t s) {
+  const u64 bb = g->cbytes(c);
+  const u64 max_buckets = std::min<u64>(dg::kIdxMask, g->pool[c].reserved() / bb);
   if (min_buckets > max_buckets) return DG_ERR_OUT_OF_MEMORY;
-  if (min_buckets <= g->cap) return DG_OK;
-  cudaError_t e = g->pool.ensure(min_buckets * g->bucket_bytes, 0xFF, s);
+  if (min_buckets <= g->cap[c]) return DG_OK;
+  static const bool debug = std::getenv("DG_DEBUG") != nullptr;
+  if (debug)
+    std::fprintf(stderr, "dg: pool class %d grows %u -> %llu buckets\n", c, g->cap[c],
+                 (unsigned long long)min_buckets);
+  cudaError_t e = g->pool[c].ensure(min_buckets * bb, 0xFF, s);
   if (e == cudaErrorMemoryAllocation) {
     cudaGetLastError();
     return DG_ERR_OUT_OF_MEMORY;
   }
   DG_CK(e);
-  const u64 nb = std::min<u64>(max_buckets, g->pool.mapped() / g->bucket_bytes);
-  e = g->stack.ensure(nb * 4, -1, s);
+  const u64 nb = std::min<u64>(max_buckets, g->pool[c].mapped() / bb);
+  e = g->stack[c].ensure(nb * 4, -1, s);
   if (e == cudaErrorMemoryAllocation) {
     cudaGetLastError();
     return DG_ERR_OUT_OF_MEMORY;
   }
   DG_CK(e);
-  g->cap = (u32)nb;
+  g->cap[c] = (u32)nb;
   return DG_OK;
 }
 
@@ -244,43 +265,53 @@ namespace {
 // Make sure an insert launch that may allocate `need` buckets cannot fail, if
 // that is cheap; returns whether the launch must run in retry mode (check for
 // failed ops after the launch and re-run them after growing the pool).
+// (every size class must be able to absorb the worst case: all ops of the launch
+// may extend chains of one class)
 dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) {
   *retry_mode = false;
   if (g->snap_pending && cudaEventQuery(g->snap_event) == cudaSuccess) {
     g->snap_pending = false;
-    g->bump_ub = g->hctl->bump;  // exact as of the snapshot; nothing launched since
+    for (int c = 0; c < g->ncls; ++c)  // exact as of the snapshot; nothing launched since
+      g->bump_ub[c] = g->hctl->bump[c];
   }
-  if ((u64)g->cap >= g->bump_ub + need) return DG_OK;
-  // exact free count
+  bool ok = true;
+  for (int c = 0; c < g->ncls; ++c) ok = ok && (u64)g->cap[c] >= g->bump_ub[c] + need;
+  if (ok) return DG_OK;
+  // exact free counts
   DG_TRY(read_ctl(g, s));
   g->snap_pending = false;
-  g->bump_ub = g->hctl->bump;
-  const u64 free_exact = (u64)g->cap - g->hctl->bump + g->hctl->stack_size;
-  if (free_exact >= need) {
-    // pops come from the stack first; the bump cursor moves by at most need - stack
-    return DG_OK;
-  }
-  const u64 missing = need - free_exact;
   static const bool no_upfront = std::getenv("DG_TEST_RETRY_PATH") != nullptr;
   // Reserve the worst case (one new bucket per op) up front when it is bounded
   // (<= 4 GB and half of free device memory): steady-state batches then never
   // synchronise.  Larger batches (bulk builds) launch in retry mode and grow by what
   // actually failed.
-  const u64 limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
-  if (!no_upfront && missing * g->bucket_bytes <= limit) {
-    const u64 want = (u64)g->cap + missing + std::max<u64>(missing / 4, 65536);
-    dg_status st = grow_pool(g, want, s);
-    if (st == DG_OK) return DG_OK;
-    if (st != DG_ERR_OUT_OF_MEMORY) return st;
+  u64 limit = 0;  // cudaMemGetInfo is slow: query it only when a pool must grow
+  for (int c = 0; c < g->ncls; ++c) {
+    g->bump_ub[c] = g->hctl->bump[c];
+    const u64 free_exact = (u64)g->cap[c] - g->hctl->bump[c] + g->hctl->stack_size[c];
+    // pops come from the stack first; the bump cursor moves by at most need - stack
+    if (free_exact >= need) continue;
+    const u64 missing = need - free_exact;
+    if (!limit) limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
+    if (!no_upfront && missing * g->cbytes(c) <= limit) {
+      const u64 want = (u64)g->cap[c] + missing + std::max<u64>(missing / 4, 65536);
+      dg_status st = grow_pool(g, c, want, s);
+      if (st == DG_OK) continue;
+      if (st != DG_ERR_OUT_OF_MEMORY) return st;
+    }
+    *retry_mode = true;
   }
-  *retry_mode = true;
   return DG_OK;
 }
 
 void note_launch(dg_graph g, u64 need, cudaStream_t s) {
-  g->bump_ub = std::min<u64>(g->cap, g->bump_ub + need);
+  bool tight = false;
+  for (int c = 0; c < g->ncls; ++c) {
+    g->bump_ub[c] = std::min<u64>(g->cap[c], g->bump_ub[c] + need);
+    tight = tight || (u64)g->cap[c] < g->bump_ub[c] + need;
+  }
   // snapshot the allocator cursors asynchronously when the bound gets tight
-  if ((u64)g->cap < g->bump_ub + need && !g->snap_pending) {
+  if (tight && !g->snap_pending) {
     if (cudaMemcpyAsync(g->hctl, g->ctl, sizeof(dg::DevCtl), cudaMemcpyDeviceToHost, s) ==
             cudaSuccess &&
         cudaEventRecord(g->snap_event, s) == cudaSuccess)
@@ -306,6 +337,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   }
   DG_TRY(plan_capacity(g, need, s, &retry_mode));
   DG_TRY(ensure_retry(g, 0, n_ops));
+  DG_TRY(ensure_ret(g, n_ops));
   t = g->tables();
   dg::EdgeBatch a{};
   a.src = src;
@@ -335,12 +367,15 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   int cur = 0;
   for (int round = 0;; ++round) {
     DG_TRY(read_ctl(g, s));
-    g->bump_ub = g->hctl->bump;
+    for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = g->hctl->bump[c];
     const u64 failed = g->hctl->retry_count;
     if (failed == 0) break;
     if (round > 64) return DG_ERR_OUT_OF_MEMORY;
-    const u64 want = (u64)g->cap + failed + dg::max_groups(g->G, g->sms) + (u64)g->cap / 4;
-    DG_TRY(grow_pool(g, want, s));
+    for (int c = 0; c < g->ncls; ++c) {  // grow the pools that ran dry
+      if (g->hctl->bump[c] < g->cap[c] && g->ncls > 1) continue;
+      const u64 want = (u64)g->cap[c] + failed + dg::max_groups(g->G, g->sms) + (u64)g->cap[c] / 4;
+      DG_TRY(grow_pool(g, c, want, s));
+    }
     DG_TRY(ensure_retry(g, cur ^ 1, failed));
     DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, sizeof(u32), s));
     t = g->tables();
@@ -407,36 +442,51 @@ dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
     ~Guard() { g->in_rehash = false; }
   } guard{g};
   const u64 m = (u64)n + 1;
-  DG_CK(ensure_buf(g->rh[0], 7 * m * 8));
-  u64* nbnew = reinterpret_cast<u64*>(g->rh[0].p);
+  DG_CK(ensure_buf(g->rh[0], (6 + dg::kClasses) * m * 8));
+  u64* nbnew = reinterpret_cast<u64*>(g->rh[0].p);  // #buckets | class << 40
   u64* nbold = nbnew + m;
   u64* degs = nbold + m;
-  u64* nboff = degs + m;
-  u64* obo = nboff + m;
+  u64* obo = degs + m;
   u64* doff = obo + m;
   u64* cursor = doff + m;
+  u64* nboff = cursor + m;  // per class: kClasses arrays of m
   dg::Tables t = g->tables();
-  DG_CK(dg::launch_hot_sizes(t, n, g->lf_milli, g->BC, flush ? 1u : 0u, nbnew, nbold, degs, s));
-  DG_CK(dg::scan_exclusive_u64(nbnew, nboff, m, &g->scan_temp, &g->scan_bytes, s));
+  DG_CK(dg::launch_hot_sizes(t, n, g->lf_milli, g->BC, flush ? 1u : 0u, g->adaptive ? 1u : 0u,
+                             g->set ? 1u : 0u, nbnew, nbold, degs, s));
+  u64 tot[2 + dg::kClasses] = {};
+  for (int c = 0; c < g->ncls; ++c) {
+    DG_CK(dg::scan_class_offsets(nbnew, n, (u32)c, nboff + c * m, &g->scan_temp, &g->scan_bytes, s));
+    DG_CK(cudaMemcpyAsync(&tot[2 + c], nboff + c * m + n, 8, cudaMemcpyDeviceToHost, s));
+  }
   DG_CK(dg::scan_exclusive_u64(nbold, obo, m, &g->scan_temp, &g->scan_bytes, s));
   DG_CK(dg::scan_exclusive_u64(degs, doff, m, &g->scan_temp, &g->scan_bytes, s));
-  u64 tot[3] = {0, 0, 0};
-  DG_CK(cudaMemcpyAsync(&tot[0], nboff + n, 8, cudaMemcpyDeviceToHost, s));
   DG_CK(cudaMemcpyAsync(&tot[1], doff + n, 8, cudaMemcpyDeviceToHost, s));
   if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   g->snap_pending = false;
   DG_TRY(read_ctl(g, s));
-  const u64 total_new = tot[0], total_deg = tot[1];
+  const u64 total_deg = tot[1];
   if (std::getenv("DG_DEBUG"))
-    std::fprintf(stderr, "dg: re-sizing %u rows (%llu pairs, %llu new base buckets)\n", n,
-                 (unsigned long long)total_deg, (unsigned long long)total_new);
-  const u64 bump0 = g->hctl->bump;
-  if (bump0 + total_new + 1 >= 0xFFFFFFFEull) {  // no room: forget the flags
-    DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
-    DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
-    return flush ? DG_ERR_OUT_OF_MEMORY : DG_OK;
+    std::fprintf(stderr, "dg: re-sizing %u rows (%llu pairs, %llu/%llu/%llu new base buckets)\n",
+                 n, (unsigned long long)total_deg, (unsigned long long)tot[2],
+                 (unsigned long long)tot[3], (unsigned long long)tot[4]);
+  dg::ClassBases cb{};
+  u32 newbump[dg::kClasses] = {0, 0, 0};
+  for (int c = 0; c < g->ncls; ++c) {
+    const u64 bump0 = g->hctl->bump[c];
+    if (bump0 + tot[2 + c] + 1 >= dg::kIdxMask) {  // no room: forget the flags
+      DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
+      DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
+      return flush ? DG_ERR_OUT_OF_MEMORY : DG_OK;
+    }
   }
-  DG_TRY(grow_pool(g, bump0 + total_new + g->cap / 8 + 65536, s));
+  for (int c = 0; c < g->ncls; ++c) {
+    const u64 bump0 = g->hctl->bump[c];
+    if (tot[2 + c]) DG_TRY(grow_pool(g, c, bump0 + tot[2 + c] + g->cap[c] / 8 + 65536, s));
+    cb.off[c] = nboff + c * m;
+    cb.base0[c] = (u32)bump0;
+    cb.words[c] = g->cbytes(c) / 4;
+    newbump[c] = (u32)(bump0 + tot[2 + c]);
+  }
   t = g->tables();
   DG_CK(ensure_buf(g->rh[1], total_deg * 4 + 4));
   DG_CK(ensure_buf(g->rh[2], total_deg * 4 + 4));
@@ -447,15 +497,14 @@ dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
   DG_CK(cudaMemcpyAsync(cursor, doff, n * 8, cudaMemcpyDeviceToDevice, s));
   DG_CK(dg::launch_hot_export(g->lay, t, n, obo, reinterpret_cast<unsigned long long*>(cursor), osrc,
                               odst, ow, g->rank, g->sms, s));
-  DG_CK(dg::launch_hot_release(g->G, t, n, obo, g->sms, s));
-  DG_CK(dg::launch_hot_install(t, n, nbnew, nboff, (u32)bump0, g->W, s));
-  const u32 newbump = (u32)(bump0 + total_new);
-  DG_CK(cudaMemcpyAsync(&g->ctl->bump, &newbump, 4, cudaMemcpyHostToDevice, s));
+  DG_CK(dg::launch_hot_release(g->lay, t, n, obo, g->sms, s));
+  DG_CK(dg::launch_init_rows(t, 0, n, t.hot_list, nbnew, cb, s));
+  DG_CK(cudaMemcpyAsync(g->ctl->bump, newbump, 4 * dg::kClasses, cudaMemcpyHostToDevice, s));
   DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
   DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));  // hot_count, hot_pairs
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, 4, s));
-  g->bump_ub = std::max<u64>(g->bump_ub, newbump);
+  for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::max<u64>(g->bump_ub[c], newbump[c]);
   // the pairs go back through the ordinary insert kernel (all keys distinct)
   DG_TRY(local_insert(g, osrc, odst, ow, total_deg, false, ++g->epoch, s));
   DG_CK(cudaStreamSynchronize(s));
@@ -516,8 +565,8 @@ static void destroy_graph(dg_graph g) {
   if (g->router) dg::router_destroy(g->router);
   g->dir.release();
   g->degv.release();
-  g->pool.release();
-  g->stack.release();
+  for (auto& p : g->pool) p.release();
+  for (auto& p : g->stack) p.release();
   if (g->ctl) cudaFree(g->ctl);
   if (g->hctl) cudaFreeHost(g->hctl);
   if (g->snap_event) cudaEventDestroy(g->snap_event);
@@ -556,27 +605,35 @@ static void destroy_graph(dg_graph g) {
 static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_global,
                           const u32* hints_local, u64 slack_buckets, cudaStream_t s) {
   if (count == 0) return DG_OK;
-  u64* nb = nullptr;
-  u64* off = nullptr;
+  u64* nb = nullptr;   // #buckets | class << 40
+  u64* off = nullptr;  // per class: count + 1 offsets
   DG_CK(cudaMallocAsync(&nb, (count + 1) * 8, s));
-  DG_CK(cudaMallocAsync(&off, (count + 1) * 8, s));
+  DG_CK(cudaMallocAsync(&off, (count + 1) * 8 * g->ncls, s));
   DG_CK(dg::launch_initial_buckets(nb, count, row0, hints_global, hints_local, g->nranks, g->rank,
-                                   g->lf_milli, g->BC, s));
-  DG_CK(dg::scan_exclusive_u64(nb, off, count + 1, &g->scan_temp, &g->scan_bytes, s));
-  u64 total = 0;
-  DG_CK(cudaMemcpyAsync(&total, off + count, 8, cudaMemcpyDeviceToHost, s));
-  DG_TRY(read_ctl(g, s));  // also synchronises
-  const u64 base0 = g->hctl->bump;
-  if (base0 + total + 1 >= 0xFFFFFFFEull) {
-    cudaFreeAsync(nb, s);
-    cudaFreeAsync(off, s);
-    return DG_ERR_OUT_OF_MEMORY;
+                                   g->lf_milli, g->BC, g->adaptive ? 1u : 0u, g->set ? 1u : 0u, s));
+  u64 total[dg::kClasses] = {0, 0, 0};
+  for (int c = 0; c < g->ncls; ++c) {
+    DG_CK(dg::scan_class_offsets(nb, count, (u32)c, off + c * (count + 1), &g->scan_temp,
+                                 &g->scan_bytes, s));
+    DG_CK(cudaMemcpyAsync(&total[c], off + c * (count + 1) + count, 8, cudaMemcpyDeviceToHost, s));
   }
-  dg_status st = dg::grow_pool(g, base0 + total + slack_buckets, s);
-  if (st != DG_OK) {
-    cudaFreeAsync(nb, s);
-    cudaFreeAsync(off, s);
-    return st;
+  DG_TRY(read_ctl(g, s));  // also synchronises
+  dg::ClassBases cb{};
+  u32 newbump[dg::kClasses] = {0, 0, 0};
+  for (int c = 0; c < g->ncls; ++c) {
+    const u64 base0 = g->hctl->bump[c];
+    dg_status st = DG_OK;
+    if (base0 + total[c] + 1 >= dg::kIdxMask) st = DG_ERR_OUT_OF_MEMORY;
+    if (st == DG_OK) st = dg::grow_pool(g, c, base0 + total[c] + slack_buckets, s);
+    if (st != DG_OK) {
+      cudaFreeAsync(nb, s);
+      cudaFreeAsync(off, s);
+      return st;
+    }
+    cb.off[c] = off + c * (count + 1);
+    cb.base0[c] = (u32)base0;
+    cb.words[c] = g->cbytes(c) / 4;
+    newbump[c] = (u32)(base0 + total[c]);
   }
   cudaError_t e = g->dir.ensure((row0 + count) * sizeof(dg::DirEntry), 0, s);
   if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
@@ -597,13 +654,12 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
       DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));
     }
   }
-  DG_CK(dg::launch_init_rows(g->G, g->tables(), row0, count, off, nb, (u32)base0, s));
-  const u32 newbump = (u32)(base0 + total);
-  DG_CK(cudaMemcpyAsync(&g->ctl->bump, &newbump, 4, cudaMemcpyHostToDevice, s));
+  DG_CK(dg::launch_init_rows(g->tables(), row0, count, nullptr, nb, cb, s));
+  DG_CK(cudaMemcpyAsync(g->ctl->bump, newbump, 4 * dg::kClasses, cudaMemcpyHostToDevice, s));
   DG_CK(cudaFreeAsync(nb, s));
   DG_CK(cudaFreeAsync(off, s));
   DG_CK(cudaStreamSynchronize(s));
-  g->bump_ub = std::max<u64>(g->bump_ub, newbump);
+  for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::max<u64>(g->bump_ub[c], newbump[c]);
   return DG_OK;
 }
 
@@ -618,7 +674,8 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
-  if (cfg->flags & ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER | DG_FLAG_SET))
+  if (cfg->flags &
+      ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER | DG_FLAG_SET | DG_FLAG_ADAPTIVE))
     return DG_ERR_INVALID_ARGUMENT;
 
   dg_graph g = new (std::nothrow) dg_graph_s();
@@ -638,12 +695,14 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   cudaDeviceProp prop;
   if (cudaGetDeviceProperties(&prop, g->device) != cudaSuccess) return fail(DG_ERR_CUDA);
   g->sms = prop.multiProcessorCount;
-  g->bucket_bytes = cfg->bucket_bytes;
-  g->G = (int)(cfg->bucket_bytes / 16);
-  g->W = cfg->bucket_bytes / 4;
+  g->adaptive = (cfg->flags & DG_FLAG_ADAPTIVE) != 0;
+  g->ncls = g->adaptive ? dg::kClasses : 1;
+  g->bucket_bytes = g->adaptive ? 128u : cfg->bucket_bytes;  // adaptive: largest class
+  g->G = (int)(g->bucket_bytes / 16);
+  g->W = g->bucket_bytes / 4;
   g->set = (cfg->flags & DG_FLAG_SET) != 0;
-  g->BC = g->set ? cfg->bucket_bytes / 4 - 2 : cfg->bucket_bytes / 8 - 1;  // Q15
-  g->lay = DG_LAY(g->G, g->set ? 1 : 0);
+  g->BC = g->set ? g->bucket_bytes / 4 - 2 : g->bucket_bytes / 8 - 1;  // Q15
+  g->lay = DG_LAYA(g->G, g->set ? 1 : 0, g->adaptive ? 1 : 0);
   g->lf_milli = std::max<u32>(1, (u32)std::lround((double)cfg->load_factor * 1000.0));
   g->nranks = (u32)cfg->nranks;
   g->rank = (u32)cfg->rank;
@@ -652,9 +711,11 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   g->nv = num_vertices;
 
   const size_t total_mem = prop.totalGlobalMem;
-  if (g->pool.reserve(g->device, total_mem) != cudaSuccess) return fail(DG_ERR_CUDA);
-  if (g->stack.reserve(g->device, total_mem / g->bucket_bytes * 4 + (2u << 20)) != cudaSuccess)
-    return fail(DG_ERR_CUDA);
+  for (int c = 0; c < g->ncls; ++c) {
+    if (g->pool[c].reserve(g->device, total_mem) != cudaSuccess) return fail(DG_ERR_CUDA);
+    if (g->stack[c].reserve(g->device, total_mem / g->cbytes(c) * 4 + (2u << 20)) != cudaSuccess)
+      return fail(DG_ERR_CUDA);
+  }
   const u64 max_rows = (kMaxVertices + g->nranks - 1) / g->nranks + 1;
   if (g->dir.reserve(g->device, max_rows * sizeof(dg::DirEntry)) != cudaSuccess ||
       g->degv.reserve(g->device, max_rows * sizeof(u32)) != cudaSuccess)
@@ -665,8 +726,7 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   std::memset(g->hctl, 0, sizeof(dg::DevCtl));
   if (cudaEventCreateWithFlags(&g->snap_event, cudaEventDisableTiming) != cudaSuccess)
     return fail(DG_ERR_CUDA);
-  if (cudaMalloc(&g->ret_list, dg::max_groups(g->G, g->sms) * 4 + 64) != cudaSuccess)
-    return fail(DG_ERR_CUDA);
+  if (ensure_ret(g, 0) != DG_OK) return fail(DG_ERR_CUDA);
   if (cudaMalloc(&g->small_dev, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
   if (const char* hs = std::getenv("DG_HOT_STEPS")) g->hot_steps = (u32)std::atoi(hs);
   if (cudaMalloc(&g->hot_list, (size_t)g->hot_cap * 4) != cudaSuccess) return fail(DG_ERR_CUDA);
@@ -703,7 +763,7 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (rows) {
     st = add_rows(g, 0, rows, reinterpret_cast<const u32*>(hints), nullptr, slack, s);
   } else {
-    st = dg::grow_pool(g, slack, s);
+    for (int c = 0; c < g->ncls && st == DG_OK; ++c) st = dg::grow_pool(g, c, slack, s);
   }
   if (st != DG_OK) return fail(st);
   if (cudaStreamSynchronize(s) != cudaSuccess) return fail(DG_ERR_CUDA);
@@ -785,7 +845,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     if (g->router) DG_TRY(dg::router_sum_u64(g, &cnt, s));
     if (n_added) *n_added = cnt;
     g->snap_pending = false;
-    g->bump_ub = g->hctl->bump;
+    for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = g->hctl->bump[c];
     return status_of(g, epoch);
   }
   return DG_OK;
@@ -1011,7 +1071,7 @@ dg_status dg_delete_vertices(dg_graph g, const uint32_t* ids, uint64_t n, void* 
     // directed: follow-up sweep over all tables
     DG_CK(dg::launch_vdel_sweep(g->lay, t, g->bitmap, filter, fshift, epoch, g->sms, s));
   }
-  DG_CK(dg::launch_vdel_clear(g->G, t, g->dedup, boff, epoch, g->sms, s));
+  DG_CK(dg::launch_vdel_clear(g->lay, t, g->dedup, boff, epoch, g->sms, s));
   dg::prof_mark(g, dg::PROF_VDEL, s);
   if (host) {
     if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
@@ -1088,16 +1148,21 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   out->exchange = !g->router ? 0 : dg::router_fused(g->router) ? 2 : 1;
   out->base_buckets = h.base_buckets;
   out->overflow_buckets = h.linked_buckets - h.base_buckets;
-  out->free_buckets = g->hctl->stack_size;
-  out->pool_buckets = g->cap;
-  out->bump_buckets = g->hctl->bump;
+  out->pool_bytes = g->dir.mapped() + g->degv.mapped();
+  for (int c = 0; c < g->ncls; ++c) {
+    out->free_buckets += g->hctl->stack_size[c];
+    out->pool_buckets += g->cap[c];
+    out->bump_buckets += g->hctl->bump[c];
+    out->bump_bytes += (u64)g->hctl->bump[c] * g->cbytes(c);
+    out->pool_bytes += g->pool[c].mapped() + g->stack[c].mapped();
+  }
   out->live_pairs = h.live;
   out->tombstones = h.tombs;
   out->max_chain = h.max_chain;
-  out->pool_bytes = g->pool.mapped() + g->dir.mapped() + g->degv.mapped() + g->stack.mapped();
-  out->load_factor = h.linked_buckets ? (double)h.live / ((double)h.linked_buckets * g->BC) : 0.0;
-  out->utilization =
-      h.linked_buckets ? (double)h.live * 8.0 / ((double)h.linked_buckets * g->bucket_bytes) : 0.0;
+  // realised load factor = keys / key slots of the linked buckets (Q14)
+  out->load_factor = h.slots ? (double)h.live / (double)h.slots : 0.0;
+  out->utilization = h.bytes ? (double)h.live * 8.0 / (double)h.bytes : 0.0;
+  out->table_bytes = h.bytes;
   return DG_OK;
 }
 

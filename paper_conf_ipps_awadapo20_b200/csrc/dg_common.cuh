@@ -14,6 +14,13 @@
 //                chained buckets come from the allocator.
 //   free stack : u32[pool capacity] of reclaimed bucket indices + bump cursor
 //   ctl        : DevCtl (allocator cursors, counters, validation epochs)
+//
+// Bucket ids: bits 31..30 = size class (index of the pool the bucket lives in),
+// bits 29..0 = index in that pool.  Uniform layouts use class 0 only (one pool of
+// `bucket_bytes` buckets).  The degree-adaptive layout (DG_FLAG_ADAPTIVE, SURVEY
+// §8(f) row 4, "hash tables with varying slab sizes") keeps three pools:
+// class c holds 32 << c byte buckets (32 / 64 / 128 B), and every bucket of a row
+// (base and chained) has the row's class, so a bucket id alone fixes its geometry.
 #pragma once
 #include <cstdint>
 #include <cuda_runtime.h>
@@ -27,6 +34,10 @@ constexpr u32 kEmpty = 0xFFFFFFFFu;       // empty key slot (Q18)
 constexpr u32 kTomb = 0xFFFFFFFEu;        // tombstone (deleted key)
 constexpr u32 kNil = 0xFFFFFFFFu;         // end of chain / no bucket
 constexpr u64 kEmptyPair = 0xFFFFFFFFFFFFFFFFull;
+constexpr u32 kClassShift = 30;           // bucket id = class << 30 | index
+constexpr u32 kIdxMask = (1u << kClassShift) - 1u;
+constexpr int kClasses = 3;               // adaptive size classes: 32, 64, 128 B
+constexpr u64 kNbMask = (1ull << 40) - 1; // packed (#buckets | class << 40) entries
 
 struct __align__(8) DirEntry {
   u32 base;    // first base bucket
@@ -34,9 +45,10 @@ struct __align__(8) DirEntry {
 };
 
 struct DevCtl {
-  u32 pop_count;     // pops taken from the free stack during the current insert phase
-  u32 stack_size;    // reclaimed buckets on the free stack
-  u32 bump;          // next never-used bucket index
+  // allocator, per size class (uniform layouts use class 0)
+  u32 pop_count[kClasses];   // pops taken from the free stack during the current insert phase
+  u32 stack_size[kClasses];  // reclaimed buckets on the free stack
+  u32 bump[kClasses];        // next never-used bucket index
   u32 ret_count;     // unused spare buckets handed back during the current insert phase
   u32 retry_count;   // ops that found no free bucket (pool exhausted) this launch
   u32 fail_epoch;    // highest batch epoch rejected by validation (0 = none)
@@ -51,12 +63,12 @@ struct DevCtl {
 struct Tables {
   DirEntry* dir;
   u32* deg;          // exact degree per local row
-  u32* pool;
-  u32* stack;
+  u32* pool[kClasses];   // bucket pool per size class
+  u32* stack[kClasses];  // free stack per size class (bucket ids)
   DevCtl* ctl;
   u32* ret_list;     // spare buckets returned (<= number of groups launched)
   u64 rows;          // local rows
-  u32 cap;           // buckets mapped in the pool
+  u32 cap[kClasses]; // buckets mapped in each pool
   u32 nranks;        // row = global id / nranks at nranks > 1
   u32* hot_flags;    // bit per local row: flagged for re-sizing (nullable = off)
   u32* hot_list;     // flagged rows
@@ -180,8 +192,79 @@ struct Lay {
   static __device__ __forceinline__ u32 word(u32 uu, int k) { return 4 * uu + (S ? k : 2 * k); }
 };
 
-// layout code passed to the launchers: G | set << 5
+// Per-class fields of a kernel-parameter Tables, selected without dynamic indexing
+// (a runtime index into a parameter array makes the compiler copy the whole struct
+// to local memory).
+template <typename T>
+__device__ __forceinline__ T by_class(const T (&a)[kClasses], u32 c) {
+  return c == 0 ? a[0] : (c == 1 ? a[1] : a[2]);
+}
+
+// Geometry of one bucket: where it lives and how many 16-B units it has.  Uniform
+// layouts (A = false) fold to the compile-time Lay<G, S> (pool 0, G units); the
+// adaptive layout (A = true, G = 8 lanes = the largest class) reads the size class
+// from the id: class c = 2 << c units in pool c.  Slot k of unit uu exists iff
+// uu < units and (uu is not the last unit or k < SPU/2); the last unit's words z, w
+// hold the next link and the owner row, as in Lay.
+template <int G, int S, bool A>
+struct Geo {
+  typedef Lay<G, S> LY;
+  u32* p;     // first word of the bucket
+  u32 units;  // 16-B units
+  __device__ __forceinline__ Geo(const Tables& t, u32 id) {
+    if constexpr (A) {
+      const u32 c = id >> kClassShift;
+      units = 2u << c;
+      p = by_class(t.pool, c) + (u64)(id & kIdxMask) * (8u << c);
+    } else {
+      units = G;
+      p = t.pool[0] + (u64)id * LY::W;
+    }
+  }
+  __device__ __forceinline__ u32 words() const { return 4 * units; }
+  __device__ __forceinline__ u32 next_word() const { return 4 * units - 2; }
+  __device__ __forceinline__ u32 owner_word() const { return 4 * units - 1; }
+  __device__ __forceinline__ bool has(u32 uu, int k) const { return has_u(units, uu, k); }
+  __device__ __forceinline__ u32 bc() const { return bc_u(units); }
+  // the same from a unit count alone (no pointer arithmetic)
+  static __device__ __forceinline__ bool has_u(u32 units, u32 uu, int k) {
+    if constexpr (A) return uu < units && (uu != units - 1 || k < LY::SPU / 2);
+    else return LY::has(uu, k);
+  }
+  static __device__ __forceinline__ u32 bc_u(u32 units) {  // slots per bucket (Q15)
+    if constexpr (A) return S ? 4 * units - 2 : 2 * units - 1;
+    else return LY::BC;
+  }
+};
+
+// units of a bucket id (no pool access)
+template <int G, bool A>
+__device__ __forceinline__ u32 units_of(u32 id) {
+  if constexpr (A) return 2u << (id >> kClassShift);
+  else return (u32)G;
+}
+
+// Degree-adaptive layout (adaptive = 1): the row gets the
+// smallest size class whose single bucket holds its hint at the load factor
+// (32 B: hint <= lf*Bc_0, 64 B: hint <= lf*Bc_1), else 128-B buckets sized by the
+// same rule.  Returns #buckets | class << 40 (kNbMask selects the count).
+__device__ __forceinline__ u64 class_size(u64 hint, u32 lf_milli, u32 set) {
+  for (u32 c = 0; c + 1 < (u32)kClasses; ++c) {
+    const u64 bcc = set ? (8u << c) - 2 : (4u << c) - 1;
+    if (hint * 1000 <= (u64)lf_milli * bcc) return 1ull | ((u64)c << 40);
+  }
+  const u64 den = (u64)lf_milli * (set ? 30u : 15u);
+  const u64 b = (hint * 1000 + den - 1) / den;
+  return (b ? b : 1ull) | ((u64)(kClasses - 1) << 40);
+}
+
+// layout code passed to the launchers: G | set << 5 | adaptive << 6
 #define DG_LAY(G, S) ((G) | ((S) << 5))
+#define DG_LAYA(G, S, A) ((G) | ((S) << 5) | ((A) << 6))
+#define DG_ADAPTIVE_BIT 64
 #define DG_FOR_LAYOUTS(X) X(2, 0) X(4, 0) X(8, 0) X(2, 1) X(4, 1) X(8, 1)
+// every layout incl. the adaptive ones (G = 8 lanes, runtime class)
+#define DG_FOR_LAYOUTS_A(X) \
+  X(2, 0, 0) X(4, 0, 0) X(8, 0, 0) X(2, 1, 0) X(4, 1, 0) X(8, 1, 0) X(8, 0, 1) X(8, 1, 1)
 
 }  // namespace dg

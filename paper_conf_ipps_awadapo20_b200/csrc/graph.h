@@ -18,12 +18,14 @@ struct dg_graph_s {
   dg_config cfg{};
   int device = 0;
   int sms = 148;
-  int G = 8;              // lanes per bucket (bucket_bytes / 16)
+  int G = 8;              // lanes per bucket (bucket_bytes / 16; adaptive: 8)
   bool set = false;       // set variant: keys only (DG_FLAG_SET)
+  bool adaptive = false;  // degree-adaptive bucket sizes (DG_FLAG_ADAPTIVE)
+  int ncls = 1;           // size classes in use (uniform 1, adaptive 3)
   int lay = DG_LAY(8, 0); // layout code for the launchers
-  uint32_t W = 32;        // words per bucket
-  uint32_t BC = 15;       // pairs (keys, set variant) per bucket
-  uint32_t bucket_bytes = 128;
+  uint32_t W = 32;        // words per bucket (uniform layouts)
+  uint32_t BC = 15;       // pairs (keys, set variant) per bucket (uniform layouts)
+  uint32_t bucket_bytes = 128;  // uniform layouts; adaptive: the largest class
   uint32_t lf_milli = 700;
   uint32_t nranks = 1, rank = 0;
   bool directed = true;
@@ -32,15 +34,19 @@ struct dg_graph_s {
   uint64_t nv = 0;        // global vertex capacity
   uint64_t rows = 0;      // local rows
 
-  dg::VmmArray dir, degv, pool, stack;
-  uint32_t cap = 0;       // buckets mapped in the pool
-  uint64_t bump_ub = 0;   // host upper bound of the device bump cursor
+  dg::VmmArray dir, degv;
+  dg::VmmArray pool[dg::kClasses], stack[dg::kClasses];  // per size class
+  uint32_t cap[dg::kClasses] = {0, 0, 0};      // buckets mapped in each pool
+  uint64_t bump_ub[dg::kClasses] = {0, 0, 0};  // host upper bounds of the device bump cursors
+  // bytes of one bucket of class c
+  uint32_t cbytes(int c) const { return adaptive ? (32u << c) : bucket_bytes; }
 
   dg::DevCtl* ctl = nullptr;       // device
   dg::DevCtl* hctl = nullptr;      // pinned host mirror (snapshots)
   cudaEvent_t snap_event = nullptr;
   bool snap_pending = false;
   uint32_t* ret_list = nullptr;
+  uint64_t ret_cap = 0;
   uint64_t* retry[2] = {nullptr, nullptr};
   uint64_t retry_cap[2] = {0, 0};
   uint32_t* bitmap = nullptr;
@@ -92,12 +98,14 @@ struct dg_graph_s {
     dg::Tables t;
     t.dir = reinterpret_cast<dg::DirEntry*>(dir.ptr());
     t.deg = reinterpret_cast<uint32_t*>(degv.ptr());
-    t.pool = reinterpret_cast<uint32_t*>(pool.ptr());
-    t.stack = reinterpret_cast<uint32_t*>(stack.ptr());
+    for (int c = 0; c < dg::kClasses; ++c) {
+      t.pool[c] = c < ncls ? reinterpret_cast<uint32_t*>(pool[c].ptr()) : nullptr;
+      t.stack[c] = c < ncls ? reinterpret_cast<uint32_t*>(stack[c].ptr()) : nullptr;
+      t.cap[c] = c < ncls ? cap[c] : 0;
+    }
     t.ctl = ctl;
     t.ret_list = ret_list;
     t.rows = rows;
-    t.cap = cap;
     t.nranks = nranks;
     t.hot_flags = hot_steps ? hot_flags : nullptr;
     t.hot_list = hot_list;
@@ -118,7 +126,7 @@ enum ProfKind { PROF_INSERT = 0, PROF_DELETE = 1, PROF_QUERY = 2, PROF_VDEL = 3,
 void prof_mark(dg_graph g, int k, cudaStream_t s);
 
 // internal entry points shared by api.cu and router.cu
-dg_status grow_pool(dg_graph g, uint64_t min_buckets, cudaStream_t s);
+dg_status grow_pool(dg_graph g, int c, uint64_t min_buckets, cudaStream_t s);
 dg_status rehash_hot(dg_graph g, cudaStream_t s);
 dg_status rehash_rows(dg_graph g, uint32_t n, bool flush, cudaStream_t s);
 dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,

@@ -32,7 +32,8 @@ struct EdgeBatch {
   u32 reuse_tombstones;  // insert: install new keys in the first tombstone
 };
 
-// `lay` = DG_LAY(G, S): G 16-B units per bucket, S = 1 for the set variant
+// `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1
+// for the degree-adaptive layout (G = 8 lanes, size class per bucket id)
 // (keys only); launchers that take `G` are layout-independent.
 // edge ops (kernels_edges.cu)
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
@@ -44,18 +45,31 @@ cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s);
 u64 max_groups(int G, int sms);
 
 // graph structure (kernels_graph.cu)
-// nb[r] for rows r in [0, count): initial bucket count from a hint.
+// nb[r] for rows r in [0, count): initial bucket count from a hint,
+//   packed as #buckets | class << 40 (uniform layouts: class 0; adaptive: the size
+//   class rule of class_size()).
 //   hint source: hints_global[(row0 + r) * nranks + rank] if hints_global, else
 //   hints_local[r] if hints_local, else 0.
 cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
                                    const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
-                                   u32 bc, cudaStream_t s);
+                                   u32 bc, u32 adaptive, u32 set, cudaStream_t s);
+// off[r] = sum over r' < r of the class-c buckets of nbc[r'] (count + 1 entries)
+cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u64* off, void** temp,
+                               size_t* temp_bytes, cudaStream_t s);
 // out[i] = sum of in[0..i) for i < count (temp storage grows as needed)
 cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
                                size_t* temp_bytes, cudaStream_t s);
-// dir[row0 + r] = {base0 + off[r], nb[r], 0, 0}; owner word of each base bucket = row
-cudaError_t launch_init_rows(int G, const Tables& t, u64 row0, u64 count, const u64* off,
-                             const u64* nb, u32 base0, cudaStream_t s);
+// where the base buckets of new rows go, per size class
+struct ClassBases {
+  const u64* off[kClasses];  // per-row offsets within the class's new range
+  u32 base0[kClasses];       // first bucket index of the class's new range
+  u32 words[kClasses];       // words per bucket of the class
+};
+// dir[row] = {class << 30 | base0[c] + off[c][r], #buckets}, row = rows ? rows[r] :
+// row0 + r; owner word of each base bucket = row (rows != NULL: re-sizing, which also
+// clears the row's hot flag)
+cudaError_t launch_init_rows(const Tables& t, u64 row0, u64 count, const u32* rows,
+                             const u64* nbc, const ClassBases& cb, cudaStream_t s);
 // new-row hints for vertex insertion (scatter, max over duplicates)
 cudaError_t launch_scatter_hints(u32* hint_new, u64 row0, u64 count, const u32* ids,
                                  const u32* hints, u64 n, u32 nranks, u32 rank, cudaStream_t s);
@@ -70,6 +84,7 @@ cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst
 
 struct StatsOut {
   unsigned long long base_buckets, linked_buckets, live, tombs, max_chain;
+  unsigned long long slots, bytes;  // key slots / bytes of the linked buckets
 };
 cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s);
 
@@ -87,7 +102,7 @@ cudaError_t launch_vdel_nb(const Tables& t, const u32* dedup, u64 n_max, u64* nb
                            cudaStream_t s);
 cudaError_t launch_vdel_neighbors(int lay, const Tables& t, const u32* dedup, const u64* boff,
                                   u32 epoch, int sms, cudaStream_t s);
-cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
+cudaError_t launch_vdel_clear(int lay, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
                               int sms, cudaStream_t s);
 
 // triangle counting consumer (kernels_tc.cu)
@@ -102,16 +117,14 @@ cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u3
 // per-vertex re-sizing of long-chained tables (kernels_rehash.cu)
 // flush = 0: re-size for long chains (room to double); 1: tombstone flush (the
 // initial-size rule for the live keys)
-cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
-                             u64* nbold, u64* degs, cudaStream_t s);
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u32 adaptive,
+                             u32 set, u64* nbnew, u64* nbold, u64* degs, cudaStream_t s);
 // rows holding a tombstone -> hot flags / hot list (tombstone flush)
 cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s);
 cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
                               unsigned long long* cursor, u32* osrc, u32* odst, u32* ow, u32 rank,
                               int sms, cudaStream_t s);
-cudaError_t launch_hot_release(int G, const Tables& t, u32 n, const u64* obo, int sms,
+cudaError_t launch_hot_release(int lay, const Tables& t, u32 n, const u64* obo, int sms,
                                cudaStream_t s);
-cudaError_t launch_hot_install(const Tables& t, u32 n, const u64* nbnew, const u64* nboff,
-                               u32 base0, u32 words, cudaStream_t s);
 
 }  // namespace dg

@@ -41,11 +41,46 @@ enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 // Phase-concurrent free stack + bump cursor: during an insert
 // phase buckets are only popped, during a vertex-deletion phase only pushed, so
 // a single cursor per direction is ABA-free.
-__device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 stack_size) {
-  u32 i = atomicAdd(&t.ctl->pop_count, 1u);
-  if (i < stack_size) return t.stack[stack_size - 1 - i];
-  u32 j = atomicAdd(&t.ctl->bump, 1u);
-  return j < t.cap ? j : kNil;
+// Size class c (uniform layouts: 0); returns a bucket id of class c or NIL.
+// ss0 = class-0 stack size read at kernel start (uniform layouts); the adaptive layout
+// reads its class's size here (stack sizes are fixed during an insert phase).
+template <bool A>
+__device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 c, u32 ss0) {
+  const u32 stack_size = A ? ld_relaxed_u32(&t.ctl->stack_size[c]) : ss0;
+  u32 i = atomicAdd(&t.ctl->pop_count[c], 1u);
+  if (i < stack_size) return by_class(t.stack, c)[stack_size - 1 - i];
+  u32 j = atomicAdd(&t.ctl->bump[c], 1u);
+  return j < by_class(t.cap, c) ? (c << kClassShift) | j : kNil;
+}
+
+// Warp-aggregated allocation: the lanes that need a bucket of the same class take
+// consecutive pops (one atomic per class per warp instead of one per lane; a hot
+// single-address atomic otherwise serialises chain growth), and the ones past the
+// free stack consecutive bump slots.  Called by the whole warp; returns NIL for lanes
+// with !want.
+template <bool A>
+__device__ __forceinline__ u32 alloc_bucket_warp(const Tables& t, bool want, u32 c, u32 ss0) {
+  const u32 lane = threadIdx.x & 31u;
+  const u32 below = (1u << lane) - 1u;
+  const u32 peers = __match_any_sync(0xFFFFFFFFu, want ? c : 0xFFFFFFFFu);
+  if (!want) return kNil;
+  const u32 leader = __ffs(peers) - 1;
+  u32 base = 0, ss = 0;
+  if (lane == leader) {
+    ss = A ? ld_relaxed_u32(&t.ctl->stack_size[c]) : ss0;  // fixed during the phase
+    base = atomicAdd(&t.ctl->pop_count[c], (u32)__popc(peers));
+  }
+  base = __shfl_sync(peers, base, leader);
+  ss = __shfl_sync(peers, ss, leader);
+  const u32 i = base + __popc(peers & below);
+  const bool from_stack = i < ss;
+  const u32 over = __ballot_sync(peers, !from_stack);
+  if (from_stack) return by_class(t.stack, c)[ss - 1 - i];
+  const u32 l2 = __ffs(over) - 1;
+  u32 b = 0;
+  if (lane == l2) b = atomicAdd(&t.ctl->bump[c], (u32)__popc(over));
+  const u32 j = __shfl_sync(over, b, l2) + __popc(over & below);
+  return j < by_class(t.cap, c) ? (c << kClassShift) | j : kNil;
 }
 
 // ------------------------------------------------------------- main kernel ----
@@ -89,14 +124,16 @@ struct Lanes {
   static constexpr int K = G / L;
 };
 
-template <int G, int S, int OP, bool MAIN>
+// A: degree-adaptive layout (bucket geometry from the id's size class, G = 8 lanes
+// cover the largest class; lanes past a smaller bucket load nothing).
+template <int G, int S, int OP, bool MAIN, bool A>
 __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
                                         const Group<Lanes<G, OP>::L>& g, const bool valid,
-                                        const u64 opid, const u64 j, const u32 stack_size,
+                                        const u64 opid, const u64 j, const u32 ss0,
                                         const bool reuse, u32& my_count, u32& spare,
                                         bool& bad_range) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
+  typedef Geo<G, S, A> GEO;
   constexpr int L = Lanes<G, OP>::L;
   constexpr int K = Lanes<G, OP>::K;
   constexpr u32 FULL = 0xFFFFFFFFu;
@@ -143,11 +180,13 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
 #pragma unroll
     for (int r = 0; r < L; ++r) {
       const u32 cr = __shfl_sync(FULL, cur, g.base + r);
-      const u32* p = t.pool + (u64)cr * W + 4 * K * g.gl;
+      const GEO gr(t, cr);
+      const u32* p = gr.p + 4 * K * g.gl;
       const bool pr = (pm >> (g.base + r)) & 1u;
 #pragma unroll
       for (int c = 0; c < K; ++c) {
-        if (pr) q[r][c] = (OP == OP_QUERY) ? ld_nc_v4(p + 4 * c) : ld_relaxed_v4(p + 4 * c);
+        if (pr && (!A || K * g.gl + c < gr.units))
+          q[r][c] = (OP == OP_QUERY) ? ld_nc_v4(p + 4 * c) : ld_relaxed_v4(p + 4 * c);
         else q[r][c] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
       }
     }
@@ -159,6 +198,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       const bool pr = (pm >> srcl) & 1u;
       const u32 vr = __shfl_sync(FULL, v, srcl);
       const u32 cr = __shfl_sync(FULL, cur, srcl);
+      const u32 units = units_of<G, A>(cr);
       bool lhit = false, lempty = false, lfree = false;
       u32 hslot = 0, hval = 0, fslot = 0;   // key word indices in the bucket
       unsigned long long fcont = 0;
@@ -168,7 +208,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
         const u32 uu = K * g.gl + c;               // 16-B unit index in the bucket
 #pragma unroll
         for (int k = 0; k < LY::SPU; ++k) {
-          if (!LY::has(uu, k)) continue;           // (next, owner) words of the last unit
+          if (!GEO::has_u(units, uu, k)) continue;  // (next, owner) words of the last unit
           const u32 kk = LY::key(x, k);
           if (pr && !lhit && kk == vr) { lhit = true; hslot = LY::word(uu, k); hval = LY::val(x, k); }
           const bool e = kk == kEmpty;
@@ -181,7 +221,8 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       }
       const u32 hit = (__ballot_sync(FULL, lhit) >> g.base) & GBITS;
       const u32 em = (__ballot_sync(FULL, lempty) >> g.base) & GBITS;
-      const u32 next = __shfl_sync(FULL, q[r][K - 1].z, g.base + L - 1);
+      // the last unit (odd index) is unit K-1 of lane (units-1)/K
+      const u32 next = __shfl_sync(FULL, q[r][K - 1].z, g.base + (units - 1) / K);
       const bool end = em != 0 || next == kNil;  // EMPTY slots only exist at the tail
       const u32 lh = hit ? __ffs(hit) - 1 : 0;
       const bool mine = pr && g.gl == (u32)r;
@@ -195,13 +236,13 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       } else if (OP == OP_DELETE) {
         const u32 hs = __shfl_sync(FULL, hslot, g.base + lh);
         if (mine) {
-          if (hit) { act = ACT_CAS_DEL; ff = t.pool + (u64)cur * W + hs; }
+          if (hit) { act = ACT_CAS_DEL; ff = GEO(t, cur).p + hs; }
           else if (end) pend = false;
           else cur = next;
         }
       } else {  // insert
         const u32 wr = __shfl_sync(FULL, w, srcl);
-        if (!S && lhit && g.gl == lh) st_relaxed_u32(t.pool + (u64)cr * W + hslot + 1, wr);  // replace
+        if (!S && lhit && g.gl == lh) st_relaxed_u32(GEO(t, cr).p + hslot + 1, wr);  // replace
         const u32 fm = (__ballot_sync(FULL, lfree) >> g.base) & GBITS;
         const u32 lf = fm ? __ffs(fm) - 1 : 0;
         const u32 sslot = __shfl_sync(FULL, fslot, g.base + lf);
@@ -210,7 +251,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
           if (hit) {
             pend = false;
           } else {
-            if (!ff && fm) { ff = t.pool + (u64)cur * W + sslot; ffo = so; }
+            if (!ff && fm) { ff = GEO(t, cur).p + sslot; ffo = so; }
             if (end) {
               act = ff ? ACT_CAS_INS : ACT_EXTEND;
             } else {
@@ -220,7 +261,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
               // metric + rehash)
               if (++steps == t.hot_steps && t.hot_flags) {
                 const u32 dr = ld_relaxed_u32(t.deg + row);
-                if (dr > nbase * LY::BC) {
+                if (dr > nbase * GEO::bc_u(units)) {
                   const u32 bit = 1u << (row & 31);
                   if (!(atomicOr(&t.hot_flags[row >> 5], bit) & bit)) {
                     const u32 k = atomicAdd(&t.ctl->hot_count, 1u);
@@ -259,15 +300,28 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
         ff = nullptr;
       }
     }
+    if (OP == OP_INSERT) {
+      // chain full: link a new bucket at the tail (a8), of the row's class
+      const bool ext = act == ACT_EXTEND;
+      const u32 cls = A ? cur >> kClassShift : 0u;
+      if (A && ext && spare != kNil && (spare >> kClassShift) != cls) {  // spare of another class
+        t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
+        spare = kNil;
+      }
+      const bool want = ext && spare == kNil;
+      if (__any_sync(FULL, want)) {
+        const u32 got = alloc_bucket_warp<A>(t, want, cls, ss0);
+        if (want) spare = got;
+      }
+    }
     if (OP == OP_INSERT && act == ACT_EXTEND) {
-      // chain full: link a new bucket at the tail (a8)
-      if (spare == kNil) spare = alloc_bucket(t, stack_size);
       if (spare == kNil) {  // pool exhausted: the host grows it and re-runs this op
         a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
         pend = false;
       } else {
-        st_relaxed_u32(t.pool + (u64)spare * W + LY::OWNER, row);
-        const u32 old = atomicCAS(t.pool + (u64)cur * W + LY::NEXT, kNil, spare);
+        const GEO gs(t, spare), gc(t, cur);
+        st_relaxed_u32(gs.p + gs.owner_word(), row);
+        const u32 old = atomicCAS(gc.p + gc.next_word(), kNil, spare);
         if (old == kNil) {
           cur = spare;
           spare = kNil;
@@ -304,15 +358,15 @@ template <int OP>
 struct MinBlocks {
   static constexpr int v = OP == OP_INSERT ? DG_MINB_INS : OP == OP_QUERY ? DG_MINB_QRY : DG_MINB_DEL;
 };
-template <int G, int S, int OP>
+template <int G, int S, int OP, bool A>
 __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<Lanes<G, OP>::L> g;
   if (OP != OP_QUERY) {
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
   }
-  const u32 stack_size = (OP == OP_INSERT) ? ld_relaxed_u32(&t.ctl->stack_size) : 0u;
   const bool reuse = a.reuse_tombstones != 0;
+  const u32 ss0 = (OP == OP_INSERT && !A) ? ld_relaxed_u32(&t.ctl->stack_size[0]) : 0u;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
   u32 my_count = 0;
@@ -327,8 +381,8 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
     const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
-    const bool d = run_ops<G, S, OP, true>(t, a, g, valid, opid, j, stack_size, reuse, my_count,
-                                        spare, bad_range);
+    const bool d = run_ops<G, S, OP, true, A>(t, a, g, valid, opid, j, ss0, reuse, my_count, spare,
+                                           bad_range);
     const u32 dm = __ballot_sync(FULL, d);
     if (d) bl[nbl + __popc(dm & below)] = OP == OP_QUERY ? j : opid;
     nbl += __popc(dm);
@@ -337,8 +391,8 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
       nbl -= 32;
       const u64 op2 = bl[nbl + g.lane];
       __syncwarp();
-      run_ops<G, S, OP, false>(t, a, g, true, op2, op2, stack_size, reuse, my_count, spare,
-                            bad_range);
+      run_ops<G, S, OP, false, A>(t, a, g, true, op2, op2, ss0, reuse, my_count, spare,
+                                  bad_range);
     }
   }
   while (nbl > 0) {  // drain the backlog
@@ -347,8 +401,8 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const bool valid = g.lane < take;
     const u64 op2 = valid ? bl[nbl + g.lane] : 0;
     __syncwarp();
-    run_ops<G, S, OP, false>(t, a, g, valid, op2, op2, stack_size, reuse, my_count, spare,
-                          bad_range);
+    run_ops<G, S, OP, false, A>(t, a, g, valid, op2, op2, ss0, reuse, my_count, spare,
+                                bad_range);
   }
   // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
   if (OP == OP_INSERT && spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
@@ -378,34 +432,40 @@ __global__ void k_validate(const u32* __restrict__ src, const u32* __restrict__ 
   if (__any_sync(0xFFFFFFFFu, bad) && (threadIdx.x & 31) == 0) atomicMax(&ctl->fail_epoch, epoch);
 }
 
-// After an insert phase: drop the popped entries from the free stack, clamp the
-// bump cursor, and push the spare buckets that were handed back.
+// After an insert phase: drop the popped entries from each class's free stack,
+// clamp the bump cursors, and push the spare buckets that were handed back onto the
+// stack of their class.
 __global__ void k_fixup_alloc(Tables t) {
-  __shared__ u32 s_ss, s_rc;
+  __shared__ u32 s_ss[kClasses], s_rc;
   DevCtl* c = t.ctl;
-  if (threadIdx.x == 0) {
-    const u32 pc = c->pop_count, ss = c->stack_size;
-    s_ss = pc >= ss ? 0u : ss - pc;
-    s_rc = c->ret_count;
-    if (c->bump > t.cap) c->bump = t.cap;
+  if (threadIdx.x < kClasses) {
+    const u32 k = threadIdx.x;
+    const u32 pc = c->pop_count[k], ss = c->stack_size[k];
+    s_ss[k] = pc >= ss ? 0u : ss - pc;
+    if (c->bump[k] > by_class(t.cap, k)) c->bump[k] = by_class(t.cap, k);
+  }
+  if (threadIdx.x == 0) s_rc = c->ret_count;
+  __syncthreads();
+  for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) {
+    const u32 id = t.ret_list[k];
+    const u32 cl = id >> kClassShift;
+    by_class(t.stack, cl)[atomicAdd(&s_ss[cl], 1u)] = id;
   }
   __syncthreads();
-  for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) t.stack[s_ss + k] = t.ret_list[k];
-  __syncthreads();
-  if (threadIdx.x == 0) {
-    c->stack_size = s_ss + s_rc;
-    c->pop_count = 0;
-    c->ret_count = 0;
+  if (threadIdx.x < kClasses) {
+    c->stack_size[threadIdx.x] = s_ss[threadIdx.x];
+    c->pop_count[threadIdx.x] = 0;
   }
+  if (threadIdx.x == 0) c->ret_count = 0;
 }
 
 // ---------------------------------------------------------------- launchers ----
-template <int G, int S, int OP>
+template <int G, int S, int OP, bool A>
 static int grid_for() {
   static int blocks_per_sm = -1;
   if (blocks_per_sm < 0) {
     int b = 0;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_edges<G, S, OP>, kEdgeBlock, 0) !=
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, k_edges<G, S, OP, A>, kEdgeBlock, 0) !=
             cudaSuccess || b <= 0)
       b = 1;
     blocks_per_sm = b;
@@ -413,23 +473,23 @@ static int grid_for() {
   return blocks_per_sm;
 }
 
-template <int G, int S, int OP>
+template <int G, int S, int OP, bool A>
 static cudaError_t launch_g(const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
   if (a.n_ops == 0) return cudaSuccess;
   const u64 warps_needed = (a.n_ops + 31) / 32;
   const u64 per_block = kEdgeBlock / 32;
   u64 blocks = (warps_needed + per_block - 1) / per_block;
-  const u64 maxb = (u64)sms * grid_for<G, S, OP>();
+  const u64 maxb = (u64)sms * grid_for<G, S, OP, A>();
   if (blocks > maxb) blocks = maxb;
-  k_edges<G, S, OP><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
+  k_edges<G, S, OP, A><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
   return cudaGetLastError();
 }
 
 template <int OP>
 static cudaError_t launch_op(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s) {
   switch (lay) {
-#define DG_CASE(G, S) case DG_LAY(G, S): return launch_g<G, S, OP>(t, a, sms, s);
-    DG_FOR_LAYOUTS(DG_CASE)
+#define DG_CASE(G, S, A) case DG_LAYA(G, S, A): return launch_g<G, S, OP, A>(t, a, sms, s);
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }

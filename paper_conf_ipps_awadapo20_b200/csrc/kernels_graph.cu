@@ -14,7 +14,7 @@ namespace dg {
 // ceiling is an exact integer decision (reading R-LF).
 __global__ void k_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
                                   const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
-                                  u32 bc) {
+                                  u32 bc, u32 adaptive, u32 set) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r <= count; r += stride) {
     if (r == count) {
@@ -24,6 +24,10 @@ __global__ void k_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints
     u64 hint = 0;
     if (hints_global) hint = hints_global[(row0 + r) * nranks + rank];
     else if (hints_local) hint = hints_local[r];
+    if (adaptive) {
+      nb[r] = class_size(hint, lf_milli, set);
+      continue;
+    }
     const u64 den = (u64)lf_milli * bc;
     u64 b = hint ? (hint * 1000 + den - 1) / den : 1;
     nb[r] = b ? b : 1;
@@ -32,11 +36,12 @@ __global__ void k_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints
 
 cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hints_global,
                                    const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
-                                   u32 bc, cudaStream_t s) {
+                                   u32 bc, u32 adaptive, u32 set, cudaStream_t s) {
   u64 blocks = (count + 1 + 255) / 256;
   if (blocks > 65535) blocks = 65535;
   k_initial_buckets<<<(unsigned)blocks, 256, 0, s>>>(nb, count, row0, hints_global, hints_local,
-                                                     nranks, rank, lf_milli, bc); note_kernel(1);
+                                                     nranks, rank, lf_milli, bc, adaptive, set);
+  note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -57,35 +62,68 @@ cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
   return cub::DeviceScan::ExclusiveSum(*temp, need, in, out, (int64_t)count, s);
 }
 
-// dir[row0 + r] = {base0 + off[r], nb[r], 0, 0}; each base bucket records its owner row.
-template <int G>
-__global__ void k_init_rows(Tables t, u64 row0, u64 count, const u64* off, const u64* nb,
-                            u32 base0) {
-  constexpr int W = Group<G>::W;
+// buckets of class c in a packed (#buckets | class << 40) entry
+struct ClassCount {
+  const u64* nbc;
+  u64 n;
+  u32 c;
+  __host__ __device__ u64 operator()(u64 i) const {
+    if (i >= n) return 0ull;
+    const u64 v = nbc[i];
+    return (u32)(v >> 40) == c ? (v & kNbMask) : 0ull;
+  }
+};
+
+cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u64* off, void** temp,
+                               size_t* temp_bytes, cudaStream_t s) {
+  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0),
+                                            ClassCount{nbc, count, c});
+  size_t need = 0;
+  cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, off, (int64_t)(count + 1), s);
+  if (e != cudaSuccess) return e;
+  if (need > *temp_bytes) {
+    if (*temp) cudaFree(*temp);
+    *temp = nullptr;
+    *temp_bytes = 0;
+    e = cudaMalloc(temp, need);
+    if (e != cudaSuccess) return e;
+    *temp_bytes = need;
+  }
+  note_kernel(2);
+  return cub::DeviceScan::ExclusiveSum(*temp, need, it, off, (int64_t)(count + 1), s);
+}
+
+// Row r gets nbc[r] consecutive base buckets of its class c, starting at
+// cb.base0[c] + cb.off[c][r]; each base bucket records its owner row.  `rows`
+// (nullable) maps r to a directory row (re-sizing), else row = row0 + r.
+__global__ void k_init_rows(Tables t, u64 row0, u64 count, const u32* rows, const u64* nbc,
+                            ClassBases cb) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < count; r += stride) {
-    const u32 base = base0 + (u32)off[r];
-    const u32 n = (u32)nb[r];
+    const u64 v = nbc[r];
+    const u32 c = (u32)(v >> 40);
+    const u32 n = (u32)(v & kNbMask);
+    const u32 idx = by_class(cb.base0, c) + (u32)by_class(cb.off, c)[r];
+    const u32 row = rows ? rows[r] : (u32)(row0 + r);
     DirEntry e;
-    e.base = base;
+    e.base = (c << kClassShift) | idx;
     e.nb = n;
-    t.dir[row0 + r] = e;
-    t.deg[row0 + r] = 0;
-    for (u32 k = 0; k < n; ++k) t.pool[(u64)(base + k) * W + Group<G>::OWNER] = (u32)(row0 + r);
+    t.dir[row] = e;
+    t.deg[row] = 0;
+    const u32 wc = by_class(cb.words, c);
+    u32* pool = by_class(t.pool, c);
+    for (u32 k = 0; k < n; ++k) pool[(u64)(idx + k) * wc + wc - 1] = row;
+    if (rows && t.hot_flags) atomicAnd(&t.hot_flags[row >> 5], ~(1u << (row & 31)));
   }
 }
 
-cudaError_t launch_init_rows(int G, const Tables& t, u64 row0, u64 count, const u64* off,
-                             const u64* nb, u32 base0, cudaStream_t s) {
+cudaError_t launch_init_rows(const Tables& t, u64 row0, u64 count, const u32* rows,
+                             const u64* nbc, const ClassBases& cb, cudaStream_t s) {
   if (count == 0) return cudaSuccess;
   u64 blocks = (count + 255) / 256;
   if (blocks > 65535) blocks = 65535;
-  switch (G) {
-    case 2: k_init_rows<2><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
-    case 4: k_init_rows<4><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
-    case 8: k_init_rows<8><<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, off, nb, base0); note_kernel(1); break;
-    default: return cudaErrorInvalidValue;
-  }
+  k_init_rows<<<(unsigned)blocks, 256, 0, s>>>(t, row0, count, rows, nbc, cb);
+  note_kernel(1);
   return cudaGetLastError();
 }
 
@@ -174,22 +212,22 @@ cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t*
 // buckets (hubs) are listed in big[1..] (count in big[0]) and exported by
 // k_export_big, one block per row, so one group never walks a hub's thousands of
 // buckets alone.  The order of a row's entries is unspecified.
-template <int G, int S>
-__device__ __forceinline__ u32 export_bucket(const Group<G>& g, const uint4& q, u32* dst, u32* w,
-                                             u64 pos) {
+template <int G, int S, bool A>
+__device__ __forceinline__ u32 export_bucket(const Group<G>& g, const Geo<G, S, A>& gb,
+                                             const uint4& q, u32* dst, u32* w, u64 pos) {
   typedef Lay<G, S> LY;
   const u32 below = (1u << g.gl) - 1u;
   u32 before = 0, total = 0;
 #pragma unroll
   for (int j = 0; j < LY::SPU; ++j) {
-    const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+    const u32 m = g.ballot(gb.has(g.gl, j) && LY::key(q, j) < kTomb);
     before += __popc(m & below);
     total += __popc(m);
   }
   u64 at = pos + before;
 #pragma unroll
   for (int j = 0; j < LY::SPU; ++j) {
-    if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
+    if (gb.has(g.gl, j) && LY::key(q, j) < kTomb) {
       dst[at] = LY::key(q, j);
       if (w) w[at] = LY::val(q, j);
       ++at;
@@ -198,10 +236,16 @@ __device__ __forceinline__ u32 export_bucket(const Group<G>& g, const uint4& q, 
   return total;
 }
 
-template <int G, int S>
+// load lane gl's 16-B unit of bucket gb (lanes past a smaller adaptive bucket get EMPTY)
+template <int G, int S, bool A>
+__device__ __forceinline__ uint4 ld_unit(const Geo<G, S, A>& gb, u32 gl) {
+  if (A && gl >= gb.units) return make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+  return ld_nc_v4(gb.p + 4 * gl);
+}
+
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u32* dst, u32* w,
                                                      u32* big) {
-  constexpr int W = Lay<G, S>::W;
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
@@ -215,18 +259,18 @@ __global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u3
     for (u32 k = 0; k < de.nb; ++k) {
       u32 b = de.base + k;
       while (b != kNil) {
-        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
-        pos += export_bucket<G, S>(g, q, dst, w, pos);
-        b = g.shfl(q.z, G - 1);
+        const Geo<G, S, A> gb(t, b);
+        const uint4 q = ld_unit(gb, g.gl);
+        pos += export_bucket(g, gb, q, dst, w, pos);
+        b = g.shfl(q.z, gb.units - 1);
       }
     }
   }
 }
 
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_export_big(Tables t, const u64* ro, u32* dst, u32* w,
                                                     const u32* big) {
-  constexpr int W = Lay<G, S>::W;
   __shared__ unsigned long long cursor;
   const Group<G> g;
   const u32 gib = threadIdx.x / G, ngb = blockDim.x / G;
@@ -240,15 +284,16 @@ __global__ void __launch_bounds__(256) k_export_big(Tables t, const u64* ro, u32
     for (u32 k = gib; k < de.nb; k += ngb) {
       u32 b = de.base + k;
       while (b != kNil) {
-        const uint4 q = ld_nc_v4(t.pool + (u64)b * W + 4 * g.gl);
+        const Geo<G, S, A> gb(t, b);
+        const uint4 q = ld_unit(gb, g.gl);
         u32 cnt = 0;
 #pragma unroll
         for (int j = 0; j < Lay<G, S>::SPU; ++j)
-          cnt += __popc(g.ballot(Lay<G, S>::has(g.gl, j) && Lay<G, S>::key(q, j) < kTomb));
+          cnt += __popc(g.ballot(gb.has(g.gl, j) && Lay<G, S>::key(q, j) < kTomb));
         unsigned long long pos = 0;
         if (g.gl == 0 && cnt) pos = atomicAdd(&cursor, (unsigned long long)cnt);
-        export_bucket<G, S>(g, q, dst, w, g.shfl(pos, 0));
-        b = g.shfl(q.z, G - 1);
+        export_bucket(g, gb, q, dst, w, g.shfl(pos, 0));
+        b = g.shfl(q.z, gb.units - 1);
       }
     }
   }
@@ -263,12 +308,12 @@ cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst
   cudaError_t e = cudaMemsetAsync(big, 0, 4, s);
   if (e != cudaSuccess) return e;
   switch (lay) {
-#define DG_CASE(G_, S_)                                                                   \
-  case DG_LAY(G_, S_):                                                                    \
-    k_export_fill<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w, big);           \
-    k_export_big<G_, S_><<<(unsigned)sms * 2, 256, 0, s>>>(t, ro, dst, w, big); \
+#define DG_CASE(G_, S_, A_)                                                               \
+  case DG_LAYA(G_, S_, A_):                                                               \
+    k_export_fill<G_, S_, A_><<<(unsigned)blocks, 256, 0, s>>>(t, ro, dst, w, big);       \
+    k_export_big<G_, S_, A_><<<(unsigned)sms * 2, 256, 0, s>>>(t, ro, dst, w, big);       \
     break;
-    DG_FOR_LAYOUTS(DG_CASE)
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
@@ -278,35 +323,54 @@ cudaError_t launch_export_fill(int lay, const Tables& t, const u64* ro, u32* dst
 
 // --------------------------------------------------------------- statistics ----
 // one base-bucket chain: live / tombstone slots and its length
-template <int G, int S>
+// per-thread accumulators of k_stats / k_stats_big
+struct StatsAcc {
+  unsigned long long linked = 0, live = 0, tombs = 0, maxc = 0, slots = 0, bytes = 0;
+};
+
+template <int G, int S, bool A>
 __device__ __forceinline__ void stats_chain(const Tables& t, const Group<G>& g, u32 b,
-                                            unsigned long long& live, unsigned long long& tombs,
-                                            unsigned long long& linked, unsigned long long& maxc) {
+                                            StatsAcc& a) {
   typedef Lay<G, S> LY;
   unsigned long long len = 0;
   while (b != kNil) {
-    const uint4 q = ld_nc_v4(t.pool + (u64)b * LY::W + 4 * g.gl);
+    const Geo<G, S, A> gb(t, b);
+    const uint4 q = ld_unit(gb, g.gl);
 #pragma unroll
     for (int j = 0; j < LY::SPU; ++j) {
-      const bool h = LY::has(g.gl, j);
-      live += __popc(g.ballot(h && LY::key(q, j) < kTomb));
-      tombs += __popc(g.ballot(h && LY::key(q, j) == kTomb));
+      const bool h = gb.has(g.gl, j);
+      a.live += __popc(g.ballot(h && LY::key(q, j) < kTomb));
+      a.tombs += __popc(g.ballot(h && LY::key(q, j) == kTomb));
     }
     ++len;
-    b = g.shfl(q.z, G - 1);
+    a.slots += gb.bc();
+    a.bytes += 16 * gb.units;
+    b = g.shfl(q.z, gb.units - 1);
   }
-  linked += len;
-  if (len > maxc) maxc = len;
+  a.linked += len;
+  if (len > a.maxc) a.maxc = len;
+}
+
+__device__ __forceinline__ void stats_flush(StatsOut* out, const StatsAcc& a) {
+  if (a.linked | a.live | a.tombs) {
+    atomicAdd(&out->linked_buckets, a.linked);
+    atomicAdd(&out->live, a.live);
+    atomicAdd(&out->tombs, a.tombs);
+    atomicAdd(&out->slots, a.slots);
+    atomicAdd(&out->bytes, a.bytes);
+    atomicMax(&out->max_chain, a.maxc);
+  }
 }
 
 // group per row; hub rows (> kBigRowBuckets base buckets) are split over the
 // groups of one block by k_stats_big
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out, u32* big) {
   const Group<G> g;
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
-  unsigned long long nbase = 0, linked = 0, live = 0, tombs = 0, maxc = 0;
+  unsigned long long nbase = 0;
+  StatsAcc a;
   for (u64 row = gid; row < t.rows; row += ng) {
     const DirEntry de = t.dir[row];
     nbase += de.nb;
@@ -314,33 +378,25 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out, u32* big
       if (g.gl == 0) big[1 + atomicAdd(big, 1u)] = (u32)row;
       continue;
     }
-    for (u32 k = 0; k < de.nb; ++k) stats_chain<G, S>(t, g, de.base + k, live, tombs, linked, maxc);
+    for (u32 k = 0; k < de.nb; ++k) stats_chain<G, S, A>(t, g, de.base + k, a);
   }
   if (g.gl == 0) {
-    atomicAdd(&out->base_buckets, nbase);
-    atomicAdd(&out->linked_buckets, linked);
-    atomicAdd(&out->live, live);
-    atomicAdd(&out->tombs, tombs);
-    atomicMax(&out->max_chain, maxc);
+    if (nbase) atomicAdd(&out->base_buckets, nbase);
+    stats_flush(out, a);
   }
 }
 
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_stats_big(Tables t, StatsOut* out, const u32* big) {
   const Group<G> g;
   const u32 gib = threadIdx.x / G, ngb = blockDim.x / G;
-  unsigned long long linked = 0, live = 0, tombs = 0, maxc = 0;
+  StatsAcc a;
   const u32 nbig = big[0];
   for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
     const DirEntry de = t.dir[big[1 + i]];
-    for (u32 k = gib; k < de.nb; k += ngb) stats_chain<G, S>(t, g, de.base + k, live, tombs, linked, maxc);
+    for (u32 k = gib; k < de.nb; k += ngb) stats_chain<G, S, A>(t, g, de.base + k, a);
   }
-  if (g.gl == 0 && (linked | live | tombs)) {
-    atomicAdd(&out->linked_buckets, linked);
-    atomicAdd(&out->live, live);
-    atomicAdd(&out->tombs, tombs);
-    atomicMax(&out->max_chain, maxc);
-  }
+  if (g.gl == 0) stats_flush(out, a);
 }
 
 cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s) {
@@ -351,12 +407,12 @@ cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int 
   u64 blocks = (t.rows * G + 255) / 256;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   switch (lay) {
-#define DG_CASE(G_, S_)                                                      \
-  case DG_LAY(G_, S_):                                                       \
-    k_stats<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, out, big);           \
-    k_stats_big<G_, S_><<<(unsigned)sms * 2, 256, 0, s>>>(t, out, big); \
+#define DG_CASE(G_, S_, A_)                                                  \
+  case DG_LAYA(G_, S_, A_):                                                  \
+    k_stats<G_, S_, A_><<<(unsigned)blocks, 256, 0, s>>>(t, out, big);       \
+    k_stats_big<G_, S_, A_><<<(unsigned)sms * 2, 256, 0, s>>>(t, out, big);  \
     break;
-    DG_FOR_LAYOUTS(DG_CASE)
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
@@ -407,10 +463,11 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // vertices in all hash tables"): one streaming pass over every allocated bucket
 // of the pool (coalesced, G lanes per bucket); every live key in D becomes a
 // tombstone and the owner row's degree drops by one.
+// One launch per size class c: the pool of class c holds buckets of G units.
 template <int G, int S>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     const u32* __restrict__ filter, u32 fshift,
-                                                    u32 epoch) {
+                                                    u32 epoch, u32 cls) {
   typedef Lay<G, S> LY;
   constexpr int W = LY::W;
   constexpr int U = 4;  // buckets in flight per group (memory-level parallelism)
@@ -419,7 +476,8 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   for (u32 i = threadIdx.x; i < kVdelFilterBits / 32; i += blockDim.x) sf[i] = filter[i];
   __syncthreads();
-  const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
+  const u32 nbk = ld_relaxed_u32(&t.ctl->bump[cls]);
+  u32* const pool = by_class(t.pool, cls);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b0 = gid; b0 < nbk; b0 += ng * U) {
@@ -427,13 +485,13 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const u64 b = b0 + (u64)k * ng;
-      q[k] = b < nbk ? *reinterpret_cast<const uint4*>(t.pool + b * W + 4 * g.gl)
+      q[k] = b < nbk ? *reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl)
                      : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
     }
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const u64 b = b0 + (u64)k * ng;
-      u32* bp = t.pool + b * W;
+      u32* bp = pool + b * W;
       const uint4 x = q[k];
       const u32 owner = g.shfl(x.w, G - 1);
       u32 dec = 0;
@@ -454,10 +512,23 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const u32* filter,
                               u32 fshift, u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
+  if (lay & DG_ADAPTIVE_BIT) {  // one sweep per size class pool (32 / 64 / 128 B)
+    if (lay & 32) {
+      k_vdel_sweep<2, 1><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);
+      k_vdel_sweep<4, 1><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 1);
+      k_vdel_sweep<8, 1><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 2);
+    } else {
+      k_vdel_sweep<2, 0><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);
+      k_vdel_sweep<4, 0><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 1);
+      k_vdel_sweep<8, 0><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 2);
+    }
+    note_kernel(3);
+    return cudaGetLastError();
+  }
   switch (lay) {
-#define DG_CASE(G_, S_)                                                                  \
-  case DG_LAY(G_, S_):                                                                   \
-    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch); \
+#define DG_CASE(G_, S_)                                                                    \
+  case DG_LAY(G_, S_):                                                                     \
+    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);      \
     break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
@@ -468,18 +539,19 @@ cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const
 }
 
 // probe used by the undirected purge: delete key v from the table starting at b
-template <int G, int S>
+template <int G, int S, bool A>
 __device__ __forceinline__ int purge_delete(const Tables& t, const Group<G>& g, u32 b, u32 v) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
   while (true) {
-    u32* bp = t.pool + (u64)b * W;
-    const uint4 q = ld_relaxed_v4(bp + 4 * g.gl);
+    const Geo<G, S, A> gb(t, b);
+    u32* bp = gb.p;
+    const uint4 q = (A && g.gl >= gb.units) ? make_uint4(kEmpty, kEmpty, kEmpty, kEmpty)
+                                            : ld_relaxed_v4(bp + 4 * g.gl);
     bool m = false, e = false;
     u32 wd = 0;
 #pragma unroll
     for (int j = 0; j < LY::SPU; ++j) {
-      const bool h = LY::has(g.gl, j);
+      const bool h = gb.has(g.gl, j);
       if (h && !m && LY::key(q, j) == v) { m = true; wd = LY::word(g.gl, j); }
       e |= h && LY::key(q, j) == kEmpty;
     }
@@ -491,7 +563,7 @@ __device__ __forceinline__ int purge_delete(const Tables& t, const Group<G>& g, 
       return g.shfl(old, l) == v ? 1 : 0;
     }
     if (g.ballot(e)) return 0;
-    const u32 next = g.shfl(q.z, G - 1);
+    const u32 next = g.shfl(q.z, gb.units - 1);
     if (next == kNil) return 0;
     b = next;
   }
@@ -532,11 +604,10 @@ __device__ __forceinline__ u32 owner_of(const u64* boff, u32 cnt, u64 x) {
 // Undirected purge, Alg. 2: for every deleted vertex u,
 // iterate over A_u (L11-12) and delete u from A_v of every neighbour v (L13-17).
 // Valid only for graphs kept symmetric (directed = 0, single rank).
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* dedup,
                                                         const u64* boff, u32 epoch) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
@@ -549,20 +620,22 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
     const u32 u = dedup[k];
     u32 b = t.dir[u].base + (u32)(x - boff[k]);
     while (b != kNil) {
-      const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
+      const Geo<G, S, A> gb(t, b);
+      const uint4 q = (A && g.gl >= gb.units) ? make_uint4(kEmpty, kEmpty, kEmpty, kEmpty)
+                                              : ld_relaxed_v4(gb.p + 4 * g.gl);
 #pragma unroll
       for (int j = 0; j < LY::SPU; ++j) {
-        u32 lm = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+        u32 lm = g.ballot(gb.has(g.gl, j) && LY::key(q, j) < kTomb);
         while (lm) {
           const u32 l = __ffs(lm) - 1;
           lm &= lm - 1;
           const u32 v = g.shfl(LY::key(q, j), l);
           const DirEntry dv = t.dir[v];
-          if (purge_delete<G, S>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
+          if (purge_delete<G, S, A>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
             atomicSub(&t.deg[v], 1u);
         }
       }
-      b = g.shfl(q.z, G - 1);
+      b = g.shfl(q.z, gb.units - 1);
     }
   }
 }
@@ -571,9 +644,11 @@ cudaError_t launch_vdel_neighbors(int lay, const Tables& t, const u32* dedup, co
                                   u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (lay) {
-#define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_vdel_neighbors<G_, S_><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); break;
-    DG_FOR_LAYOUTS(DG_CASE)
+#define DG_CASE(G_, S_, A_)                                                               \
+  case DG_LAYA(G_, S_, A_):                                                               \
+    k_vdel_neighbors<G_, S_, A_><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch);           \
+    break;
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
@@ -585,10 +660,9 @@ cudaError_t launch_vdel_neighbors(int lay, const Tables& t, const u32* dedup, co
 // pushed on the free stack (dynamic memory reclaimed); base buckets
 // are reset to EMPTY in place (Q9: static memory is kept but must not keep stale
 // keys); degree := 0.  One group per (vertex, base bucket).
-template <int G>
+template <int G, bool A>
 __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, const u64* boff,
                                                     u32 epoch) {
-  constexpr int W = Group<G>::W;
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   const u32 cnt = ld_relaxed_u32(&t.ctl->dedup_count);
@@ -604,12 +678,17 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
     u32 b = t.dir[row].base + j;
     bool base_bucket = true;
     while (b != kNil) {
-      u32* bp = t.pool + (u64)b * W + 4 * g.gl;
-      const uint4 q = ld_relaxed_v4(bp);
-      const u32 next = g.shfl(q.z, G - 1);
-      if (g.last()) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
-      else st_v4(bp, empty4);
-      if (!base_bucket && g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
+      const Geo<G, 0, A> gb(t, b);
+      const bool in = !A || g.gl < gb.units;
+      u32* bp = gb.p + 4 * g.gl;
+      const uint4 q = in ? ld_relaxed_v4(bp) : empty4;
+      const u32 next = g.shfl(q.z, gb.units - 1);
+      if (g.gl == gb.units - 1) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
+      else if (in) st_v4(bp, empty4);
+      if (!base_bucket && g.gl == 0) {
+        const u32 c = b >> kClassShift;
+        by_class(t.stack, c)[atomicAdd(&t.ctl->stack_size[c], 1u)] = b;
+      }
       base_bucket = false;
       b = next;
     }
@@ -617,13 +696,18 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
   }
 }
 
-cudaError_t launch_vdel_clear(int G, const Tables& t, const u32* dedup, const u64* boff, u32 epoch,
-                              int sms, cudaStream_t s) {
+cudaError_t launch_vdel_clear(int lay, const Tables& t, const u32* dedup, const u64* boff,
+                              u32 epoch, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
-  switch (G) {
-    case 2: k_vdel_clear<2><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
-    case 4: k_vdel_clear<4><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
-    case 8: k_vdel_clear<8><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+  if (lay & DG_ADAPTIVE_BIT) {
+    k_vdel_clear<8, true><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch);
+    note_kernel(1);
+    return cudaGetLastError();
+  }
+  switch (lay & 31) {
+    case 2: k_vdel_clear<2, false><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 4: k_vdel_clear<4, false><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
+    case 8: k_vdel_clear<8, false><<<blocks, 256, 0, s>>>(t, dedup, boff, epoch); note_kernel(1); break;
     default: return cudaErrorInvalidValue;
   }
   return cudaGetLastError();

@@ -5,10 +5,12 @@
 // An insert that walks more than `hot_steps` chained buckets flags its row
 // (k_edges).  Before the next insert batch the host re-sizes the flagged rows:
 //   k_hot_sizes    : new #base buckets = max(nb+1, ceil(2*deg / (lf*Bc))), old nb, deg
+//                    (degree-adaptive layout: the size class is chosen again for 2*deg,
+//                    so a growing row moves up to larger buckets)
 //   k_hot_export   : live pairs of the flagged tables -> (src, dst, w) lists
 //   k_hot_release  : every bucket of the old tables (base and chained) reset to
 //                    EMPTY and pushed on the free stack
-//   k_hot_install  : new directory entries over a fresh consecutive base range
+//   k_init_rows    : new directory entries over a fresh consecutive base range
 // and the exported pairs are inserted again with the ordinary insert kernel.  The
 // logical graph is unchanged (same keys, same values, exact degrees); only chain
 // lengths (and any tombstones of those rows) go away.
@@ -17,8 +19,8 @@
 
 namespace dg {
 
-__global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
-                            u64* nbold, u64* degs) {
+__global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u32 flush, u32 adaptive,
+                            u32 set, u64* nbnew, u64* nbold, u64* degs) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k <= n; k += stride) {
     if (k == n) {
@@ -28,6 +30,16 @@ __global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u32 flush, u6
     const u32 row = t.hot_list[k];
     const DirEntry de = t.dir[row];
     const u64 d = t.deg[row];
+    if (adaptive) {  // size class and #buckets by the initial rule (k_initial_buckets)
+      u64 v = class_size(flush ? d : 2 * d, lf_milli, set);
+      const u32 oc = de.base >> kClassShift;
+      if (!flush && (u32)(v >> 40) == oc && (v & kNbMask) < (u64)de.nb + 1)
+        v = ((u64)oc << 40) | ((u64)de.nb + 1);
+      nbnew[k] = v;
+      nbold[k] = de.nb;
+      degs[k] = d;
+      continue;
+    }
     const u64 den = (u64)lf_milli * bc;
     u64 want;
     if (flush) {  // tombstone flush: the initial-size rule for the live keys
@@ -54,12 +66,11 @@ __device__ __forceinline__ u32 seg_of(const u64* off, u32 cnt, u64 x) {
 }
 
 // one group per (flagged row, old base bucket): walk the chain, append live pairs
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* obo,
                                                     unsigned long long* cursor, u32* osrc,
                                                     u32* odst, u32* ow, u32 rank) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
   const Group<G> g;
   const u64 total = obo[n];
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
@@ -71,11 +82,13 @@ __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* 
     const u32 gid_u = row * t.nranks + rank;  // global source id
     u32 b = t.dir[row].base + (u32)(x - obo[k]);
     while (b != kNil) {
-      const uint4 q = ld_relaxed_v4(t.pool + (u64)b * W + 4 * g.gl);
+      const Geo<G, S, A> gb(t, b);
+      const uint4 q = (A && g.gl >= gb.units) ? make_uint4(kEmpty, kEmpty, kEmpty, kEmpty)
+                                              : ld_relaxed_v4(gb.p + 4 * g.gl);
       u32 before = 0, cnt = 0;
 #pragma unroll
       for (int j = 0; j < LY::SPU; ++j) {
-        const u32 m = g.ballot(LY::has(g.gl, j) && LY::key(q, j) < kTomb);
+        const u32 m = g.ballot(gb.has(g.gl, j) && LY::key(q, j) < kTomb);
         before += __popc(m & below);
         cnt += __popc(m);
       }
@@ -84,23 +97,22 @@ __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* 
       u64 at = g.shfl(pos, 0) + before;
 #pragma unroll
       for (int j = 0; j < LY::SPU; ++j) {
-        if (LY::has(g.gl, j) && LY::key(q, j) < kTomb) {
+        if (gb.has(g.gl, j) && LY::key(q, j) < kTomb) {
           osrc[at] = gid_u;
           odst[at] = LY::key(q, j);
           ow[at] = LY::val(q, j);
           ++at;
         }
       }
-      b = g.shfl(q.z, G - 1);
+      b = g.shfl(q.z, gb.units - 1);
     }
   }
 }
 
 // every bucket of the old tables -> EMPTY, onto the free stack (base ones too: the
 // row moves to a new base range)
-template <int G>
+template <int G, bool A>
 __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64* obo) {
-  constexpr int W = Group<G>::W;
   const Group<G> g;
   const u64 total = obo[n];
   const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
@@ -111,30 +123,18 @@ __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64*
     const u32 row = t.hot_list[k];
     u32 b = t.dir[row].base + (u32)(x - obo[k]);
     while (b != kNil) {
-      u32* bp = t.pool + (u64)b * W + 4 * g.gl;
-      const uint4 q = ld_relaxed_v4(bp);
-      const u32 next = g.shfl(q.z, G - 1);
-      st_v4(bp, empty4);
-      if (g.gl == 0) t.stack[atomicAdd(&t.ctl->stack_size, 1u)] = b;
+      const Geo<G, 0, A> gb(t, b);
+      const bool in = !A || g.gl < gb.units;
+      u32* bp = gb.p + 4 * g.gl;
+      const uint4 q = in ? ld_relaxed_v4(bp) : empty4;
+      const u32 next = g.shfl(q.z, gb.units - 1);
+      if (in) st_v4(bp, empty4);
+      if (g.gl == 0) {
+        const u32 c = b >> kClassShift;
+        by_class(t.stack, c)[atomicAdd(&t.ctl->stack_size[c], 1u)] = b;
+      }
       b = next;
     }
-  }
-}
-
-__global__ void k_hot_install(Tables t, u32 n, const u64* nbnew, const u64* nboff, u32 base0,
-                              u32 words) {
-  const u64 stride = (u64)gridDim.x * blockDim.x;
-  for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k < n; k += stride) {
-    const u32 row = t.hot_list[k];
-    const u32 base = base0 + (u32)nboff[k];
-    const u32 nb = (u32)nbnew[k];
-    DirEntry e;
-    e.base = base;
-    e.nb = nb;
-    t.dir[row] = e;
-    t.deg[row] = 0;
-    for (u32 j = 0; j < nb; ++j) t.pool[(u64)(base + j) * words + words - 1] = row;
-    atomicAnd(&t.hot_flags[row >> 5], ~(1u << (row & 31)));
   }
 }
 
@@ -143,14 +143,15 @@ __global__ void k_hot_install(Tables t, u32 n, const u64* nbnew, const u64* nbof
 // holding a tombstone flags its owner row (bucket word W-1) for a compacting
 // re-build (the rows are then re-sized with flush = 1).
 template <int G, int S>
-__global__ void __launch_bounds__(256) k_tomb_sweep(Tables t) {
+__global__ void __launch_bounds__(256) k_tomb_sweep(Tables t, u32 cls) {
   typedef Lay<G, S> LY;
   const Group<G> g;
-  const u32 nbk = ld_relaxed_u32(&t.ctl->bump);
+  const u32 nbk = ld_relaxed_u32(&t.ctl->bump[cls]);
+  const u32* const pool = by_class(t.pool, cls);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b = gid; b < nbk; b += ng) {
-    const uint4 x = *reinterpret_cast<const uint4*>(t.pool + b * LY::W + 4 * g.gl);
+    const uint4 x = *reinterpret_cast<const uint4*>(pool + b * LY::W + 4 * g.gl);
     bool tomb = false;
 #pragma unroll
     for (int j = 0; j < LY::SPU; ++j) tomb |= LY::has(g.gl, j) && LY::key(x, j) == kTomb;
@@ -167,9 +168,22 @@ __global__ void __launch_bounds__(256) k_tomb_sweep(Tables t) {
 
 cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
+  if (lay & DG_ADAPTIVE_BIT) {  // one sweep per size class pool
+    if (lay & 32) {
+      k_tomb_sweep<2, 1><<<blocks, 256, 0, s>>>(t, 0);
+      k_tomb_sweep<4, 1><<<blocks, 256, 0, s>>>(t, 1);
+      k_tomb_sweep<8, 1><<<blocks, 256, 0, s>>>(t, 2);
+    } else {
+      k_tomb_sweep<2, 0><<<blocks, 256, 0, s>>>(t, 0);
+      k_tomb_sweep<4, 0><<<blocks, 256, 0, s>>>(t, 1);
+      k_tomb_sweep<8, 0><<<blocks, 256, 0, s>>>(t, 2);
+    }
+    note_kernel(3);
+    return cudaGetLastError();
+  }
   switch (lay) {
 #define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_tomb_sweep<G_, S_><<<blocks, 256, 0, s>>>(t); break;
+  case DG_LAY(G_, S_): k_tomb_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, 0); break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
@@ -178,10 +192,10 @@ cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s)
   return cudaGetLastError();
 }
 
-cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u64* nbnew,
-                             u64* nbold, u64* degs, cudaStream_t s) {
+cudaError_t launch_hot_sizes(const Tables& t, u32 n, u32 lf_milli, u32 bc, u32 flush, u32 adaptive,
+                             u32 set, u64* nbnew, u64* nbold, u64* degs, cudaStream_t s) {
   const unsigned blocks = (n + 256) / 256;
-  k_hot_sizes<<<blocks, 256, 0, s>>>(t, n, lf_milli, bc, flush, nbnew, nbold, degs);
+  k_hot_sizes<<<blocks, 256, 0, s>>>(t, n, lf_milli, bc, flush, adaptive, set, nbnew, nbold, degs);
   note_kernel(1);
   return cudaGetLastError();
 }
@@ -191,11 +205,11 @@ cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
                               int sms, cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
   switch (lay) {
-#define DG_CASE(G_, S_)                                                                    \
-  case DG_LAY(G_, S_):                                                                     \
-    k_hot_export<G_, S_><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); \
+#define DG_CASE(G_, S_, A_)                                                                \
+  case DG_LAYA(G_, S_, A_):                                                                \
+    k_hot_export<G_, S_, A_><<<blocks, 256, 0, s>>>(t, n, obo, cursor, osrc, odst, ow, rank); \
     break;
-    DG_FOR_LAYOUTS(DG_CASE)
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
@@ -203,23 +217,20 @@ cudaError_t launch_hot_export(int lay, const Tables& t, u32 n, const u64* obo,
   return cudaGetLastError();
 }
 
-cudaError_t launch_hot_release(int G, const Tables& t, u32 n, const u64* obo, int sms,
+cudaError_t launch_hot_release(int lay, const Tables& t, u32 n, const u64* obo, int sms,
                                cudaStream_t s) {
   const unsigned blocks = (unsigned)sms * 8;
-  switch (G) {
-    case 2: k_hot_release<2><<<blocks, 256, 0, s>>>(t, n, obo); break;
-    case 4: k_hot_release<4><<<blocks, 256, 0, s>>>(t, n, obo); break;
-    case 8: k_hot_release<8><<<blocks, 256, 0, s>>>(t, n, obo); break;
+  if (lay & DG_ADAPTIVE_BIT) {
+    k_hot_release<8, true><<<blocks, 256, 0, s>>>(t, n, obo);
+    note_kernel(1);
+    return cudaGetLastError();
+  }
+  switch (lay & 31) {
+    case 2: k_hot_release<2, false><<<blocks, 256, 0, s>>>(t, n, obo); break;
+    case 4: k_hot_release<4, false><<<blocks, 256, 0, s>>>(t, n, obo); break;
+    case 8: k_hot_release<8, false><<<blocks, 256, 0, s>>>(t, n, obo); break;
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
-  return cudaGetLastError();
-}
-
-cudaError_t launch_hot_install(const Tables& t, u32 n, const u64* nbnew, const u64* nboff,
-                               u32 base0, u32 words, cudaStream_t s) {
-  const unsigned blocks = (n + 255) / 256;
-  k_hot_install<<<blocks, 256, 0, s>>>(t, n, nbnew, nboff, base0, words);
   note_kernel(1);
   return cudaGetLastError();
 }

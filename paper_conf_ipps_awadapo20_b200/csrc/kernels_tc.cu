@@ -150,17 +150,16 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill_big(const u64* ro, const
 // 16-B load per lane per candidate), then decides all G with group ballots.  Warp
 // loops are warp-uniform so every intrinsic uses the full mask.  The rare probes
 // whose key may sit further down a chain are walked by their own lane.
-template <int G, int S>
+template <int G, int S, bool A>
 __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __restrict__ oadj,
                                                       const u32* __restrict__ oend, u64 n_units,
                                                       unsigned long long* count) {
   typedef Lay<G, S> LY;
-  constexpr int W = LY::W;
+  typedef Geo<G, S, A> GEO;
   constexpr u32 FULL = 0xFFFFFFFFu;
   constexpr u32 GBITS = (G == 32) ? 0xFFFFFFFFu : ((1u << G) - 1u);
   constexpr int PER_WARP = 32 / G;
   const Group<G> g;
-  const bool lastl = g.last();
   u32 hits = 0;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
@@ -170,6 +169,9 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
     const u32 v = ev ? __ldg(oadj + e) : 0u;
     const u32 ncand = ev ? __ldg(oend + e) - (u32)e - 1u : 0u;
     const uint2 dv = ev ? ld_nc_dir(t.dir + v) : make_uint2(0, 1);
+    const u32 units = units_of<G, A>(dv.x);  // every probe of the group is into A_v
+    const bool lastl = g.gl == units - 1;
+    const bool inb = g.gl < units;
     const u32 maxc = __reduce_max_sync(FULL, ncand);
     for (u32 k0 = 0; k0 < maxc; k0 += G) {
       const bool act = k0 + g.gl < ncand;
@@ -180,7 +182,7 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
 #pragma unroll
       for (int r = 0; r < G; ++r) {
         const u32 hr = __shfl_sync(FULL, head, g.base + r);
-        if ((amask >> (g.base + r)) & 1u) q[r] = ld_nc_v4(t.pool + (u64)hr * W + 4 * g.gl);
+        if (((amask >> (g.base + r)) & 1u) && inb) q[r] = ld_nc_v4(GEO(t, hr).p + 4 * g.gl);
         else q[r] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
       }
       bool walk = false;
@@ -193,13 +195,13 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
         bool m = false, e = false;
 #pragma unroll
         for (int j = 0; j < LY::SPU; ++j) {
-          const bool h = !lastl || j < LY::SPU / 2;
+          const bool h = inb && (!lastl || j < LY::SPU / 2);
           m |= h && LY::key(x, j) == wr;
           e |= h && LY::key(x, j) == kEmpty;
         }
         const u32 hit = (__ballot_sync(FULL, pr && m) >> g.base) & GBITS;
         const u32 em = (__ballot_sync(FULL, e) >> g.base) & GBITS;
-        const u32 next = __shfl_sync(FULL, x.z, g.base + G - 1);
+        const u32 next = __shfl_sync(FULL, x.z, g.base + units - 1);
         if (pr && g.gl == (u32)r) {
           if (hit) ++hits;
           else if (!em && next != kNil) { walk = true; nxt = next; }
@@ -209,20 +211,22 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
       if (walk) {
         u32 b = nxt;
         while (b != kNil) {
-          const uint4* bp = reinterpret_cast<const uint4*>(t.pool + (u64)b * W);
+          const GEO gb(t, b);
+          const uint4* bp = reinterpret_cast<const uint4*>(gb.p);
           bool found = false, ended = false;
           u32 nb2 = kNil;
 #pragma unroll
           for (int c = 0; c < G; ++c) {
+            if (A && (u32)c >= gb.units) break;
             const uint4 y = __ldg(bp + c);
 #pragma unroll
             for (int j = 0; j < LY::SPU; ++j) {
-              if (LY::has(c, j)) {
+              if (gb.has(c, j)) {
                 found |= LY::key(y, j) == w;
                 ended |= LY::key(y, j) == kEmpty;
               }
             }
-            if (c == G - 1) nb2 = y.z;
+            if ((u32)c == gb.units - 1) nb2 = y.z;
           }
           if (found) { ++hits; break; }
           if (ended) break;
@@ -264,11 +268,11 @@ cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u3
   u64 blocks = (n_units * G + 255) / 256;
   if (blocks > (u64)sms * 4) blocks = (u64)sms * 4;
   switch (lay) {
-#define DG_CASE(G_, S_)                                                                     \
-  case DG_LAY(G_, S_):                                                                      \
-    k_tc_wedges<G_, S_><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); \
+#define DG_CASE(G_, S_, A_)                                                                 \
+  case DG_LAYA(G_, S_, A_):                                                                 \
+    k_tc_wedges<G_, S_, A_><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); \
     break;
-    DG_FOR_LAYOUTS(DG_CASE)
+    DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }

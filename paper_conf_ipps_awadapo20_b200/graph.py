@@ -64,13 +64,18 @@ class Graph:
     ``num_vertices``) sizes each vertex's initial table; ``None`` gives
     every vertex one bucket.  ``set_variant`` stores keys only (twice
     as many per bucket): weights are ignored on insert and read as 0.
+    ``adaptive`` (or ``bucket_bytes=0``) gives each vertex a bucket size (32 / 64 /
+    128 B) chosen from its degree (DG_FLAG_ADAPTIVE).
     """
 
     def __init__(self, num_vertices: int, degree_hints=None, *, load_factor: float = 0.7,
                  bucket_bytes: int = 128, directed: bool = True, pool_bytes: int = 0,
                  device: int | None = None, rank: int = 0, nranks: int = 1,
                  nccl_unique_id: bytes | None = None, reuse_tombstones: bool = True,
-                 force_router: bool = False, set_variant: bool = False, stream=None):
+                 force_router: bool = False, set_variant: bool = False,
+                 adaptive: bool = False, stream=None):
+        if bucket_bytes == 0:
+            adaptive, bucket_bytes = True, 128
         cfg = dg_config()
         lib.dg_config_init(ctypes.byref(cfg))
         cfg.load_factor = float(load_factor)
@@ -84,7 +89,8 @@ class Graph:
         cfg.nranks = int(nranks)
         cfg.flags = (0 if reuse_tombstones else _lib.DG_FLAG_NO_TOMBSTONE_REUSE) | \
             (_lib.DG_FLAG_FORCE_ROUTER if force_router else 0) | \
-            (_lib.DG_FLAG_SET if set_variant else 0)
+            (_lib.DG_FLAG_SET if set_variant else 0) | \
+            (_lib.DG_FLAG_ADAPTIVE if adaptive else 0)
         self._uid = None
         if nccl_unique_id is not None:
             self._uid = ctypes.create_string_buffer(bytes(nccl_unique_id), 128)
@@ -98,6 +104,7 @@ class Graph:
         self.directed = directed
         self.bucket_bytes = bucket_bytes
         self.set_variant = set_variant
+        self.adaptive = adaptive
         self.rank, self.nranks = rank, nranks
         check(lib.dg_create(ctypes.byref(cfg), int(num_vertices), hp, _stream(stream),
                             ctypes.byref(self._h)), "dg_create")

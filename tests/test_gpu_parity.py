@@ -20,6 +20,7 @@ from tests.gpu_util import GpuAdapter, check_against_oracle, check_queries, cuda
 pytestmark = pytest.mark.gpu
 
 GEOMS = [32, 64, 128]
+GEOMS_A = GEOMS + [0]  # 0 = degree-adaptive bucket sizes (DG_FLAG_ADAPTIVE)
 
 
 @pytest.fixture(autouse=True)
@@ -29,7 +30,7 @@ def _dev(cuda_ok):
     torch.cuda.synchronize()
 
 
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 @pytest.mark.parametrize("name", ["edge_ops_directed.txt", "edge_ops_undirected.txt"])
 def test_golden_scripts_on_gpu(name, bb):
     run_script(load(name), lambda n, directed: GpuAdapter(n, directed, bucket_bytes=bb))
@@ -111,24 +112,24 @@ def _config1_stream(bb, hints, directed, seed=1, reuse=True, set_variant=False):
     g.close()
 
 
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 @pytest.mark.parametrize("hints", [False, True])
 def test_config1_directed(bb, hints):
     _config1_stream(bb, hints, True)
 
 
-@pytest.mark.parametrize("bb", [32, 128])
+@pytest.mark.parametrize("bb", [32, 128, 0])
 def test_config1_undirected(bb):
     _config1_stream(bb, False, False, seed=3)
 
 
-@pytest.mark.parametrize("bb", [32, 128])
+@pytest.mark.parametrize("bb", [32, 128, 0])
 def test_config1_append_only(bb):
     """The paper's default policy: tombstones are never reused."""
     _config1_stream(bb, False, True, seed=4, reuse=False)
 
 
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 @pytest.mark.parametrize("directed", [True, False])
 def test_config1_set_variant(bb, directed):
     """Set variant (keys only): the config-1 stream
@@ -187,7 +188,7 @@ def test_churn_tombstone_policy(reuse):
         assert st["tombstones"] >= 6 * 190_000
 
 
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 def test_large_random_ragged(bb):
     """|V| = 100,000; 3 insert batches of 700,001 (ragged tail), queries, deletes."""
     nv = 100_000
@@ -204,7 +205,7 @@ def test_large_random_ragged(bb):
     check_against_oracle(g, o, "deleted")
 
 
-@pytest.mark.parametrize("bb", [32, 128])
+@pytest.mark.parametrize("bb", [32, 128, 0])
 def test_rmat_hubs_without_hints(bb):
     """Scale-free input with one bucket per vertex (Tab. VI-style incremental build):
     long chains, many concurrent chain extensions and same-key races."""
@@ -290,13 +291,14 @@ def test_host_buffers_match_device_buffers():
     assert np.array_equal(ea[0], eb[0].cpu().numpy())
 
 
+@pytest.mark.parametrize("bb", [128, 0])
 @pytest.mark.parametrize("directed", [True, False])
-def test_vertex_deletion_modes(directed):
+def test_vertex_deletion_modes(directed, bb):
     """Directed: streaming purge sweep; undirected: Alg. 2."""
     from paper_conf_ipps_awadapo20_b200 import Graph
     nv = 20_000
     s, d = wl.rmat_edges(8, 0, 200_000, 15, wl.GRAPH500, nv=nv)
-    g = Graph(nv, directed=directed)
+    g = Graph(nv, wl.out_degrees(np.concatenate([s, d]), nv), directed=directed, bucket_bytes=bb)
     o = Oracle(nv, directed)
     g.insert_edges(cuda(s), cuda(d))
     o.insert_edges(s, d)
@@ -335,7 +337,7 @@ def test_geometry_invariance():
     w = (s.astype(np.uint64) * 2654435761 ^ d).astype(np.uint32)  # equal weights for equal keys
     hint = wl.out_degrees(s, nv)
     ref = None
-    for bb in GEOMS:
+    for bb in GEOMS_A:
         for lf in (0.35, 0.7, 2.0):
             for h in (None, hint):
                 g = Graph(nv, h, bucket_bytes=bb, load_factor=lf)
@@ -389,9 +391,10 @@ print("OK", g.stats()["pool_buckets"])
     assert r.returncode == 0 and "OK" in r.stdout, r.stderr[-3000:]
 
 
+@pytest.mark.parametrize("bb", [128, 0])
 @pytest.mark.parametrize("directed", [True, False])
 @pytest.mark.parametrize("exchange", ["fused", "nccl"])
-def test_routed_single_gpu(directed, exchange, monkeypatch):
+def test_routed_single_gpu(directed, exchange, bb, monkeypatch):
     """The multi-GPU batch router (partition -> exchange -> local probe -> answers
     back in caller order) on a 1-rank communicator: results identical to the oracle,
     through the fused partition + window stores (default) and the NCCL exchange.
@@ -400,7 +403,7 @@ def test_routed_single_gpu(directed, exchange, monkeypatch):
     if exchange == "nccl":
         monkeypatch.setenv("DG_ROUTER", "nccl")
     nv = 30_000
-    g = Graph(nv, directed=directed, force_router=True)
+    g = Graph(nv, directed=directed, force_router=True, bucket_bytes=bb)
     assert g.stats()["exchange"] == (2 if exchange == "fused" else 1)
     o = Oracle(nv, directed)
     s, d, w = wl.uniform_edges(17, 1000, 1_300_000, nv)  # > the 2^20-op initial window
@@ -455,7 +458,7 @@ def _golden_triangles():
 
 
 @pytest.mark.parametrize("set_variant", [False, True])
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 def test_tc_golden_and_closed_forms(bb, set_variant):
     import math
     from paper_conf_ipps_awadapo20_b200 import Graph
@@ -471,7 +474,7 @@ def test_tc_golden_and_closed_forms(bb, set_variant):
 
 
 @pytest.mark.parametrize("set_variant", [False, True])
-@pytest.mark.parametrize("bb", GEOMS)
+@pytest.mark.parametrize("bb", GEOMS_A)
 def test_tc_matches_oracle_rmat(bb, set_variant):
     """Hash-intersection TC (GPU) vs the forward algorithm on sorted lists (oracle)
     on a symmetrised R-MAT graph; the part/nparts split sums to the total."""
@@ -522,7 +525,7 @@ def test_host_query_pipeline_large():
     assert np.array_equal(rf, fh[idx]) and np.array_equal(rw, wh[idx])
 
 
-@pytest.mark.parametrize("bb", [32, 128])
+@pytest.mark.parametrize("bb", [32, 128, 0])
 def test_rehash_long_chains_without_hints(bb):
     """Per-vertex re-sizing: an R-MAT graph built
     incrementally with one bucket per vertex grows hub chains; flagged tables are
@@ -550,9 +553,10 @@ def test_rehash_long_chains_without_hints(bb):
     assert st["live_pairs"] == o.num_edges() and st["tombstones"] < 50_000
 
 
+@pytest.mark.parametrize("bb", [128, 0])
 @pytest.mark.parametrize("set_variant", [False, True])
 @pytest.mark.parametrize("hints", [False, True])
-def test_hub_rows_export_stats_tc(hints, set_variant):
+def test_hub_rows_export_stats_tc(hints, set_variant, bb):
     """Hub rows (more than 32 base buckets / 1,024 neighbours) are exported, counted
     and oriented by the block-per-row kernels: a wheel W_n (hub 0 joined to the cycle
     1..n) has exactly n triangles for n >= 4 and 4n directed entries."""
@@ -563,7 +567,7 @@ def test_hub_rows_export_stats_tc(hints, set_variant):
     d = np.concatenate([rim, np.roll(rim, -1)])
     nv = n + 1
     h = wl.out_degrees(np.concatenate([s, d]), nv) if hints else None
-    g = Graph(nv, h, directed=False, set_variant=set_variant)
+    g = Graph(nv, h, directed=False, set_variant=set_variant, bucket_bytes=bb)
     o = Oracle(nv, directed=False)
     g.insert_edges(cuda(s), cuda(d))
     o.insert_edges(s, d)
@@ -618,16 +622,17 @@ def test_async_host_batches():
     g.close()
 
 
+@pytest.mark.parametrize("bb", [64, 0])
 @pytest.mark.parametrize("set_variant", [False, True])
 @pytest.mark.parametrize("reuse", [False, True])
-def test_flush_tombstones(reuse, set_variant):
+def test_flush_tombstones(reuse, set_variant, bb):
     """Tombstone flush: after insert/delete churn the
     tables hold tombstones; flushing rebuilds every such table compactly (several
     rounds: > 65,536 rows carry tombstones), the logical graph is unchanged, no
     tombstone is left and the freed buckets serve later inserts."""
     from paper_conf_ipps_awadapo20_b200 import Graph
     nv = 200_000
-    g = Graph(nv, reuse_tombstones=reuse, set_variant=set_variant, bucket_bytes=64)
+    g = Graph(nv, reuse_tombstones=reuse, set_variant=set_variant, bucket_bytes=bb)
     o = Oracle(nv)
 
     def ow(w):
@@ -649,3 +654,98 @@ def test_flush_tombstones(reuse, set_variant):
     assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, ow(w))[1]
     check_against_oracle(g, o, "inserts after flush")
     g.close()
+
+
+def _class_bytes(h, lf_milli, set_variant):
+    """Bytes of the base table the degree-adaptive layout gives a vertex with hint h
+    (include/dg.h DG_FLAG_ADAPTIVE; reading R-ADAPT): the smallest bucket
+    whose single instance holds h at the load factor — 32 B (3 pairs / 6 keys), 64 B
+    (7 / 14) — else 128-B buckets (15 / 30) by the initial rule."""
+    from oracle import initial_buckets
+    for size in (32, 64):
+        bc = size // 4 - 2 if set_variant else size // 8 - 1
+        if h * 1000 <= lf_milli * bc:
+            return size
+    return 128 * initial_buckets(int(h), lf_milli, 30 if set_variant else 15)
+
+
+@pytest.mark.parametrize("set_variant", [False, True])
+def test_adaptive_size_classes(set_variant):
+    """Degree-adaptive bucket sizes: the base tables
+    of dg_create take exactly the bytes of the size-class rule for every hint, far
+    less than uniform 128-B buckets on a low-degree graph, and a 32-B table overflows
+    into a chained 32-B bucket after its 3 pairs (6 keys)."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    hints = np.array([0, 1, 2, 3, 4, 5, 6, 9, 10, 11, 20, 21, 22, 100, 105, 106, 1000, 20000],
+                     np.uint32)
+    for lf in (0.7, 0.5, 1.0):
+        g = Graph(hints.size, hints, bucket_bytes=0, load_factor=lf, set_variant=set_variant)
+        st = g.stats()
+        want = sum(_class_bytes(int(h), int(round(lf * 1000)), set_variant) for h in hints)
+        assert st["table_bytes"] == want, (lf, st["table_bytes"], want)
+        assert st["overflow_buckets"] == 0
+        g.close()
+    nv = 64
+    g = Graph(nv, bucket_bytes=0, set_variant=set_variant)
+    assert g.stats()["table_bytes"] == 32 * nv
+    bc = 6 if set_variant else 3
+    g.insert_edges(cuda(np.zeros(bc, np.uint32)), cuda(np.arange(1, bc + 1, dtype=np.uint32)))
+    assert g.stats()["overflow_buckets"] == 0
+    g.insert_edges(cuda([0]), cuda([bc + 1]))
+    st = g.stats()
+    assert st["overflow_buckets"] == 1 and st["table_bytes"] == 32 * (nv + 1)
+    g.close()
+
+
+def test_adaptive_promotion_and_memory():
+    """Without hints every vertex starts with one 32-B bucket; the re-sizing pass moves
+    rows whose chains grow to larger size classes (P:L309-313 + P:L947-955).  The graph
+    equals the oracle throughout, chains end short, and the adaptive tables of an
+    R-MAT graph (many low-degree vertices) take fewer bytes than uniform 128-B ones."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    scale = 15
+    nv = 1 << scale
+    g = Graph(nv, bucket_bytes=0)
+    o = Oracle(nv)
+    for b in range(6):
+        s, d = wl.rmat_edges(23, b, 100_000, scale, wl.GRAPH500)
+        w = wl.weights(23, b, s.size)
+        assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+    e = torch.empty(0, dtype=torch.uint32, device="cuda")
+    g.insert_edges(e, e)  # re-sizing runs at the start of an insert batch
+    cand = check_against_oracle(g, o, "adaptive promotion")
+    st = g.stats()
+    assert st["max_chain"] <= 8, st
+    qs, qd, _ = wl.uniform_edges(23, 9, 50_000, nv)
+    check_queries(g, o, qs, qd, cand, "adaptive queries")
+    # same graph from exact hints: adaptive vs uniform 128-B memory
+    ro, dd, _ = g.export()
+    ro, dd = ro.cpu().numpy(), dd.cpu().numpy()
+    src = np.repeat(np.arange(nv, dtype=np.uint32), np.diff(ro).astype(np.int64))
+    hint = wl.out_degrees(src, nv)
+    a = Graph(nv, hint, bucket_bytes=0)
+    u = Graph(nv, hint, bucket_bytes=128)
+    for x in (a, u):
+        x.insert_edges(cuda(src), cuda(dd))
+    sa, su = a.stats(), u.stats()
+    assert sa["live_pairs"] == su["live_pairs"] == o.num_edges()
+    assert sa["table_bytes"] < su["table_bytes"], (sa["table_bytes"], su["table_bytes"])
+    for x in (g, a, u):
+        x.close()
+    # road-like grid (degree <= 4): every table fits one 32-B or 64-B bucket
+    gs, gd = wl.grid_edges(3, 300, 300, 0.6025)
+    nv = 300 * 300
+    hint = wl.out_degrees(gs, nv)
+    a = Graph(nv, hint, bucket_bytes=0)
+    u = Graph(nv, hint, bucket_bytes=128)
+    o = Oracle(nv)
+    o.insert_edges(gs, gd)
+    for x in (a, u):
+        x.insert_edges(cuda(gs), cuda(gd))
+        check_against_oracle(x, o, "grid")
+    sa, su = a.stats(), u.stats()
+    assert sa["overflow_buckets"] == 0
+    assert sa["table_bytes"] == sum(_class_bytes(int(h), 700, False) for h in hint)
+    assert sa["table_bytes"] <= su["table_bytes"] // 2
+    a.close()
+    u.close()
