@@ -94,3 +94,15 @@ def test_product_has_no_oracle_dependency():
             if f.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
                 txt = open(os.path.join(dirpath, f)).read()
                 assert "oracle" not in txt.replace("Oracle-free", ""), f
+
+
+def test_flag_values_match_header():
+    """The binding's DG_FLAG_* constants are the header's (include/dg.h)."""
+    import re
+    from paper_conf_ipps_awadapo20_b200 import _lib
+    hdr = open(os.path.join(ROOT, "include", "dg.h")).read()
+    flags = dict(re.findall(r"#define (DG_FLAG_\w+) (\d+)u", hdr))
+    assert set(flags) == {"DG_FLAG_NO_TOMBSTONE_REUSE", "DG_FLAG_FORCE_ROUTER", "DG_FLAG_SET",
+                          "DG_FLAG_ADAPTIVE"}
+    for k, v in flags.items():
+        assert getattr(_lib, k) == int(v), k
