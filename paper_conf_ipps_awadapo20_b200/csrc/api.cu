@@ -184,7 +184,7 @@ dg_status ensure_dedup(dg_graph g, u64 n) {
 // (adaptive layout) one per op — a lane hands back its spare when the next chain it
 // extends has another size class, which happens at most once per lost link race
 dg_status ensure_ret(dg_graph g, u64 n_ops) {
-  const u64 want = dg::max_groups(g->G, g->sms) + (g->adaptive ? n_ops : 0) + 16;
+  const u64 want = dg::max_groups(g->G, g->sms) + (g->adaptive ? n_ops : 0) + 64;
   if (want > g->ret_cap) {
     if (g->ret_list) DG_CK(cudaFree(g->ret_list));
     g->ret_list = nullptr;
@@ -353,6 +353,14 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
+  static const bool trace_alloc = std::getenv("DG_TRACE_ALLOC") != nullptr;
+  if (trace_alloc) {  // diagnostic: allocator activity of this launch (synchronises)
+    const u32 b0 = g->hctl->bump[0];
+    DG_TRY(read_ctl(g, s));
+    std::fprintf(stderr, "dg: insert %llu ops: pops %u/%u stack, bump %u -> %u, spares back %u\n",
+                 (unsigned long long)n_ops, g->hctl->pop_count[0], g->hctl->stack_size[0], b0,
+                 g->hctl->bump[0], g->hctl->ret_count);
+  }
   DG_CK(dg::launch_fixup_alloc(t, s));
   if (g->hot_steps && !g->in_rehash) {  // chain-length metric, read before the next batch
     DG_CK(cudaMemcpyAsync(g->h_hot, &g->ctl->hot_count, 8, cudaMemcpyDeviceToHost, s));

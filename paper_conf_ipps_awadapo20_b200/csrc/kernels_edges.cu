@@ -83,6 +83,80 @@ __device__ __forceinline__ u32 alloc_bucket_warp(const Tables& t, bool want, u32
   return j < by_class(t.cap, c) ? (c << kClassShift) | j : kNil;
 }
 
+// Per-warp bucket chunks (uniform layouts): a warp takes kChunk consecutive pops of
+// the free stack, or kChunk consecutive bump slots once the stack is exhausted, with
+// ONE atomic, and hands them to its extending lanes over later rounds.  Chain growth
+// is otherwise serialised on the two allocator counters: in the cfg4 R-MAT insert
+// batches (~3% of ops extend a chain) the per-warp-round atomics on one address took
+// a fifth of the kernel's stall samples.  The unused rest of a chunk goes back with
+// the spare buckets at kernel end.  Chunk state lives in shared memory (warp-uniform,
+// touched only when a lane extends): {pos, end, mode (0 = stack, 1 = bump)}.
+constexpr u32 kChunk = 32;
+
+__device__ __forceinline__ u32* warp_chunk() {
+  __shared__ u32 s_chunk[kEdgeBlock / 32][4];
+  return s_chunk[threadIdx.x >> 5];
+}
+
+// Called by the whole warp (uniform layouts); returns a class-0 bucket id (or NIL when
+// the pool is exhausted) for lanes with `want`, NIL for the others.
+__device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u32 ss0) {
+  const u32 lane = threadIdx.x & 31u;
+  const u32 below = (1u << lane) - 1u;
+  u32* sc = warp_chunk();
+  u32 id = kNil;
+  bool need = want;
+  while (true) {
+    const u32 m = __ballot_sync(0xFFFFFFFFu, need);
+    if (m == 0) break;
+    const u32 n = __popc(m), rank = __popc(m & below);
+    const u32 pos = sc[0], end = sc[1], mode = sc[2];
+    const u32 avail = end - pos;
+    const u32 take = n < avail ? n : avail;
+    if (need && rank < take) {
+      const u32 k = pos + rank;
+      id = mode == 0 ? t.stack[0][ss0 - 1 - k] : (k < t.cap[0] ? k : kNil);
+      need = false;
+    }
+    __syncwarp();
+    if (lane == 0) {
+      sc[0] = pos + take;
+      if (n > avail) {  // refill: the chunk is used up
+        bool stack = sc[2] == 0;
+        if (stack) {
+          const u32 i0 = atomicAdd(&t.ctl->pop_count[0], kChunk);
+          if (i0 < ss0) {
+            sc[0] = i0;
+            sc[1] = i0 + kChunk < ss0 ? i0 + kChunk : ss0;
+          } else {
+            stack = false;
+          }
+        }
+        if (!stack) {
+          const u32 b0 = atomicAdd(&t.ctl->bump[0], kChunk);
+          sc[0] = b0;
+          sc[1] = b0 + kChunk;
+          sc[2] = 1;
+        }
+      }
+    }
+    __syncwarp();
+  }
+  return id;
+}
+
+// hand the unused rest of the warp's chunk back (kernel end; whole warp)
+__device__ __forceinline__ void release_chunk(const Tables& t, u32 ss0) {
+  const u32 lane = threadIdx.x & 31u;
+  const u32* sc = warp_chunk();
+  const u32 pos = sc[0], end = sc[1], mode = sc[2];
+  if (lane < end - pos) {
+    const u32 k = pos + lane;
+    const u32 id = mode == 0 ? t.stack[0][ss0 - 1 - k] : (k < t.cap[0] ? k : kNil);
+    if (id != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = id;
+  }
+}
+
 // ------------------------------------------------------------- main kernel ----
 // Per warp iteration (32 ops of the batch):
 //   1. lane L stages op L (coalesced loads) and gathers its directory entry; its
@@ -310,7 +384,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       }
       const bool want = ext && spare == kNil;
       if (__any_sync(FULL, want)) {
-        const u32 got = alloc_bucket_warp<A>(t, want, cls, ss0);
+        const u32 got = A ? alloc_bucket_warp<A>(t, want, cls, ss0) : alloc_bucket_chunk(t, want, ss0);
         if (want) spare = got;
       }
     }
@@ -372,6 +446,12 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
   u32 my_count = 0;
   u32 spare = kNil;  // a fresh bucket this lane allocated but could not link
   bool bad_range = false;
+  if (OP == OP_INSERT && !A && g.lane == 0) {  // empty bucket chunk (alloc_bucket_chunk)
+    u32* sc = warp_chunk();
+    sc[0] = sc[1] = 0;
+    sc[2] = ss0 ? 0u : 1u;
+  }
+  __syncwarp();
   // per-warp backlog of deferred op ids (shared memory)
   __shared__ unsigned long long backlog[kEdgeBlock / 32][64];
   unsigned long long* bl = backlog[threadIdx.x >> 5];
@@ -404,8 +484,12 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     run_ops<G, S, OP, false, A>(t, a, g, valid, op2, op2, ss0, reuse, my_count, spare,
                                 bad_range);
   }
-  // ---- epilogue: hand back an unused spare bucket, reduce the batch counter
+  // ---- epilogue: hand back unused spare buckets, reduce the batch counter
   if (OP == OP_INSERT && spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
+  if (OP == OP_INSERT && !A) {
+    __syncwarp();
+    release_chunk(t, ss0);
+  }
   if (OP == OP_QUERY) {
     if (__any_sync(FULL, bad_range) && g.lane == 0) atomicMax(&t.ctl->fail_epoch, a.epoch);
   } else {
@@ -506,9 +590,11 @@ cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, 
 }
 
 u64 max_groups(int G, int sms) {
-  // upper bound on threads resident in one launch: each may hold one spare bucket
+  // upper bound on the buckets an insert launch takes beyond the ones it links: each
+  // resident thread may hold one spare bucket, each resident warp the unused rest of
+  // a chunk (kChunk - 1)
   (void)G;
-  return (u64)sms * 2048;
+  return (u64)sms * 2048 * 2;
 }
 
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
