@@ -814,8 +814,12 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     const cudaError_t q = cudaEventQuery(g->hot_event);
     if (q == cudaSuccess) {
       g->hot_pending = false;
-      // worth a re-sizing pass: enough pairs to move, or the flag list filling up
-      if (g->h_hot[1] >= 2048 || g->h_hot[0] >= g->hot_cap / 2) DG_TRY(dg::rehash_hot(g, s));
+      // worth a re-sizing pass (it synchronises): flagged pairs reach 1/1024 of the
+      // table slots (at least 2,048), or the flag list is filling up
+      u64 slots = 0;
+      for (int c = 0; c < g->ncls; ++c) slots += g->bump_ub[c] * (g->adaptive ? (4u << c) - 1 : g->BC);
+      const u64 thr = std::max<u64>(2048, slots / 1024);
+      if (g->h_hot[1] >= thr || g->h_hot[0] >= g->hot_cap / 2) DG_TRY(dg::rehash_hot(g, s));
     } else if (q != cudaErrorNotReady) {
       DG_CK(q);
     }

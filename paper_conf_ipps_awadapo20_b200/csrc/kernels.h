@@ -30,6 +30,7 @@ struct EdgeBatch {
   uint8_t* found;     // query
   u32* wout;          // query, nullable
   u32 reuse_tombstones;  // insert: install new keys in the first tombstone
+  u32 chunk;             // insert: buckets per per-warp allocation chunk (set by the launcher)
 };
 
 // `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1

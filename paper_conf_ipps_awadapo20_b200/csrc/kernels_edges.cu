@@ -91,7 +91,7 @@ __device__ __forceinline__ u32 alloc_bucket_warp(const Tables& t, bool want, u32
 // a fifth of the kernel's stall samples.  The unused rest of a chunk goes back with
 // the spare buckets at kernel end.  Chunk state lives in shared memory (warp-uniform,
 // touched only when a lane extends): {pos, end, mode (0 = stack, 1 = bump)}.
-constexpr u32 kChunk = 32;
+constexpr u32 kChunk = 32;  // largest chunk; a launch uses a.chunk (small batches less)
 
 __device__ __forceinline__ u32* warp_chunk() {
   __shared__ u32 s_chunk[kEdgeBlock / 32][4];
@@ -100,7 +100,7 @@ __device__ __forceinline__ u32* warp_chunk() {
 
 // Called by the whole warp (uniform layouts); returns a class-0 bucket id (or NIL when
 // the pool is exhausted) for lanes with `want`, NIL for the others.
-__device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u32 ss0) {
+__device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u32 ss0, u32 chunk) {
   const u32 lane = threadIdx.x & 31u;
   const u32 below = (1u << lane) - 1u;
   u32* sc = warp_chunk();
@@ -124,18 +124,18 @@ __device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u3
       if (n > avail) {  // refill: the chunk is used up
         bool stack = sc[2] == 0;
         if (stack) {
-          const u32 i0 = atomicAdd(&t.ctl->pop_count[0], kChunk);
+          const u32 i0 = atomicAdd(&t.ctl->pop_count[0], chunk);
           if (i0 < ss0) {
             sc[0] = i0;
-            sc[1] = i0 + kChunk < ss0 ? i0 + kChunk : ss0;
+            sc[1] = i0 + chunk < ss0 ? i0 + chunk : ss0;
           } else {
             stack = false;
           }
         }
         if (!stack) {
-          const u32 b0 = atomicAdd(&t.ctl->bump[0], kChunk);
+          const u32 b0 = atomicAdd(&t.ctl->bump[0], chunk);
           sc[0] = b0;
-          sc[1] = b0 + kChunk;
+          sc[1] = b0 + chunk;
           sc[2] = 1;
         }
       }
@@ -384,7 +384,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       }
       const bool want = ext && spare == kNil;
       if (__any_sync(FULL, want)) {
-        const u32 got = A ? alloc_bucket_warp<A>(t, want, cls, ss0) : alloc_bucket_chunk(t, want, ss0);
+        const u32 got = A ? alloc_bucket_warp<A>(t, want, cls, ss0) : alloc_bucket_chunk(t, want, ss0, a.chunk);
         if (want) spare = got;
       }
     }
@@ -530,10 +530,16 @@ __global__ void k_fixup_alloc(Tables t) {
   }
   if (threadIdx.x == 0) s_rc = c->ret_count;
   __syncthreads();
-  for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) {
-    const u32 id = t.ret_list[k];
-    const u32 cl = id >> kClassShift;
-    by_class(t.stack, cl)[atomicAdd(&s_ss[cl], 1u)] = id;
+  if (t.cap[1] == 0) {  // uniform layouts: one class, a straight copy
+    for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) t.stack[0][s_ss[0] + k] = t.ret_list[k];
+    __syncthreads();
+    if (threadIdx.x == 0) s_ss[0] += s_rc;
+  } else {
+    for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) {
+      const u32 id = t.ret_list[k];
+      const u32 cl = id >> kClassShift;
+      by_class(t.stack, cl)[atomicAdd(&s_ss[cl], 1u)] = id;
+    }
   }
   __syncthreads();
   if (threadIdx.x < kClasses) {
@@ -565,7 +571,12 @@ static cudaError_t launch_g(const Tables& t, const EdgeBatch& a, int sms, cudaSt
   u64 blocks = (warps_needed + per_block - 1) / per_block;
   const u64 maxb = (u64)sms * grid_for<G, S, OP, A>();
   if (blocks > maxb) blocks = maxb;
-  k_edges<G, S, OP, A><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, a); note_kernel(1);
+  // bucket chunk per warp: ~1/4 of the ops a warp handles, 1..kChunk (a small batch
+  // would otherwise strand most of every chunk)
+  const u64 per_warp = a.n_ops / (blocks * per_block);
+  EdgeBatch ab = a;
+  ab.chunk = (u32)(per_warp / 4 < 1 ? 1 : per_warp / 4 > kChunk ? kChunk : per_warp / 4);
+  k_edges<G, S, OP, A><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, ab); note_kernel(1);
   return cudaGetLastError();
 }
 
