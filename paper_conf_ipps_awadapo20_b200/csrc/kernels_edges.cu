@@ -40,18 +40,9 @@ enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 // ----------------------------------------------------------- allocator (a8) ----
 // Phase-concurrent free stack + bump cursor: during an insert
 // phase buckets are only popped, during a vertex-deletion phase only pushed, so
-// a single cursor per direction is ABA-free.
-// Size class c (uniform layouts: 0); returns a bucket id of class c or NIL.
-// ss0 = class-0 stack size read at kernel start (uniform layouts); the adaptive layout
-// reads its class's size here (stack sizes are fixed during an insert phase).
-template <bool A>
-__device__ __forceinline__ u32 alloc_bucket(const Tables& t, u32 c, u32 ss0) {
-  const u32 stack_size = A ? ld_relaxed_u32(&t.ctl->stack_size[c]) : ss0;
-  u32 i = atomicAdd(&t.ctl->pop_count[c], 1u);
-  if (i < stack_size) return by_class(t.stack, c)[stack_size - 1 - i];
-  u32 j = atomicAdd(&t.ctl->bump[c], 1u);
-  return j < by_class(t.cap, c) ? (c << kClassShift) | j : kNil;
-}
+// a single cursor per direction is ABA-free.  Pops take stack entries from the top
+// (index stack_size - 1 - i for the i-th pop); past the stack, buckets come from the
+// bump cursor.  Stack sizes are fixed during an insert phase.
 
 // Warp-aggregated allocation: the lanes that need a bucket of the same class take
 // consecutive pops (one atomic per class per warp instead of one per lane; a hot
@@ -416,6 +407,22 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
   return deferred;
 }
 
+#ifndef DG_QUERY_PREFETCH
+#define DG_QUERY_PREFETCH 1
+#endif
+#ifndef DG_DELETE_PREFETCH
+#define DG_DELETE_PREFETCH 0
+#endif
+#ifndef DG_INSERT_PREFETCH
+#define DG_INSERT_PREFETCH 0
+#endif
+template <int OP>
+struct Prefetch {
+  static constexpr bool on = OP == OP_QUERY    ? DG_QUERY_PREFETCH != 0
+                             : OP == OP_DELETE ? DG_DELETE_PREFETCH != 0
+                                               : DG_INSERT_PREFETCH != 0;
+};
+
 // resident blocks per SM the register allocation targets (measured on B200, cfg2
 // 2^24 batches: insert 1.41 -> 1.35 ms and query 0.625 -> 0.603 ms at 3 blocks of
 // 256 threads, 85 registers, no spills; delete is faster at 4: 1.07 vs 1.12 ms)
@@ -461,8 +468,15 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
     const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
+    // load the NEXT chunk's sources now and prefetch their directory entries into L2
+    // after this chunk is probed, so the next chunk's directory gather (a DRAM miss:
+    // the bucket stream evicts the directory) overlaps this chunk's probe
+    const u64 nj = j + (u64)nwarps * 32;
+    const bool pf = Prefetch<OP>::on && !a.idx && nj < a.n_ops;
+    const u32 nsrc = pf ? (nj < a.n ? __ldg(a.src + nj) : __ldg(a.dst + (nj - a.n))) : 0u;
     const bool d = run_ops<G, S, OP, true, A>(t, a, g, valid, opid, j, ss0, reuse, my_count, spare,
                                            bad_range);
+    if (pf && (u64)nsrc < a.nv) prefetch_l2(t.dir + (t.nranks == 1 ? nsrc : nsrc / t.nranks));
     const u32 dm = __ballot_sync(FULL, d);
     if (d) bl[nbl + __popc(dm & below)] = OP == OP_QUERY ? j : opid;
     nbl += __popc(dm);
