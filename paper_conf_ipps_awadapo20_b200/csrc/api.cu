@@ -336,7 +336,15 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
     DG_CK(cudaEventSynchronize(g->snap_event));
   }
   DG_TRY(plan_capacity(g, need, s, &retry_mode));
-  DG_TRY(ensure_retry(g, 0, n_ops));
+  // Retry mode records the ops that found no bucket, up to a bounded list (128 MB);
+  // when more fail, the whole batch runs again after the pool grows (an insert batch
+  // is idempotent: re-applied keys are replaced by a weight of the same batch, Q1,
+  // and only keys still missing count as added).
+  static const u64 retry_cap_max = std::getenv("DG_TEST_RETRY_CAP")
+                                       ? std::strtoull(std::getenv("DG_TEST_RETRY_CAP"), nullptr, 10)
+                                       : (1ull << 24);
+  const u64 rcap = retry_mode ? std::min<u64>(n_ops, retry_cap_max) : 0;
+  if (rcap) DG_TRY(ensure_retry(g, 0, rcap));
   DG_TRY(ensure_ret(g, n_ops));
   t = g->tables();
   dg::EdgeBatch a{};
@@ -347,6 +355,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   a.idx = nullptr;
   a.n_ops = n_ops;
   a.retry_out = g->retry[0];
+  a.retry_cap = rcap;
   a.reuse_tombstones = g->reuse_tombstones ? 1u : 0u;
   a.epoch = epoch;
   a.nv = g->nv;
@@ -384,12 +393,15 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
       const u64 want = (u64)g->cap[c] + failed + dg::max_groups(g->G, g->sms) + (u64)g->cap[c] / 4;
       DG_TRY(grow_pool(g, c, want, s));
     }
-    DG_TRY(ensure_retry(g, cur ^ 1, failed));
+    const bool whole = failed > a.retry_cap;  // the list overflowed: run the batch again
+    const u64 next_cap = std::min<u64>(whole ? n_ops : failed, rcap);
+    DG_TRY(ensure_retry(g, cur ^ 1, next_cap));
     DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, sizeof(u32), s));
     t = g->tables();
-    a.idx = g->retry[cur];
-    a.n_ops = failed;
+    a.idx = whole ? nullptr : g->retry[cur];
+    a.n_ops = whole ? n_ops : failed;
     a.retry_out = g->retry[cur ^ 1];
+    a.retry_cap = next_cap;
     DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
     DG_CK(dg::launch_fixup_alloc(t, s));
     cur ^= 1;

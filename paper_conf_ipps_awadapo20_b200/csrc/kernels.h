@@ -24,7 +24,8 @@ struct EdgeBatch {
   u64 n;              // entries in src/dst/w
   const u64* idx;     // nullable: op ids to process (retry list)
   u64 n_ops;          // ops to process (n, 2n for undirected mirror, or |idx|)
-  u64* retry_out;     // insert: op ids that found no free bucket
+  u64* retry_out;     // insert: op ids that found no free bucket (first retry_cap of them)
+  u64 retry_cap;      // capacity of retry_out (0: the launch cannot run out of buckets)
   u32 epoch;          // batch epoch (validation)
   u64 nv;             // global vertex capacity (query range check)
   uint8_t* found;     // query

@@ -381,7 +381,8 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
     }
     if (OP == OP_INSERT && act == ACT_EXTEND) {
       if (spare == kNil) {  // pool exhausted: the host grows it and re-runs this op
-        a.retry_out[atomicAdd(&t.ctl->retry_count, 1u)] = opid;
+        const u32 k = atomicAdd(&t.ctl->retry_count, 1u);
+        if (k < a.retry_cap) a.retry_out[k] = opid;
         pend = false;
       } else {
         const GEO gs(t, spare), gc(t, cur);
@@ -408,7 +409,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
 }
 
 #ifndef DG_QUERY_PREFETCH
-#define DG_QUERY_PREFETCH 1
+#define DG_QUERY_PREFETCH 0
 #endif
 #ifndef DG_DELETE_PREFETCH
 #define DG_DELETE_PREFETCH 0
@@ -468,9 +469,11 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
     const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
-    // load the NEXT chunk's sources now and prefetch their directory entries into L2
-    // after this chunk is probed, so the next chunk's directory gather (a DRAM miss:
-    // the bucket stream evicts the directory) overlaps this chunk's probe
+    // (off by default) load the NEXT chunk's sources now and prefetch their directory
+    // entries into L2 after this chunk is probed, so the next chunk's directory gather
+    // overlaps this chunk's probe.  Measured on cfg2: query 0.603 -> 0.658 ms, insert +
+    // delete with it as well 1.20/1.07 -> 1.24/1.18 ms: the extra request per op costs
+    // more than the latency it hides.
     const u64 nj = j + (u64)nwarps * 32;
     const bool pf = Prefetch<OP>::on && !a.idx && nj < a.n_ops;
     const u32 nsrc = pf ? (nj < a.n ? __ldg(a.src + nj) : __ldg(a.dst + (nj - a.n))) : 0u;

@@ -52,10 +52,10 @@ def _rows_equal(g_export, o, rows, where):
     return cand
 
 
-def _run_config(nv, bs, bd, bw, B, seed, sample_frac=1 / 256):
+def _run_config(nv, bs, bd, bw, B, seed, sample_frac=1 / 256, bucket_bytes=128):
     from paper_conf_ipps_awadapo20_b200 import Graph
     hints = torch.bincount(_cu(bs.astype(np.int64)), minlength=nv).to(torch.int32)
-    g = Graph(nv, hints)
+    g = Graph(nv, hints, bucket_bytes=bucket_bytes)
     added = g.insert_edges(_cu(bs), _cu(bd), _cu(bw), count=True)
     distinct = _distinct_nonloop(bs, bd)
     assert added == distinct
@@ -103,12 +103,14 @@ def test_config2_fullsize_sampled():
     g.close()
 
 
-def test_config3_fullsize_sampled():
-    """Road-like grid 4,894 x 4,894 (23,951,236 V, 57.7M directed edges)."""
+@pytest.mark.parametrize("bb", [128, 0])
+def test_config3_fullsize_sampled(bb):
+    """Road-like grid 4,894 x 4,894 (23,951,236 V, 57.7M directed edges); uniform
+    128-B buckets and the degree-adaptive layout (bb = 0)."""
     bs, bd = wl.grid_edges(3, 4894, 4894, 0.6025)
     nv = 4894 * 4894
     bw = wl.weights(3, 0, bs.size)
-    g, o, R, inR = _run_config(nv, bs, bd, bw, 1 << 22, 3)
+    g, o, R, inR = _run_config(nv, bs, bd, bw, 1 << 22, 3, bucket_bytes=bb)
     g.close()
 
 

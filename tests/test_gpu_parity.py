@@ -366,9 +366,11 @@ def test_initial_bucket_rule_matches_oracle():
             assert g.stats()["base_buckets"] == want
 
 
-def test_pool_exhaustion_retry_path():
+@pytest.mark.parametrize("retry_cap", [None, 1000])
+def test_pool_exhaustion_retry_path(retry_cap):
     """Pool exhaustion mid-kernel: failed ops are re-run after the pool grows
-    (forced with DG_TEST_RETRY_PATH, which disables up-front growth)."""
+    (forced with DG_TEST_RETRY_PATH, which disables up-front growth).  With a retry
+    list smaller than the failures (DG_TEST_RETRY_CAP) the whole batch runs again."""
     code = r"""
 import numpy as np, torch, sys
 sys.path.insert(0, %r)
@@ -386,6 +388,8 @@ check_against_oracle(g, o, "retry")
 print("OK", g.stats()["pool_buckets"])
 """ % os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
     env = dict(os.environ, DG_TEST_RETRY_PATH="1")
+    if retry_cap:
+        env["DG_TEST_RETRY_CAP"] = str(retry_cap)
     r = subprocess.run([sys.executable, "-c", code], env=env, capture_output=True, text=True,
                        timeout=600)
     assert r.returncode == 0 and "OK" in r.stdout, r.stderr[-3000:]
