@@ -12,7 +12,7 @@ for row in rows:
     name = row[hdr.index('Kernel Name')]
     if 'k_edges' not in name:
         continue
-    op = ops[name.split('<')[1].split('>')[0].split(',')[-1].strip()]
+    op = ops[name.split('<')[1].split('>')[0].split(',')[2].strip()]  # <G, S, OP, A>
     b = 0.0
     for m in ('dram__bytes_read.sum', 'dram__bytes_write.sum'):
         i = hdr.index(m)
