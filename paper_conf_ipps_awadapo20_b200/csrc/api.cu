@@ -184,7 +184,8 @@ dg_status ensure_dedup(dg_graph g, u64 n) {
 // (adaptive layout) one per op — a lane hands back its spare when the next chain it
 // extends has another size class, which happens at most once per lost link race
 dg_status ensure_ret(dg_graph g, u64 n_ops) {
-  const u64 want = dg::max_groups(g->G, g->sms) + (g->adaptive ? n_ops : 0) + 64;
+  // (adaptive: chunk remainders of three classes per warp)
+  const u64 want = dg::max_groups(g->G, g->sms) * (g->adaptive ? 2 : 1) + (g->adaptive ? n_ops : 0) + 64;
   if (want > g->ret_cap) {
     if (g->ret_list) DG_CK(cudaFree(g->ret_list));
     g->ret_list = nullptr;

@@ -44,87 +44,79 @@ enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 // (index stack_size - 1 - i for the i-th pop); past the stack, buckets come from the
 // bump cursor.  Stack sizes are fixed during an insert phase.
 
-// Warp-aggregated allocation: the lanes that need a bucket of the same class take
-// consecutive pops (one atomic per class per warp instead of one per lane; a hot
-// single-address atomic otherwise serialises chain growth), and the ones past the
-// free stack consecutive bump slots.  Called by the whole warp; returns NIL for lanes
-// with !want.
-template <bool A>
-__device__ __forceinline__ u32 alloc_bucket_warp(const Tables& t, bool want, u32 c, u32 ss0) {
-  const u32 lane = threadIdx.x & 31u;
-  const u32 below = (1u << lane) - 1u;
-  const u32 peers = __match_any_sync(0xFFFFFFFFu, want ? c : 0xFFFFFFFFu);
-  if (!want) return kNil;
-  const u32 leader = __ffs(peers) - 1;
-  u32 base = 0, ss = 0;
-  if (lane == leader) {
-    ss = A ? ld_relaxed_u32(&t.ctl->stack_size[c]) : ss0;  // fixed during the phase
-    base = atomicAdd(&t.ctl->pop_count[c], (u32)__popc(peers));
-  }
-  base = __shfl_sync(peers, base, leader);
-  ss = __shfl_sync(peers, ss, leader);
-  const u32 i = base + __popc(peers & below);
-  const bool from_stack = i < ss;
-  const u32 over = __ballot_sync(peers, !from_stack);
-  if (from_stack) return by_class(t.stack, c)[ss - 1 - i];
-  const u32 l2 = __ffs(over) - 1;
-  u32 b = 0;
-  if (lane == l2) b = atomicAdd(&t.ctl->bump[c], (u32)__popc(over));
-  const u32 j = __shfl_sync(over, b, l2) + __popc(over & below);
-  return j < by_class(t.cap, c) ? (c << kClassShift) | j : kNil;
-}
-
-// Per-warp bucket chunks (uniform layouts): a warp takes kChunk consecutive pops of
-// the free stack, or kChunk consecutive bump slots once the stack is exhausted, with
-// ONE atomic, and hands them to its extending lanes over later rounds.  Chain growth
-// is otherwise serialised on the two allocator counters: in the cfg4 R-MAT insert
-// batches (~3% of ops extend a chain) the per-warp-round atomics on one address took
-// a fifth of the kernel's stall samples.  The unused rest of a chunk goes back with
-// the spare buckets at kernel end.  Chunk state lives in shared memory (warp-uniform,
-// touched only when a lane extends): {pos, end, mode (0 = stack, 1 = bump)}.
+// Per-warp bucket chunks: a warp takes `chunk` consecutive pops of a class's free
+// stack (or, once the stack is exhausted, `chunk` consecutive bump slots) with ONE
+// atomic and hands them to its extending lanes over later rounds.  Chain growth is
+// otherwise serialised on the two allocator counters of the class: in the cfg4 R-MAT
+// insert batches (~3% of ops extend a chain) per-warp-round atomics on one address
+// took a fifth of the kernel's stall samples.  The unused rest of every chunk goes
+// back with the spare buckets at kernel end.  Chunk state lives in shared memory
+// (warp-uniform, touched only when a lane extends), per size class:
+// {pos, end, mode (0 = stack, 1 = bump), stack size at kernel start}.
 constexpr u32 kChunk = 32;  // largest chunk; a launch uses a.chunk (small batches less)
 
-__device__ __forceinline__ u32* warp_chunk() {
-  __shared__ u32 s_chunk[kEdgeBlock / 32][4];
-  return s_chunk[threadIdx.x >> 5];
+__device__ __forceinline__ u32* warp_chunk(u32 c) {
+  __shared__ u32 s_chunk[kEdgeBlock / 32][kClasses][4];
+  return s_chunk[threadIdx.x >> 5][c];
 }
 
-// Called by the whole warp (uniform layouts); returns a class-0 bucket id (or NIL when
-// the pool is exhausted) for lanes with `want`, NIL for the others.
-__device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u32 ss0, u32 chunk) {
+// lane 0 of each warp, at kernel start (stack sizes are fixed during an insert phase)
+template <bool A>
+__device__ __forceinline__ void init_chunks(const Tables& t) {
+  for (u32 c = 0; c < (A ? (u32)kClasses : 1u); ++c) {
+    u32* sc = warp_chunk(c);
+    const u32 ss = ld_relaxed_u32(&t.ctl->stack_size[c]);
+    sc[0] = sc[1] = 0;
+    sc[2] = ss ? 0u : 1u;
+    sc[3] = ss;
+  }
+}
+
+__device__ __forceinline__ u32 chunk_id(const Tables& t, u32 c, u32 mode, u32 ss, u32 k) {
+  if (mode == 0) return by_class(t.stack, c)[ss - 1 - k];
+  return k < by_class(t.cap, c) ? (c << kClassShift) | k : kNil;
+}
+
+// Called by the whole warp; returns a bucket id of class c (NIL when the pool is
+// exhausted) for lanes with `want`, NIL for the others.
+template <bool A>
+__device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u32 c, u32 chunk) {
   const u32 lane = threadIdx.x & 31u;
   const u32 below = (1u << lane) - 1u;
-  u32* sc = warp_chunk();
   u32 id = kNil;
   bool need = want;
   while (true) {
-    const u32 m = __ballot_sync(0xFFFFFFFFu, need);
-    if (m == 0) break;
+    const u32 nm = __ballot_sync(0xFFFFFFFFu, need);
+    if (nm == 0) break;
+    // serve the lanes of one class per pass (uniform layouts: class 0 only)
+    const u32 cc = A ? __shfl_sync(0xFFFFFFFFu, c, __ffs(nm) - 1) : 0u;
+    const bool mine = need && (!A || c == cc);
+    const u32 m = A ? __ballot_sync(0xFFFFFFFFu, mine) : nm;
+    u32* sc = warp_chunk(cc);
     const u32 n = __popc(m), rank = __popc(m & below);
-    const u32 pos = sc[0], end = sc[1], mode = sc[2];
+    const u32 pos = sc[0], end = sc[1], mode = sc[2], ss = sc[3];
     const u32 avail = end - pos;
     const u32 take = n < avail ? n : avail;
-    if (need && rank < take) {
-      const u32 k = pos + rank;
-      id = mode == 0 ? t.stack[0][ss0 - 1 - k] : (k < t.cap[0] ? k : kNil);
+    if (mine && rank < take) {
+      id = chunk_id(t, cc, mode, ss, pos + rank);
       need = false;
     }
     __syncwarp();
     if (lane == 0) {
       sc[0] = pos + take;
       if (n > avail) {  // refill: the chunk is used up
-        bool stack = sc[2] == 0;
+        bool stack = mode == 0;
         if (stack) {
-          const u32 i0 = atomicAdd(&t.ctl->pop_count[0], chunk);
-          if (i0 < ss0) {
+          const u32 i0 = atomicAdd(&t.ctl->pop_count[cc], chunk);
+          if (i0 < ss) {
             sc[0] = i0;
-            sc[1] = i0 + chunk < ss0 ? i0 + chunk : ss0;
+            sc[1] = i0 + chunk < ss ? i0 + chunk : ss;
           } else {
             stack = false;
           }
         }
         if (!stack) {
-          const u32 b0 = atomicAdd(&t.ctl->bump[0], chunk);
+          const u32 b0 = atomicAdd(&t.ctl->bump[cc], chunk);
           sc[0] = b0;
           sc[1] = b0 + chunk;
           sc[2] = 1;
@@ -136,15 +128,17 @@ __device__ __forceinline__ u32 alloc_bucket_chunk(const Tables& t, bool want, u3
   return id;
 }
 
-// hand the unused rest of the warp's chunk back (kernel end; whole warp)
-__device__ __forceinline__ void release_chunk(const Tables& t, u32 ss0) {
+// hand the unused rest of the warp's chunks back (kernel end; whole warp)
+template <bool A>
+__device__ __forceinline__ void release_chunks(const Tables& t) {
   const u32 lane = threadIdx.x & 31u;
-  const u32* sc = warp_chunk();
-  const u32 pos = sc[0], end = sc[1], mode = sc[2];
-  if (lane < end - pos) {
-    const u32 k = pos + lane;
-    const u32 id = mode == 0 ? t.stack[0][ss0 - 1 - k] : (k < t.cap[0] ? k : kNil);
-    if (id != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = id;
+  for (u32 c = 0; c < (A ? (u32)kClasses : 1u); ++c) {
+    const u32* sc = warp_chunk(c);
+    const u32 pos = sc[0], end = sc[1], mode = sc[2], ss = sc[3];
+    for (u32 k = pos + lane; k < end; k += 32) {
+      const u32 id = chunk_id(t, c, mode, ss, k);
+      if (id != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = id;
+    }
   }
 }
 
@@ -194,8 +188,7 @@ struct Lanes {
 template <int G, int S, int OP, bool MAIN, bool A>
 __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
                                         const Group<Lanes<G, OP>::L>& g, const bool valid,
-                                        const u64 opid, const u64 j, const u32 ss0,
-                                        const bool reuse, u32& my_count, u32& spare,
+                                        const u64 opid, const u64 j, const bool reuse, u32& my_count, u32& spare,
                                         bool& bad_range) {
   typedef Lay<G, S> LY;
   typedef Geo<G, S, A> GEO;
@@ -375,7 +368,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       }
       const bool want = ext && spare == kNil;
       if (__any_sync(FULL, want)) {
-        const u32 got = A ? alloc_bucket_warp<A>(t, want, cls, ss0) : alloc_bucket_chunk(t, want, ss0, a.chunk);
+        const u32 got = alloc_bucket_chunk<A>(t, want, cls, a.chunk);
         if (want) spare = got;
       }
     }
@@ -448,17 +441,12 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
   }
   const bool reuse = a.reuse_tombstones != 0;
-  const u32 ss0 = (OP == OP_INSERT && !A) ? ld_relaxed_u32(&t.ctl->stack_size[0]) : 0u;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
   u32 my_count = 0;
   u32 spare = kNil;  // a fresh bucket this lane allocated but could not link
   bool bad_range = false;
-  if (OP == OP_INSERT && !A && g.lane == 0) {  // empty bucket chunk (alloc_bucket_chunk)
-    u32* sc = warp_chunk();
-    sc[0] = sc[1] = 0;
-    sc[2] = ss0 ? 0u : 1u;
-  }
+  if (OP == OP_INSERT && g.lane == 0) init_chunks<A>(t);  // empty bucket chunks
   __syncwarp();
   // per-warp backlog of deferred op ids (shared memory)
   __shared__ unsigned long long backlog[kEdgeBlock / 32][64];
@@ -477,7 +465,7 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const u64 nj = j + (u64)nwarps * 32;
     const bool pf = Prefetch<OP>::on && !a.idx && nj < a.n_ops;
     const u32 nsrc = pf ? (nj < a.n ? __ldg(a.src + nj) : __ldg(a.dst + (nj - a.n))) : 0u;
-    const bool d = run_ops<G, S, OP, true, A>(t, a, g, valid, opid, j, ss0, reuse, my_count, spare,
+    const bool d = run_ops<G, S, OP, true, A>(t, a, g, valid, opid, j, reuse, my_count, spare,
                                            bad_range);
     if (pf && (u64)nsrc < a.nv) prefetch_l2(t.dir + (t.nranks == 1 ? nsrc : nsrc / t.nranks));
     const u32 dm = __ballot_sync(FULL, d);
@@ -488,7 +476,7 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
       nbl -= 32;
       const u64 op2 = bl[nbl + g.lane];
       __syncwarp();
-      run_ops<G, S, OP, false, A>(t, a, g, true, op2, op2, ss0, reuse, my_count, spare,
+      run_ops<G, S, OP, false, A>(t, a, g, true, op2, op2, reuse, my_count, spare,
                                   bad_range);
     }
   }
@@ -498,14 +486,14 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     const bool valid = g.lane < take;
     const u64 op2 = valid ? bl[nbl + g.lane] : 0;
     __syncwarp();
-    run_ops<G, S, OP, false, A>(t, a, g, valid, op2, op2, ss0, reuse, my_count, spare,
+    run_ops<G, S, OP, false, A>(t, a, g, valid, op2, op2, reuse, my_count, spare,
                                 bad_range);
   }
   // ---- epilogue: hand back unused spare buckets, reduce the batch counter
   if (OP == OP_INSERT && spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
-  if (OP == OP_INSERT && !A) {
+  if (OP == OP_INSERT) {
     __syncwarp();
-    release_chunk(t, ss0);
+    release_chunks<A>(t);
   }
   if (OP == OP_QUERY) {
     if (__any_sync(FULL, bad_range) && g.lane == 0) atomicMax(&t.ctl->fail_epoch, a.epoch);
