@@ -293,6 +293,14 @@ dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) 
     // pops come from the stack first; the bump cursor moves by at most need - stack
     if (free_exact >= need) continue;
     const u64 missing = need - free_exact;
+    // Adaptive layout: the worst case (every op extends a chain) applies to each of
+    // the three pools but can only happen in one of them, so reserving it everywhere
+    // would map ~3x the memory; such a batch runs in retry mode instead (one
+    // synchronisation; pools grow by what actually failed).
+    if (g->ncls > 1 && missing > std::max<u64>(g->cap[c] / 4, 1u << 20)) {
+      *retry_mode = true;
+      continue;
+    }
     if (!limit) limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
     if (!no_upfront && missing * g->cbytes(c) <= limit) {
       const u64 want = (u64)g->cap[c] + missing + std::max<u64>(missing / 4, 65536);
@@ -395,6 +403,9 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
       DG_TRY(grow_pool(g, c, want, s));
     }
     const bool whole = failed > a.retry_cap;  // the list overflowed: run the batch again
+    if (std::getenv("DG_DEBUG"))
+      std::fprintf(stderr, "dg: retry round %d: %llu ops found no bucket%s\n", round,
+                   (unsigned long long)failed, whole ? " (whole batch again)" : "");
     const u64 next_cap = std::min<u64>(whole ? n_ops : failed, rcap);
     DG_TRY(ensure_retry(g, cur ^ 1, next_cap));
     DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, sizeof(u32), s));

@@ -6,9 +6,13 @@ import numpy as np, torch
 import workloads as wl
 from paper_conf_ipps_awadapo20_b200 import Graph
 
-nv, m = 4_847_571, 68_993_773
 adaptive = os.environ.get("ADAPTIVE", "0") == "1"
-s, d = wl.rmat_edges(2, 0, m, 23, wl.LJLIKE, nv=nv)
+if os.environ.get("CFG", "cfg2") == "cfg3":
+    s, d = wl.grid_edges(3, 4894, 4894, 0.6025)
+    nv, m = 4894 * 4894, s.size
+else:
+    nv, m = 4_847_571, 68_993_773
+    s, d = wl.rmat_edges(2, 0, m, 23, wl.LJLIKE, nv=nv)
 w = wl.weights(2, 0, m)
 dev = torch.device("cuda", 0)
 hints = torch.bincount(torch.from_numpy(s.astype(np.int64)).to(dev), minlength=nv).to(torch.int32)
