@@ -470,7 +470,10 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
                                                     u32 epoch, u32 cls) {
   typedef Lay<G, S> LY;
   constexpr int W = LY::W;
-  constexpr int U = 4;  // buckets in flight per group (memory-level parallelism)
+#ifndef DG_SWEEP_U
+#define DG_SWEEP_U 4
+#endif
+  constexpr int U = DG_SWEEP_U;  // buckets in flight per group (memory-level parallelism)
   __shared__ u32 sf[kVdelFilterBits / 32];
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
@@ -485,8 +488,13 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const u64 b = b0 + (u64)k * ng;
+#ifdef DG_SWEEP_LDCS
+      q[k] = b < nbk ? __ldcs(reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl))
+                     : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+#else
       q[k] = b < nbk ? *reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl)
                      : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+#endif
     }
 #pragma unroll
     for (int k = 0; k < U; ++k) {
