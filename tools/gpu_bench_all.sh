@@ -14,7 +14,7 @@ nvcc -gencode arch=compute_100a,code=sm_100a -O3 -o /tmp/gc tools/gather_ceiling
 timeout 1200 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file $D/launches_bench_cfg2.csv \
    python bench.py --steps 3 --warmup 3 > $D/ncu_launches_bench.log 2>&1
 timeout 1200 ncu --set full --clock-control none --import-source on -k regex:k_edges --launch-skip 4 --launch-count 3 \
-   -o $D/k_edges_cfg2 -f python bench.py --steps 1 --warmup 0 --no-e2e --no-vdel --no-cpu-baseline > $D/ncu_full.log 2>&1
+   -o $D/k_edges_cfg2 -f python bench.py --steps 1 --warmup 0 --no-e2e --no-vdel --no-cpu-baseline --no-sorted-build > $D/ncu_full.log 2>&1
 timeout 1200 ncu --set full --clock-control none --import-source on -k regex:k_edges --launch-skip 1 --launch-count 1 \
    -o $D/k_edges_cfg4_insert -f python bench.py --config cfg4 --steps 1 --warmup 3 --no-cpu-baseline --no-e2e > $D/ncu_full_cfg4.log 2>&1
 for f in $D/*.err; do echo "== $f"; tail -n 2 $f; done
