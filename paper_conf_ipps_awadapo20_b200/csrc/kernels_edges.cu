@@ -524,7 +524,19 @@ __global__ void k_validate(const u32* __restrict__ src, const u32* __restrict__ 
 // After an insert phase: drop the popped entries from each class's free stack,
 // clamp the bump cursors, and push the spare buckets that were handed back onto the
 // stack of their class.
-__global__ void k_fixup_alloc(Tables t) {
+// Uniform layouts: the returned buckets go back onto the stack with a grid-wide
+// copy (tens of thousands of chunk remainders per large batch took a single block
+// ~0.1 ms); k_fixup_alloc then only moves the cursors.
+__global__ void k_fixup_copy(Tables t) {
+  const DevCtl* c = t.ctl;
+  const u32 pc = c->pop_count[0], ss = c->stack_size[0], rc = c->ret_count;
+  const u32 base = pc >= ss ? 0u : ss - pc;
+  const u32 stride = gridDim.x * blockDim.x;
+  for (u32 k = blockIdx.x * blockDim.x + threadIdx.x; k < rc; k += stride)
+    t.stack[0][base + k] = t.ret_list[k];
+}
+
+__global__ void k_fixup_alloc(Tables t, bool copied) {
   __shared__ u32 s_ss[kClasses], s_rc;
   DevCtl* c = t.ctl;
   if (threadIdx.x < kClasses) {
@@ -535,9 +547,7 @@ __global__ void k_fixup_alloc(Tables t) {
   }
   if (threadIdx.x == 0) s_rc = c->ret_count;
   __syncthreads();
-  if (t.cap[1] == 0) {  // uniform layouts: one class, a straight copy
-    for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) t.stack[0][s_ss[0] + k] = t.ret_list[k];
-    __syncthreads();
+  if (copied) {  // uniform layouts: k_fixup_copy already pushed them
     if (threadIdx.x == 0) s_ss[0] += s_rc;
   } else {
     for (u32 k = threadIdx.x; k < s_rc; k += blockDim.x) {
@@ -623,7 +633,12 @@ cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 e
 }
 
 cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s) {
-  k_fixup_alloc<<<1, 256, 0, s>>>(t); note_kernel(1);
+  const bool uniform = t.cap[1] == 0;
+  if (uniform) {
+    k_fixup_copy<<<148, 256, 0, s>>>(t);
+    note_kernel(1);
+  }
+  k_fixup_alloc<<<1, 256, 0, s>>>(t, uniform); note_kernel(1);
   return cudaGetLastError();
 }
 
