@@ -86,7 +86,7 @@ typedef struct dg_config {
   float load_factor;      /* target keys per bucket slot for the initial bucket count,
                              default 0.7; used as round(lf*1000)/1000 */
   uint32_t bucket_bytes;  /* 128 (default, 15 pairs = the paper's Bc),
-                             64 (7 pairs) or 32 (3 pairs) */
+                             64 (7 pairs) or 32 (3 pairs); ignored with DG_FLAG_ADAPTIVE */
   uint32_t directed;      /* 1 (default); 0 = every edge op is applied in both
                              directions */
   uint64_t pool_bytes;    /* initial overflow-bucket pool beyond the base buckets;
@@ -132,12 +132,14 @@ typedef struct dg_stats {
   uint64_t base_buckets;      /* buckets allocated at create / vertex insertion */
   uint64_t overflow_buckets;  /* chained buckets currently linked into tables */
   uint64_t free_buckets;      /* buckets on the free stack */
-  uint64_t pool_buckets;      /* buckets mapped in the pool */
-  uint64_t bump_buckets;      /* high-water mark: buckets ever handed out (base + chained) */
+  uint64_t pool_buckets;      /* buckets mapped in the pool (sum over size classes) */
+  uint64_t bump_buckets;      /* high-water mark: buckets ever handed out (base + chained;
+                                 sum over size classes) */
   uint64_t live_pairs;        /* stored edges (sum of degrees) */
   uint64_t tombstones;        /* deleted-key slots not yet reclaimed */
   uint64_t max_chain;         /* longest bucket chain (in buckets) */
-  uint64_t pool_bytes;        /* bytes of table memory mapped (pool + directory + stack) */
+  uint64_t pool_bytes;        /* bytes of table memory mapped (pools + directory + free
+                                 stacks): capacity, including the worst-case reservation */
   double load_factor;         /* live_pairs / key slots of the linked (base+overflow)
                                  buckets (Q14) */
   double utilization;         /* live_pairs * 8 B / table_bytes (Fig. 2c) */
