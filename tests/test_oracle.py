@@ -378,3 +378,24 @@ def test_generators_deterministic_and_shaped():
     gs, gd = wl.grid_edges(3, 300, 300, 0.6025)
     assert abs(gs.size / 90000 - 2.41) < 0.05
     assert np.bincount(gs).max() <= 4
+
+
+def test_grid_heldout_is_the_lattice_complement():
+    """workloads.grid_heldout_edges (cfg3 road growth) = the lattice edges grid_edges
+    did not keep: disjoint from them, and together every directed lattice edge once."""
+    import workloads as wl
+    rows, cols = 37, 53
+    s, d = wl.grid_edges(3, rows, cols, 0.6025)
+    hs, hd = wl.grid_heldout_edges(3, rows, cols, 0.6025)
+    kept = set(zip(s.tolist(), d.tolist()))
+    held = set(zip(hs.tolist(), hd.tolist()))
+    assert len(kept) == s.size and len(held) == hs.size and not (kept & held)
+    lattice = set()
+    for r in range(rows):
+        for c in range(cols):
+            u = r * cols + c
+            if c + 1 < cols:
+                lattice |= {(u, u + 1), (u + 1, u)}
+            if r + 1 < rows:
+                lattice |= {(u, u + cols), (u + cols, u)}
+    assert kept | held == lattice

@@ -55,6 +55,8 @@ def _L():
             lib.wl_grid_edges.restype = ctypes.c_uint64
             lib.wl_grid_edges.argtypes = [ctypes.c_uint64, ctypes.c_uint64, ctypes.c_uint64,
                                           ctypes.c_double, U32P, U32P]
+            lib.wl_grid_heldout_edges.restype = ctypes.c_uint64
+            lib.wl_grid_heldout_edges.argtypes = lib.wl_grid_edges.argtypes
             lib.wl_out_degrees.argtypes = [U32P, ctypes.c_uint64, ctypes.c_uint64, U32P]
             _lib = lib
     return _lib
@@ -122,6 +124,16 @@ def grid_edges(seed: int, rows: int, cols: int, p: float):
     s = np.empty(m, np.uint32)
     d = np.empty(m, np.uint32)
     L.wl_grid_edges(seed, rows, cols, p, _p32(s), _p32(d))
+    return s, d
+
+
+def grid_heldout_edges(seed: int, rows: int, cols: int, p: float):
+    """The lattice edges grid_edges() did not keep (both directions): road growth."""
+    L = _L()
+    m = int(L.wl_grid_heldout_edges(seed, rows, cols, p, None, None))
+    s = np.empty(m, np.uint32)
+    d = np.empty(m, np.uint32)
+    L.wl_grid_heldout_edges(seed, rows, cols, p, _p32(s), _p32(d))
     return s, d
 
 

@@ -149,9 +149,25 @@ void wl_rmat_edges(uint64_t seed, uint64_t stream, uint64_t i0, const uint64_t* 
  * kept with probability p (keep iff rng < p*2^64); both directions are emitted.
  * Pass src==NULL to get the count only.  Output is in row-major vertex order. */
 static inline int keep_edge(uint64_t key, uint64_t idx, uint64_t thr) { return rng_k(key, idx) < thr; }
+#define KEEP(i) (keep_edge(key, (i), thr) != held_out)
+
+static uint64_t grid_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p, int held_out,
+                           uint32_t* src, uint32_t* dst);
 
 uint64_t wl_grid_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p,
                        uint32_t* src, uint32_t* dst) {
+  return grid_edges(seed, rows, cols, p, 0, src, dst);
+}
+
+/* the lattice edges the grid did NOT keep (road-network growth workload, SURVEY
+ * §8(d) cfg3 "held-out lattice edges"), both directions, same order */
+uint64_t wl_grid_heldout_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p,
+                               uint32_t* src, uint32_t* dst) {
+  return grid_edges(seed, rows, cols, p, 1, src, dst);
+}
+
+static uint64_t grid_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p, int held_out,
+                           uint32_t* src, uint32_t* dst) {
   const uint64_t key = stream_key(seed, 0x67726964ULL);
   const double two64 = 18446744073709551616.0;
   const uint64_t thr = p >= 1.0 ? 0xFFFFFFFFFFFFFFFFULL : (uint64_t)(p * two64);
@@ -164,10 +180,10 @@ uint64_t wl_grid_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p,
     for (uint64_t c = 0; c < cols; ++c) {
       uint64_t id = (uint64_t)r * cols + c;
       /* out-edges of id: right, left, down, up */
-      if (c + 1 < cols && keep_edge(key, 2 * id, thr)) cnt++;
-      if (c > 0 && keep_edge(key, 2 * (id - 1), thr)) cnt++;
-      if ((uint64_t)r + 1 < rows && keep_edge(key, 2 * id + 1, thr)) cnt++;
-      if (r > 0 && keep_edge(key, 2 * (id - cols) + 1, thr)) cnt++;
+      if (c + 1 < cols && KEEP(2 * id)) cnt++;
+      if (c > 0 && KEEP(2 * (id - 1))) cnt++;
+      if ((uint64_t)r + 1 < rows && KEEP(2 * id + 1)) cnt++;
+      if (r > 0 && KEEP(2 * (id - cols) + 1)) cnt++;
     }
     rowcnt[r + 1] = cnt;
   }
@@ -179,10 +195,10 @@ uint64_t wl_grid_edges(uint64_t seed, uint64_t rows, uint64_t cols, double p,
       uint64_t pos = rowcnt[r];
       for (uint64_t c = 0; c < cols; ++c) {
         uint64_t id = (uint64_t)r * cols + c;
-        if (c + 1 < cols && keep_edge(key, 2 * id, thr)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id + 1); pos++; }
-        if (c > 0 && keep_edge(key, 2 * (id - 1), thr)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id - 1); pos++; }
-        if ((uint64_t)r + 1 < rows && keep_edge(key, 2 * id + 1, thr)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id + cols); pos++; }
-        if (r > 0 && keep_edge(key, 2 * (id - cols) + 1, thr)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id - cols); pos++; }
+        if (c + 1 < cols && KEEP(2 * id)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id + 1); pos++; }
+        if (c > 0 && KEEP(2 * (id - 1))) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id - 1); pos++; }
+        if ((uint64_t)r + 1 < rows && KEEP(2 * id + 1)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id + cols); pos++; }
+        if (r > 0 && KEEP(2 * (id - cols) + 1)) { src[pos] = (uint32_t)id; dst[pos] = (uint32_t)(id - cols); pos++; }
       }
     }
   }
