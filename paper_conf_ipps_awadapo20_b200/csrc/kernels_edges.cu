@@ -175,8 +175,11 @@ enum { ACT_NONE = 0, ACT_CAS_DEL = 1, ACT_CAS_INS = 2, ACT_EXTEND = 3 };
 // 0.62 ms with L = 4; delete is faster with L = 8: 1.08 vs 1.54 ms)
 template <int G, int OP>
 struct Lanes {
-#ifdef DG_LANES_PER_BUCKET
+#if defined(DG_LANES_PER_BUCKET)
   static constexpr int L = (DG_LANES_PER_BUCKET < G) ? DG_LANES_PER_BUCKET : G;
+#elif defined(DG_QUERY_LANES)  // A/B switch: query lanes only
+  static constexpr int L = OP == OP_QUERY ? ((DG_QUERY_LANES < G) ? DG_QUERY_LANES : G)
+                                          : (G >= 8 && OP != OP_DELETE) ? G / 2 : G;
 #else
   static constexpr int L = (G >= 8 && OP != OP_DELETE) ? G / 2 : G;
 #endif
