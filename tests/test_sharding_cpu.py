@@ -110,3 +110,70 @@ def test_sharded_oracle_equals_unsharded():
         # rows not owned by k are empty on k
         other = res[1 - k][0]
         assert other[u + 1] == other[u]
+
+
+def _query_worker(rank, P, port, q):
+    """a2 + a11 for queries: each rank routes its slice of the query batch to
+    owner(u) = u mod P, the owner answers from its shard, and the answers travel back
+    by the reverse all-to-all and are scattered to the slice's original positions."""
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=P)
+    try:
+        from oracle import Oracle
+        nv = 2000
+        o = Oracle(nv)
+        n = 30_000
+        off, cnt = n * rank // P, n * (rank + 1) // P - n * rank // P
+        s, d, w = wl.uniform_edges(43, 0, cnt, nv, offset=off)
+        rs, rd, rw = _exchange([s, d, w], s % P, P)
+        o.insert_edges(rs, rd, rw)
+        # a query slice with self-loops and out-of-shard sources mixed in
+        qs, qd, _ = wl.uniform_edges(43, 1, 7_001 + rank, nv, offset=rank * 8_000)
+        qd[::97] = qs[::97]
+        owner = (qs % P).astype(np.int64)
+        order = np.argsort(owner, kind="stable")
+        counts = np.bincount(owner, minlength=P)
+        rqs, rqd = _exchange([qs, qd], owner, P)
+        assert (rqs % P == rank).all()
+        _, f, wq = o.query_edges(rqs, rqd)
+        recv_counts = torch.empty(P, dtype=torch.int64)
+        dist.all_to_all_single(recv_counts, torch.tensor(counts, dtype=torch.int64))
+        back = []
+        for a in (np.asarray(f, np.int64), np.asarray(wq, np.int64)):
+            out = torch.empty(int(counts.sum()), dtype=torch.int64)
+            # reverse exchange: send what was received, receive what was sent
+            dist.all_to_all_single(out, torch.from_numpy(a), counts.tolist(), recv_counts.tolist())
+            res = np.empty(len(qs), np.int64)
+            res[order] = out.numpy()  # scatter to the original positions
+            back.append(res)
+        q.put((rank, qs, qd, back[0], back[1]))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_sharded_query_return_matches_unsharded():
+    from oracle import Oracle
+    P = 2
+    port = _free_port()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_query_worker, args=(r, P, port, q)) for r in range(P)]
+    for p in procs:
+        p.start()
+    res = [q.get(timeout=300) for _ in range(P)]
+    for p in procs:
+        p.join(timeout=60)
+        assert p.exitcode == 0
+    nv = 2000
+    o = Oracle(nv)
+    s, d, w = wl.uniform_edges(43, 0, 30_000, nv)
+    o.insert_edges(s, d, w)
+    hits = 0
+    for _, qs, qd, f, wq in res:
+        _, ef, ew = o.query_edges(qs, qd)
+        assert np.array_equal(np.asarray(ef, np.int64), f)
+        assert np.array_equal(np.asarray(ew, np.int64), wq)
+        assert not f[qs == qd].any()  # self-loops are never stored (Alg1:L3)
+        hits += int(f.sum())
+    assert hits > 0
