@@ -474,6 +474,9 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
 #define DG_SWEEP_U 4
 #endif
   constexpr int U = DG_SWEEP_U;  // buckets in flight per group (memory-level parallelism)
+#ifndef DG_SWEEP_SKIP
+#define DG_SWEEP_SKIP 0
+#endif
   __shared__ u32 sf[kVdelFilterBits / 32];
   const Group<G> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
@@ -484,10 +487,25 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b0 = gid; b0 < nbk; b0 += ng * U) {
+#if DG_SWEEP_SKIP
+    // slots fill in order and EMPTY slots only exist at the tail (the probe
+    // invariant), so a bucket whose slot 0 is EMPTY holds no key: read its first
+    // word only (one 32-B sector instead of the whole bucket)
+    u32 live = 0;
+#pragma unroll
+    for (int k0 = 0; k0 < U; k0 += G) {
+      const u32 k = k0 + g.gl;
+      const u64 b = b0 + (u64)k * ng;
+      const bool l = k < (u32)U && b < nbk && pool[b * W] != kEmpty;
+      live |= g.ballot(l) << k0;
+    }
+#else
+    constexpr u32 live = 0xFFFFFFFFu;
+#endif
     uint4 q[U];
 #pragma unroll
     for (int k = 0; k < U; ++k) {
-      const u64 b = b0 + (u64)k * ng;
+      const u64 b = (live >> k) & 1u ? b0 + (u64)k * ng : nbk;
 #ifdef DG_SWEEP_LDCS
       q[k] = b < nbk ? __ldcs(reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl))
                      : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
