@@ -37,6 +37,16 @@ uint64_t kernel_launches() { return g_launches.load(std::memory_order_relaxed); 
 
 enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 
+#ifndef DG_SLOT_WALK
+#define DG_SLOT_WALK 0
+#endif
+#ifndef DG_SLOT_WALK_ONCE
+#define DG_SLOT_WALK_ONCE 0
+#endif
+#ifndef DG_SLOT_WALK_MAIN
+#define DG_SLOT_WALK_MAIN 1
+#endif
+
 // ----------------------------------------------------------- allocator (a8) ----
 // Phase-concurrent free stack + bump cursor: during an insert
 // phase buckets are only popped, during a vertex-deletion phase only pushed, so
@@ -356,9 +366,49 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
       } else if (okey == v) {  // a racing op installed the same key: replace
         if (!S) st_relaxed_u32(ff + 1, w);
         pend = false;
-      } else {  // the slot went to another key: re-scan from the head
-        cur = head;
+      } else {
+#if DG_SLOT_WALK
+        // The slot went to another key.  If it was EMPTY in this op's view it lies in
+        // the tail bucket `cur`, every slot before it holds a key other than v (the
+        // scan, and the CAS return for this one) and EMPTY slots form the chain's
+        // suffix, so v may go into the NEXT slot of the bucket: a key CAS
+        // EMPTY -> v that succeeds finds the rest of the chain empty, hence v
+        // nowhere else.  Ops racing on one bucket (src-sorted batches) then install
+        // one per slot in one round instead of re-scanning from the head each time.
+        if (DG_SLOT_WALK_MAIN || !MAIN) {
+          if ((u32)ffo == kEmpty) {
+            // word index of the slot in its bucket from the address (pools are aligned
+            // to the bucket size), so no bucket pointer is kept live
+            const u32 nw = 4 * units_of<G, A>(cur);
+            u32 off = (u32)(reinterpret_cast<uintptr_t>(ff) >> 2) & (nw - 1u);
+            u32* p = ff;
+#if DG_SLOT_WALK_ONCE
+            if ((off += (S ? 1u : 2u)) < nw - 2u) {  // one further slot, then re-scan
+#else
+            while ((off += (S ? 1u : 2u)) < nw - 2u) {
+#endif
+              p += S ? 1 : 2;
+              const u32 k2 = atomicCAS(p, kEmpty, v);
+              if (k2 == kEmpty) {
+                atomicAdd(&t.deg[row], 1u);
+                ++my_count;
+              }
+              if (k2 == kEmpty || k2 == v) {  // installed, or a racing op's v: replace
+                if (!S) st_relaxed_u32(p + 1, w);
+                pend = false;
+                off = nw;  // ends the walk (no `break`: the ONCE form is an `if`)
+              }
+            }
+          }
+        }
+        if (pend) {  // bucket full (or the slot was a tombstone): re-scan from the head
+          cur = head;
+          ff = nullptr;
+        }
+#else
+        cur = head;  // the slot went to another key: re-scan from the head
         ff = nullptr;
+#endif
       }
     }
     if (OP == OP_INSERT) {

@@ -236,6 +236,37 @@ def test_rmat_hubs_without_hints(bb):
     assert st3["base_buckets"] + st3["overflow_buckets"] + st3["free_buckets"] <= st3["bump_buckets"]
 
 
+@pytest.mark.parametrize("hints", [True, False])
+@pytest.mark.parametrize("reuse", [True, False])
+@pytest.mark.parametrize("bb", [128, 0])
+def test_src_sorted_batches(bb, reuse, hints):
+    """Src-sorted R-MAT batches (the sorted bulk build): the ops of a warp
+    hit the same tables and race for the same free slots; duplicates of one key sit
+    next to each other with different weights (Q1 membership rule)."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    scale = 15
+    nv = 1 << scale
+    s, d = wl.rmat_edges(17, 0, 600_000, scale, wl.GRAPH500)
+    w = wl.weights(17, 0, s.size)
+    order = np.lexsort((d, s))
+    s, d, w = s[order], d[order], w[order]
+    h = torch.bincount(torch.from_numpy(s.astype(np.int64)), minlength=nv).to(torch.int32)
+    g = Graph(nv, h.cuda() if hints else None, bucket_bytes=bb, reuse_tombstones=reuse)
+    o = Oracle(nv)
+    half = s.size // 2
+    for lo, hi in ((0, half), (half, s.size)):
+        assert g.insert_edges(cuda(s[lo:hi]), cuda(d[lo:hi]), cuda(w[lo:hi]), count=True) == \
+            o.insert_edges(s[lo:hi], d[lo:hi], w[lo:hi])[1]
+    cand = check_against_oracle(g, o, "sorted insert")
+    check_queries(g, o, s[::5], d[::5], cand, "sorted queries")
+    # delete a sorted third, re-insert it sorted (tombstone reuse path when enabled)
+    m = slice(0, s.size // 3)
+    assert g.delete_edges(cuda(s[m]), cuda(d[m]), count=True) == o.delete_edges(s[m], d[m])[1]
+    assert g.insert_edges(cuda(s[m]), cuda(d[m]), cuda(w[m]), count=True) == \
+        o.insert_edges(s[m], d[m], w[m])[1]
+    check_against_oracle(g, o, "sorted churn")
+
+
 def test_freed_buckets_are_reused():
     """Vertex deletion returns chained buckets to the allocator; later
     chain growth pops them before touching never-used memory."""

@@ -9,6 +9,6 @@ import json, sys
 v = sys.argv[1]
 d = json.load(open(f"gpurun_out/ab_{v}.json"))
 o = d["ops"]
-print(f"{v:12s} value {d['value']:9.0f}  ins {o['insert']['kernel_ms_per_batch']:.3f}  qry {o['query']['kernel_ms_per_batch']:.3f}  del {o['delete']['kernel_ms_per_batch']:.3f} ms  bulk {d['bulk_build']['insert_ms']:.1f} ms")
+print(f"{v:12s} value {d['value']:9.0f}  ins {o['insert']['kernel_ms_per_batch']:.3f}  qry {o['query']['kernel_ms_per_batch']:.3f}  del {o['delete']['kernel_ms_per_batch']:.3f} ms  bulk {d['bulk_build']['insert_ms']:.1f} ms (kernel {d['bulk_build'].get('insert_kernel_ms', float('nan')):.2f}, src-sorted {d['bulk_build'].get('sorted_insert_kernel_ms', float('nan')):.2f})")
 PY
 done
