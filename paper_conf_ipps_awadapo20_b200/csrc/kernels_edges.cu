@@ -37,11 +37,15 @@ uint64_t kernel_launches() { return g_launches.load(std::memory_order_relaxed); 
 
 enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 
+// After a lost install CAS on an EMPTY slot, try the next slot of the bucket once
+// before re-scanning (measured on B200, cfg2: src-sorted bulk build 10.98 -> 6.8 ms,
+// random 2^24 insert 1.20 -> 1.21 ms; walking the whole bucket spills registers and
+// costs random inserts 6%)
 #ifndef DG_SLOT_WALK
-#define DG_SLOT_WALK 0
+#define DG_SLOT_WALK 1
 #endif
 #ifndef DG_SLOT_WALK_ONCE
-#define DG_SLOT_WALK_ONCE 0
+#define DG_SLOT_WALK_ONCE 1
 #endif
 #ifndef DG_SLOT_WALK_MAIN
 #define DG_SLOT_WALK_MAIN 1
@@ -169,7 +173,8 @@ __device__ __forceinline__ void release_chunks(const Tables& t) {
 //   The insert follows Alg. 1's replace: the whole chain is scanned
 //   for the key before a new pair is installed; the install targets the FIRST free
 //   slot (first tombstone when tombstones are reused, else the first
-//   EMPTY) and a failed install CAS re-scans from the head, so two
+//   EMPTY); a failed install CAS tries the next slot of the bucket once
+//   (when the lost slot was EMPTY) and otherwise re-scans from the head, so two
 //   inserts of one key always contend for the same slot.
 enum { ACT_NONE = 0, ACT_CAS_DEL = 1, ACT_CAS_INS = 2, ACT_EXTEND = 3 };
 
