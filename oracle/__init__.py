@@ -36,7 +36,8 @@ def build(force: bool = False) -> str:
     src = os.path.join(_HERE, "oracle.cpp")
     if force or not os.path.exists(_SO) or os.path.getmtime(_SO) < os.path.getmtime(src):
         tmp = _SO + f".tmp{os.getpid()}"
-        subprocess.check_call(["g++", "-O2", "-std=c++17", "-fPIC", "-shared", "-o", tmp, src])
+        subprocess.check_call(["g++", "-O2", "-std=c++17", "-pthread", "-fPIC", "-shared", "-o", tmp,
+                               src])
         os.replace(tmp, _SO)
     return _SO
 
@@ -49,6 +50,8 @@ def _L():
             lib.orc_create.restype = VP
             lib.orc_create.argtypes = [ctypes.c_uint64, ctypes.c_int]
             lib.orc_destroy.argtypes = [VP]
+            lib.orc_set_threads.restype = ctypes.c_int
+            lib.orc_set_threads.argtypes = [VP, ctypes.c_uint]
             lib.orc_num_vertices.restype = ctypes.c_uint64
             lib.orc_num_vertices.argtypes = [VP]
             lib.orc_insert_edges.restype = ctypes.c_int
@@ -82,6 +85,17 @@ def _u32(a):
     return a, a.ctypes.data_as(U32P)
 
 
+def default_threads() -> int:
+    env = os.environ.get("ORACLE_THREADS")
+    if env:
+        return max(1, int(env))
+    try:
+        n = len(os.sched_getaffinity(0))
+    except AttributeError:
+        n = os.cpu_count() or 1
+    return max(1, min(n, 16))
+
+
 def initial_buckets(hint: int, lf_milli: int = 700, bucket_capacity: int = 15) -> int:
     """ceil(|A_u| / (lf*Bc)), 1 if unknown — PAPER.md §IV-A2 P:L411-414."""
     return int(_L().orc_initial_buckets(hint, lf_milli, bucket_capacity))
@@ -90,12 +104,18 @@ def initial_buckets(hint: int, lf_milli: int = 700, bucket_capacity: int = 15) -
 class Oracle:
     """One ``std::unordered_map`` per vertex; batches applied in order."""
 
-    def __init__(self, num_vertices: int, directed: bool = True):
+    def __init__(self, num_vertices: int, directed: bool = True, threads: int | None = None):
+        """``threads``: host threads (thread t owns the vertices u with
+        u % T == t, so every vertex's ops keep their batch order; results do not
+        depend on T).  Default: $ORACLE_THREADS, else min(usable CPUs, 16)."""
         self._L = _L()
         self.h = self._L.orc_create(num_vertices, int(directed))
         if not self.h:
             raise ValueError("num_vertices out of range")
         self.directed = directed
+        self.threads = default_threads() if threads is None else int(threads)
+        if self._L.orc_set_threads(self.h, self.threads) != OK:
+            raise ValueError("threads out of range")
 
     def __del__(self):
         h = getattr(self, "h", None)

@@ -14,11 +14,17 @@ import numpy as np
 
 
 def canonical(row_offsets, dst, w=None):
+    """Rows sorted by dst, weights carried (a stable sort of the (row, dst) keys; rows
+    are already grouped, so an export that is sorted already costs one linear pass)."""
     ro = np.asarray(row_offsets, np.uint64)
     dst = np.asarray(dst, np.uint32)
     deg = np.diff(ro).astype(np.int64)
     rows = np.repeat(np.arange(deg.size, dtype=np.uint64), deg)
-    order = np.lexsort((dst, rows))
+    key = (rows << np.uint64(32)) | dst.astype(np.uint64)
+    del rows
+    if key.size > 1 and bool((key[1:] >= key[:-1]).all()):
+        return ro, dst, (None if w is None else np.asarray(w, np.uint32))
+    order = np.argsort(key, kind="stable")
     return ro, dst[order], (None if w is None else np.asarray(w, np.uint32)[order])
 
 

@@ -28,7 +28,7 @@
 #include <algorithm>
 #include <cstdint>
 #include <cstring>
-#include <map>
+#include <thread>
 #include <unordered_map>
 #include <unordered_set>
 #include <utility>
@@ -41,15 +41,28 @@ enum { ORC_OK = 0, ORC_ERR_INVALID_ARGUMENT = 1, ORC_ERR_VERTEX_OUT_OF_RANGE = 2
 /* Q18: vertex IDs are u32 below 2^32-2 (the two top values are reserved). */
 constexpr uint64_t kMaxVertices = 0xFFFFFFFEull;
 
+/* A stored edge: its weight, plus the number of the insert batch that last wrote
+ * it.  The stamp is bookkeeping for the Q1 candidate sets only (it tells a second
+ * write of a key inside one batch from a first one); the graph is A_u : v -> w. */
+struct Entry {
+  uint32_t w;
+  uint64_t batch;
+};
+
+inline uint64_t key_of(uint32_t u, uint32_t v) { return ((uint64_t)u << 32) | v; }
+
 struct Oracle {
   uint64_t cap = 0;
   bool directed = true;
-  std::vector<std::unordered_map<uint32_t, uint32_t>> A;  // A_u : v -> w
+  unsigned T = 1;        // host threads; thread t owns the vertices u with u % T == t
+  uint64_t batch = 0;    // insert batches applied so far
+  std::vector<std::unordered_map<uint32_t, Entry>> A;  // A_u : v -> w
   /* Q1: keys (u,v) written >= 2 times by their most recent insert batch, with
-   * the set of weights that batch carried for them; any one of them is a
+   * the weights that batch carried for them (in batch order); any one of them is a
    * correct stored weight ("only the most recent edge ... will be stored",
-   * P:L469-471, and a parallel batch has no order). */
-  std::map<std::pair<uint32_t, uint32_t>, std::vector<uint32_t>> cand;
+   * P:L469-471, and a parallel batch has no order).  Sharded like the rows: the
+   * set of key (u,v) lives in cand[u % T]. */
+  std::vector<std::unordered_map<uint64_t, std::vector<uint32_t>>> cand;
 };
 
 inline bool in_range(const Oracle& g, const uint32_t* a, uint64_t n) {
@@ -73,6 +86,23 @@ void expand(const Oracle& g, const uint32_t* s, const uint32_t* d, const uint32_
   }
 }
 
+/* Run f(t) for t = 0..T-1 on T threads (T = 1: inline).  Work partitioned by vertex
+ * (u % T) keeps every vertex's ops in batch order on one thread. */
+constexpr uint64_t kParallelMin = 1u << 15;  // smaller batches: one thread
+inline unsigned threads_for(const Oracle& g, uint64_t work) { return work < kParallelMin ? 1u : g.T; }
+
+template <typename F>
+void parallel(unsigned T, F f) {
+  if (T <= 1) {
+    f(0u);
+    return;
+  }
+  std::vector<std::thread> th;
+  th.reserve(T);
+  for (unsigned t = 0; t < T; ++t) th.emplace_back(f, t);
+  for (auto& x : th) x.join();
+}
+
 }  // namespace
 
 extern "C" {
@@ -83,7 +113,21 @@ void* orc_create(uint64_t num_vertices, int directed) {
   g->cap = num_vertices;
   g->directed = directed != 0;
   g->A.resize(num_vertices);  // hints only affect performance: none taken
+  g->cand.resize(1);
   return g;
+}
+
+/* Host threads used by the following calls (default 1).  Results do not depend on
+ * it: each vertex's ops stay in batch order on one thread. */
+int orc_set_threads(void* h, unsigned threads) {
+  Oracle& g = *static_cast<Oracle*>(h);
+  if (threads < 1 || threads > 256) return ORC_ERR_INVALID_ARGUMENT;
+  std::vector<std::unordered_map<uint64_t, std::vector<uint32_t>>> c(threads);
+  for (auto& shard : g.cand)
+    for (auto& kv : shard) c[(kv.first >> 32) % threads].emplace(kv.first, std::move(kv.second));
+  g.cand.swap(c);
+  g.T = threads;
+  return ORC_OK;
 }
 
 void orc_destroy(void* h) { delete static_cast<Oracle*>(h); }
@@ -96,7 +140,10 @@ uint64_t orc_num_vertices(void* h) { return static_cast<Oracle*>(h)->cap; }
  *   - replace semantics: an existing key gets the new weight, otherwise the pair
  *     is added (fn3 P:L235-236);
  *   - *n_added counts keys that were absent before the batch (exact degree
- *     maintenance). */
+ *     maintenance);
+ *   - Q1: the first write of a key in this batch clears its old candidate set; a
+ *     second write makes {first weight, second weight} its candidates, later
+ *     writes append. */
 int orc_insert_edges(void* h, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
                      uint64_t n, uint64_t* n_added) {
   Oracle& g = *static_cast<Oracle*>(h);
@@ -105,26 +152,37 @@ int orc_insert_edges(void* h, const uint32_t* src, const uint32_t* dst, const ui
   if (!in_range(g, src, n) || !in_range(g, dst, n)) return ORC_ERR_VERTEX_OUT_OF_RANGE;
   std::vector<uint32_t> S, D, W;
   expand(g, src, dst, w, n, S, D, W);
-
-  /* weights per key in this batch, to record the Q1 candidate sets */
-  std::map<std::pair<uint32_t, uint32_t>, std::vector<uint32_t>> seen;
-  for (size_t i = 0; i < S.size(); ++i) {
-    if (S[i] == D[i]) continue;
-    seen[{S[i], D[i]}].push_back(W[i]);
-  }
-  uint64_t added = 0;
-  for (size_t i = 0; i < S.size(); ++i) {
-    const uint32_t u = S[i], v = D[i];
-    if (u == v) continue;                               // Alg1:L3
-    auto& Au = g.A[u];
-    if (Au.find(v) == Au.end()) ++added;                // replace() returned "added"
-    Au[v] = W[i];                                       // most recent value stored
-  }
-  for (auto& kv : seen) {
-    if (kv.second.size() >= 2) g.cand[kv.first] = kv.second;
-    else g.cand.erase(kv.first);
-  }
-  if (n_added) *n_added = added;
+  const uint64_t b = ++g.batch;
+  const unsigned P = threads_for(g, S.size());
+  std::vector<uint64_t> added(P, 0);
+  parallel(P, [&](unsigned t) {
+    uint64_t a = 0;
+    for (size_t i = 0; i < S.size(); ++i) {
+      const uint32_t u = S[i], v = D[i];
+      if (u % P != t) continue;                         // another thread's vertex
+      if (u == v) continue;                             // Alg1:L3
+      auto& cand = g.cand[u % g.T];
+      auto& Au = g.A[u];
+      auto it = Au.find(v);
+      if (it == Au.end()) {                             // replace() returned "added"
+        ++a;
+        Au.emplace(v, Entry{W[i], b});
+        if (!cand.empty()) cand.erase(key_of(u, v));
+      } else if (it->second.batch != b) {               // first write of the key in this batch
+        it->second = Entry{W[i], b};                    // most recent value stored
+        if (!cand.empty()) cand.erase(key_of(u, v));
+      } else {                                          // written before in this batch (Q1)
+        auto& c = cand[key_of(u, v)];
+        if (c.empty()) c.push_back(it->second.w);
+        c.push_back(W[i]);
+        it->second.w = W[i];
+      }
+    }
+    added[t] = a;
+  });
+  uint64_t total = 0;
+  for (uint64_t a : added) total += a;
+  if (n_added) *n_added = total;
   return ORC_OK;
 }
 
@@ -140,16 +198,24 @@ int orc_delete_edges(void* h, const uint32_t* src, const uint32_t* dst, uint64_t
   if (!in_range(g, src, n) || !in_range(g, dst, n)) return ORC_ERR_VERTEX_OUT_OF_RANGE;
   std::vector<uint32_t> S, D, W;
   expand(g, src, dst, nullptr, n, S, D, W);
-  uint64_t removed = 0;
-  for (size_t i = 0; i < S.size(); ++i) {
-    const uint32_t u = S[i], v = D[i];
-    if (u == v) continue;
-    if (g.A[u].erase(v)) {
-      ++removed;
-      g.cand.erase({u, v});
+  const unsigned P = threads_for(g, S.size());
+  std::vector<uint64_t> removed(P, 0);
+  parallel(P, [&](unsigned t) {
+    uint64_t r = 0;
+    for (size_t i = 0; i < S.size(); ++i) {
+      const uint32_t u = S[i], v = D[i];
+      if (u % P != t || u == v) continue;
+      if (g.A[u].erase(v)) {
+        ++r;
+        auto& cand = g.cand[u % g.T];
+        if (!cand.empty()) cand.erase(key_of(u, v));
+      }
     }
-  }
-  if (n_removed) *n_removed = removed;
+    removed[t] = r;
+  });
+  uint64_t total = 0;
+  for (uint64_t r : removed) total += r;
+  if (n_removed) *n_removed = total;
   return ORC_OK;
 }
 
@@ -161,13 +227,17 @@ int orc_query_edges(void* h, const uint32_t* src, const uint32_t* dst, uint64_t 
   Oracle& g = *static_cast<Oracle*>(h);
   if (n && (!src || !dst || !found)) return ORC_ERR_INVALID_ARGUMENT;
   if (!in_range(g, src, n) || !in_range(g, dst, n)) return ORC_ERR_VERTEX_OUT_OF_RANGE;
-  for (uint64_t i = 0; i < n; ++i) {
-    const uint32_t u = src[i], v = dst[i];
-    auto it = g.A[u].find(v);
-    const bool f = (u != v) && it != g.A[u].end();
-    found[i] = f ? 1 : 0;
-    if (weight) weight[i] = f ? it->second : 0u;
-  }
+  const unsigned P = threads_for(g, n);
+  parallel(P, [&](unsigned t) {  // read-only: any split works; contiguous ranges
+    const uint64_t lo = n * t / P, hi = n * (t + 1) / P;
+    for (uint64_t i = lo; i < hi; ++i) {
+      const uint32_t u = src[i], v = dst[i];
+      auto it = g.A[u].find(v);
+      const bool f = (u != v) && it != g.A[u].end();
+      found[i] = f ? 1 : 0;
+      if (weight) weight[i] = f ? it->second.w : 0u;
+    }
+  });
   return ORC_OK;
 }
 
@@ -179,20 +249,26 @@ int orc_delete_vertices(void* h, const uint32_t* ids, uint64_t n) {
   Oracle& g = *static_cast<Oracle*>(h);
   if (n && !ids) return ORC_ERR_INVALID_ARGUMENT;
   if (!in_range(g, ids, n)) return ORC_ERR_VERTEX_OUT_OF_RANGE;
-  std::unordered_set<uint32_t> D(ids, ids + n);
+  const std::unordered_set<uint32_t> D(ids, ids + n);
   if (D.empty()) return ORC_OK;
   for (uint32_t u : D) g.A[u].clear();
-  for (uint64_t x = 0; x < g.cap; ++x) {
-    auto& Ax = g.A[x];
-    for (auto it = Ax.begin(); it != Ax.end();) {
-      if (D.count(it->first)) it = Ax.erase(it);
-      else ++it;
+  const unsigned P = threads_for(g, g.cap);
+  parallel(P, [&](unsigned t) {
+    for (uint64_t x = t; x < g.cap; x += P) {
+      auto& Ax = g.A[x];
+      for (auto it = Ax.begin(); it != Ax.end();) {
+        if (D.count(it->first)) it = Ax.erase(it);
+        else ++it;
+      }
     }
-  }
-  for (auto it = g.cand.begin(); it != g.cand.end();) {
-    if (D.count(it->first.first) || D.count(it->first.second)) it = g.cand.erase(it);
-    else ++it;
-  }
+    for (unsigned c = t; c < g.T; c += P) {
+      auto& cand = g.cand[c];
+      for (auto it = cand.begin(); it != cand.end();) {
+        if (D.count((uint32_t)(it->first >> 32)) || D.count((uint32_t)it->first)) it = cand.erase(it);
+        else ++it;
+      }
+    }
+  });
   return ORC_OK;
 }
 
@@ -225,18 +301,27 @@ uint64_t orc_num_edges(void* h) {
 void orc_export(void* h, uint64_t* row_offsets, uint32_t* dst, uint32_t* weight) {
   Oracle& g = *static_cast<Oracle*>(h);
   uint64_t pos = 0;
-  std::vector<std::pair<uint32_t, uint32_t>> row;
   for (uint64_t u = 0; u < g.cap; ++u) {
     row_offsets[u] = pos;
-    row.assign(g.A[u].begin(), g.A[u].end());
-    std::sort(row.begin(), row.end());
-    for (auto& p : row) {
-      if (dst) dst[pos] = p.first;
-      if (weight) weight[pos] = p.second;
-      ++pos;
-    }
+    pos += g.A[u].size();
   }
   row_offsets[g.cap] = pos;
+  const unsigned P = threads_for(g, pos);
+  parallel(P, [&](unsigned t) {  // rows are independent: contiguous row ranges
+    std::vector<std::pair<uint32_t, uint32_t>> row;
+    const uint64_t lo = g.cap * t / P, hi = g.cap * (t + 1) / P;
+    for (uint64_t u = lo; u < hi; ++u) {
+      row.clear();
+      for (auto& kv : g.A[u]) row.emplace_back(kv.first, kv.second.w);
+      std::sort(row.begin(), row.end());
+      uint64_t p = row_offsets[u];
+      for (auto& e : row) {
+        if (dst) dst[p] = e.first;
+        if (weight) weight[p] = e.second;
+        ++p;
+      }
+    }
+  });
 }
 
 /* exact number of neighbours per vertex */
@@ -249,11 +334,12 @@ void orc_degrees(void* h, uint32_t* out) {
 uint64_t orc_candidates(void* h, uint32_t* u, uint32_t* v, uint32_t* w, uint64_t cap) {
   Oracle& g = *static_cast<Oracle*>(h);
   uint64_t k = 0;
-  for (auto& kv : g.cand)
-    for (uint32_t x : kv.second) {
-      if (k < cap) { u[k] = kv.first.first; v[k] = kv.first.second; w[k] = x; }
-      ++k;
-    }
+  for (auto& shard : g.cand)
+    for (auto& kv : shard)
+      for (uint32_t x : kv.second) {
+        if (k < cap) { u[k] = (uint32_t)(kv.first >> 32); v[k] = (uint32_t)kv.first; w[k] = x; }
+        ++k;
+      }
   return k;
 }
 
@@ -270,23 +356,31 @@ uint64_t orc_triangle_count(void* h) {
     return da < db || (da == db && a < b);
   };
   std::vector<std::vector<uint32_t>> Np(n);
-  for (uint64_t u = 0; u < n; ++u) {
-    for (auto& kv : g.A[u])
-      if (rank_less((uint32_t)u, kv.first)) Np[u].push_back(kv.first);
-    std::sort(Np[u].begin(), Np[u].end());
-  }
-  uint64_t count = 0;
-  for (uint64_t u = 0; u < n; ++u)
-    for (uint32_t v : Np[u]) {
-      const auto& a = Np[u];
-      const auto& b = Np[v];
-      size_t i = 0, j = 0;
-      while (i < a.size() && j < b.size()) {
-        if (a[i] < b[j]) ++i;
-        else if (a[i] > b[j]) ++j;
-        else { ++count; ++i; ++j; }
-      }
+  parallel(g.T, [&](unsigned t) {
+    for (uint64_t u = t; u < n; u += g.T) {
+      for (auto& kv : g.A[u])
+        if (rank_less((uint32_t)u, kv.first)) Np[u].push_back(kv.first);
+      std::sort(Np[u].begin(), Np[u].end());
     }
+  });
+  std::vector<uint64_t> part(g.T, 0);
+  parallel(g.T, [&](unsigned t) {
+    uint64_t count = 0;
+    for (uint64_t u = t; u < n; u += g.T)
+      for (uint32_t v : Np[u]) {
+        const auto& a = Np[u];
+        const auto& b = Np[v];
+        size_t i = 0, j = 0;
+        while (i < a.size() && j < b.size()) {
+          if (a[i] < b[j]) ++i;
+          else if (a[i] > b[j]) ++j;
+          else { ++count; ++i; ++j; }
+        }
+      }
+    part[t] = count;
+  });
+  uint64_t count = 0;
+  for (uint64_t c : part) count += c;
   return count;
 }
 

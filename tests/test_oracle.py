@@ -68,6 +68,10 @@ class Dense:
         self.P = np.zeros((n, n), bool)
         self.W = np.zeros((n, n), np.uint64)
         self.directed = directed
+        # Q1: key -> the weights its most recent insert batch wrote, for
+        # keys that batch wrote >= 2 times; a single write, a delete or the deletion
+        # of an endpoint drops the entry
+        self.cand = {}
 
     @property
     def n(self):
@@ -84,13 +88,20 @@ class Dense:
         if any(x >= self.n for x in list(s) + list(d)):
             return 2, 0
         added = 0
+        writes = {}
         for u, v, x in zip(*self._expand(s, d, w)):
             if u == v:
                 continue
+            writes.setdefault((u, v), []).append(x)
             if not self.P[u, v]:
                 added += 1
             self.P[u, v] = True
             self.W[u, v] = x
+        for k, ws in writes.items():
+            if len(ws) >= 2:
+                self.cand[k] = ws
+            else:
+                self.cand.pop(k, None)
         return 0, added
 
     def delete(self, s, d):
@@ -102,6 +113,7 @@ class Dense:
                 self.P[u, v] = False
                 self.W[u, v] = 0
                 removed += 1
+                self.cand.pop((u, v), None)
         return 0, removed
 
     def query(self, s, d):
@@ -118,7 +130,12 @@ class Dense:
             self.P[:, u] = False
             self.W[u, :] = 0
             self.W[:, u] = 0
+        D = set(int(x) for x in ids)
+        self.cand = {k: v for k, v in self.cand.items() if k[0] not in D and k[1] not in D}
         return 0
+
+    def candidates(self):
+        return sorted((u, v, int(x)) for (u, v), ws in self.cand.items() for x in ws)
 
     def insert_vertices(self, ids):
         m = max([self.n] + [int(x) + 1 for x in ids])
@@ -137,7 +154,7 @@ class Dense:
 
 def _random_sequence_check(seed, directed, n0=48, steps=40):
     rs = np.random.RandomState(seed)
-    g = Oracle(n0, directed)
+    g = Oracle(n0, directed, threads=1)
     m = Dense(n0, directed)
     for step in range(steps):
         op = rs.choice(["ins", "ins", "del", "qry", "dv", "iv", "bad"], p=[.3, .15, .2, .15, .08, .05, .07])
@@ -177,6 +194,9 @@ def _random_sequence_check(seed, directed, n0=48, steps=40):
         assert np.array_equal(ww, mww), f"step {step} op {op}"
         assert np.array_equal(g.degrees(), np.diff(ro).astype(np.uint32))
         assert check_invariants(ro, dd, g.degrees()) == []
+        cu, cv, cw = g.candidates()
+        assert sorted(zip(cu.tolist(), cv.tolist(), cw.tolist())) == m.candidates(), \
+            f"step {step} op {op}: Q1 candidate sets"
 
 
 @pytest.mark.parametrize("seed", range(6))
@@ -187,6 +207,53 @@ def test_dense_model_directed(seed):
 @pytest.mark.parametrize("seed", range(3))
 def test_dense_model_undirected(seed):
     _random_sequence_check(100 + seed, False)
+
+
+def test_threads_do_not_change_results():
+    """T threads, thread t owns the vertices u % T == t, so every
+    vertex's ops keep their batch order — the graph, counts, answers, Q1 candidate
+    sets and triangle count are those of one thread (batches above the oracle's
+    one-thread cutoff of 2^15 ops, with duplicates, misses and vertex deletions)."""
+    nv = 3000
+    res = []
+    for T in (1, 3, 8):
+        g = Oracle(nv, directed=(T != 3), threads=T)
+        out = []
+        for b in range(3):
+            s, d, w = wl.uniform_edges(21, b, 60_000, nv)
+            s[:6000], d[:6000] = s[6000:12000], d[6000:12000]  # 10% duplicate keys (Q1)
+            out.append(g.insert_edges(s, d, w))
+        qs, qd, _ = wl.uniform_edges(21, 9, 50_000, nv)
+        out.append(g.query_edges(qs, qd))
+        ds, dd, _ = wl.uniform_edges(21, 1, 40_000, nv)
+        out.append(g.delete_edges(ds, dd))
+        out.append(g.delete_vertices(wl.uniform_u32(21, 5, 50, nv)))
+        out.append(g.export())
+        cu, cv, cw = g.candidates()
+        out.append(sorted(zip(cu.tolist(), cv.tolist(), cw.tolist())))
+        out.append(g.triangle_count() if T == 3 else None)
+        res.append((T, out))
+    # T = 1 and T = 8 (both directed) agree on everything
+    a, b = res[0][1], res[2][1]
+    for x, y in zip(a, b):
+        if isinstance(x, tuple):
+            for p, q in zip(x, y):
+                assert np.array_equal(np.asarray(p), np.asarray(q))
+        else:
+            assert x == y
+    assert len(a[-2]) > 1000  # duplicates were exercised
+    # undirected T = 3 against one thread
+    g1 = Oracle(nv, directed=False, threads=1)
+    for b in range(3):
+        s, d, w = wl.uniform_edges(21, b, 60_000, nv)
+        s[:6000], d[:6000] = s[6000:12000], d[6000:12000]
+        g1.insert_edges(s, d, w)
+    ds, dd, _ = wl.uniform_edges(21, 1, 40_000, nv)
+    g1.delete_edges(ds, dd)
+    g1.delete_vertices(wl.uniform_u32(21, 5, 50, nv))
+    for p, q in zip(g1.export(), res[1][1][6]):
+        assert np.array_equal(p, q)
+    assert g1.triangle_count() == res[1][1][8]
 
 
 # --------------------------------------------------------------- invariants ---
