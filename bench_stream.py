@@ -243,7 +243,7 @@ def run_tc(args, cfg):
     flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
     IB = 1 << 22
     t_ins = t_tc = 0.0
-    wedges = 0
+    wedges = []  # edgeExist probes of each timed TC, counted on the graph it ran on
     tri = []
     clock = None
     # warm-up steps count triangles on the bulk-built graph only; the timed steps are
@@ -273,6 +273,8 @@ def run_tc(args, cfg):
             t_ins += e0.elapsed_time(e1)
             t_tc += e1.elapsed_time(e2)
             tri.append(c)
+            # the graph grows every step: count this TC's probes now (untimed, host)
+            wedges.append(_wedges(g, rank, world))
     prof = g.profile_read()
     clocks = clock.stop() if clock else None
     g.profile_enable(False)
@@ -283,9 +285,9 @@ def run_tc(args, cfg):
     K = args.steps
     wk = prof["kernel_ms"]["tc"]
     nl = max(1, prof["kernel_launches"]["tc"])
-    wedge_ops = _wedges(g, rank, world)  # per TC on this replica's part
-    wedge_ops = int(_sum(torch, pg, dev, [wedge_ops])[0])
-    edge_ops = 2 * IB * K + wedge_ops * K
+    wedges = [int(x) for x in _sum(torch, pg, dev, wedges)]  # all parts, per step
+    wedge_ops = sum(wedges) / K  # mean per TC
+    edge_ops = 2 * IB * K + sum(wedges)
     total_ms = t_ins + t_tc
     value = edge_ops / (total_ms * 1e3)
     peak, peak_src = load_peaks()
@@ -293,15 +295,27 @@ def run_tc(args, cfg):
     # mean bytes of a linked bucket
     Sb = S or st_["table_bytes"] / max(1, st_["base_buckets"] + st_["overflow_buckets"])
     bytes_per_probe = Sb + 4
+    # wk covers the nl timed launches (one per step); their probes are sum(wedges)
     roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16 if S else 'adaptive'},{variant}>",
                 "unit": "GB/s",
-                "achieved": wedge_ops / world * bytes_per_probe / (wk / nl * 1e-3) / 1e9,
+                "achieved": sum(wedges) / world * bytes_per_probe / (wk * 1e-3) / 1e9,
                 "peak": peak, "peak_source": peak_src, "traffic": None,
-                "algorithmic_bytes_per_launch": wedge_ops / world * bytes_per_probe,
-                "note": "probes largely hit L2 (small tables reused), so achieved may exceed "
-                        "the HBM copy peak; ncu DRAM bytes in profiles/",
-                "kernel_share_of_step": wk / nl * K / total_ms if total_ms else None}
+                "algorithmic_bytes_per_launch": sum(wedges) / world * bytes_per_probe / nl,
+                "note": "model bytes = one bucket of A_v + 4 B per wedge probe, wedges counted "
+                        "per step on the graph each TC ran on; probes largely hit L2 (small "
+                        "tables reused), so the model may exceed the HBM copy peak — the DRAM "
+                        "fraction from ncu is `dram_frac`",
+                "kernel_share_of_step": wk / total_ms if total_ms else None}
     roofline["frac"] = roofline["achieved"] / peak
+    tpath = os.path.join(os.path.dirname(os.path.abspath(__file__)), "profiles", "ncu_traffic.json")
+    try:
+        ent = json.load(open(tpath)).get(f"cfg5/tc/s{S}")
+    except (OSError, ValueError):
+        ent = None
+    if ent:  # ncu DRAM bytes of one wedge launch over its ncu duration
+        roofline["traffic"] = ent["dram_bytes_per_launch"]
+        roofline["dram_frac"] = ent["dram_bytes_per_launch"] / (ent["ncu_duration_ms"] * 1e-3) / 1e9 / peak
+        roofline["dram_source"] = ent.get("source")
     line = {
         "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": K,
         "warmup": args.warmup, "ms_per_step": total_ms / K, "higher_is_better": True,
@@ -316,8 +330,8 @@ def run_tc(args, cfg):
                    "parallelism": f"replicas x{world}, wedges split by u mod {world}"
                    if world > 1 else "single GPU"},
         "tc": {"triangles_per_step": tri, "tc_ms_per_step": t_tc / K,
-               "insert_ms_per_step": t_ins / K, "wedges_per_tc": wedge_ops,
-               "wedge_G_per_s": wedge_ops / (t_tc / K * 1e-3) / 1e9,
+               "insert_ms_per_step": t_ins / K, "wedges_per_tc": wedges,
+               "wedge_G_per_s": sum(wedges) / (t_tc * 1e-3) / 1e9,
                "insert_M_edges_s": 2 * IB / (t_ins / K * 1e3)},
         "bulk_build": {"insert_ms": bulk_ms},
         "roofline": roofline, "gpu_launches": prof["launches"], "clocks": clocks,

@@ -68,6 +68,8 @@ extern "C" {
 #endif
 
 typedef struct dg_graph_s* dg_graph;
+/* In-process rank group (see dg_group_create). */
+typedef struct dg_group_s* dg_group;
 
 typedef enum dg_status {
   DG_OK = 0,
@@ -96,7 +98,11 @@ typedef struct dg_config {
   int32_t nranks;         /* number of GPUs the graph is sharded over (1 = single GPU) */
   uint32_t flags;         /* DG_FLAG_* bits, default 0 */
   const void* nccl_unique_id; /* 128-byte ncclUniqueId from dg_get_unique_id() on rank 0,
-                                 broadcast by the caller; NULL when nranks == 1 */
+                                 broadcast by the caller; NULL when nranks == 1 or when
+                                 `group` is set */
+  dg_group group;         /* in-process rank group (dg_group_create) instead of NCCL:
+                             the nranks ranks are host threads of this process; NULL =
+                             one process per rank over NCCL */
 } dg_config;
 
 /* dg_config.flags: new keys are installed in the first tombstone of their chain by
@@ -125,6 +131,12 @@ typedef struct dg_config {
  * class has its own bucket pool and free stack.  `bucket_bytes` is ignored.  Results
  * are those of every other layout. */
 #define DG_FLAG_ADAPTIVE 8u
+/* Multi-GPU batch routing through the copy exchange (partition into a local send
+ * buffer, grouped send/recv, receive buffer) instead of the default fused exchange
+ * (one kernel partitions the batch and stores every op straight into its owner's
+ * NVLink-mapped receive window).  Results are identical; for A/B runs and tests.
+ * The environment variable DG_ROUTER=nccl has the same effect. */
+#define DG_FLAG_COPY_EXCHANGE 16u
 
 /* Memory / structure statistics (Fig. 2b/c quantities). */
 typedef struct dg_stats {
@@ -160,6 +172,20 @@ DG_API const char* dg_status_string(dg_status s);
 /* Multi-GPU bootstrap: writes a 128-byte ncclUniqueId to out128 (host memory).
  * Call on rank 0 only, then broadcast it (e.g. over a torch process group). */
 DG_API dg_status dg_get_unique_id(void* out128);
+
+/* In-process rank group: lets `nranks` host threads of ONE process act as the ranks
+ * of a sharded graph (each thread creates its own handle with cfg.group = the group,
+ * cfg.rank = its rank, cfg.nranks = nranks, and then makes every collective call
+ * with its own slice, exactly as separate processes would).  Ranks may share one
+ * GPU or use several (peer access is enabled where the GPUs allow it).  Each rank
+ * must use its own stream, created non-blocking (cudaStreamNonBlocking, as torch
+ * streams are): the fused exchange spins on the device until every rank's partition
+ * kernel has stored its ops, so ranks serialised on one stream would wait out the
+ * exchange timeout.  Collectives meet at a host barrier (timeout 120 s, then
+ * DG_ERR_NCCL and the handle goes bad).  The group must outlive its handles.
+ * Host-only object: creating it needs no GPU. */
+DG_API dg_status dg_group_create(int32_t nranks, dg_group* out);
+DG_API dg_status dg_group_destroy(dg_group group);
 
 /* Create a graph of `num_vertices` vertices (global capacity; IDs
  * 0..num_vertices-1 all exist, with empty adjacency lists).
@@ -259,6 +285,29 @@ DG_API dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* s
  * Requires nranks == 1 (each GPU holds a whole replica). */
 DG_API dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t* count,
                                    void* stream);
+
+/* Structural invariants of the tables (debug / test; not on the hot path).  Counts
+ * violations of what the lock-free insert's correctness rests on:
+ *   empty_not_suffix   chains with a key after an EMPTY slot ("empty locations can
+ *                      only exist at the end of each bucket's list")
+ *   misplaced_keys     live keys outside the chain their hash selects
+ *   duplicate_keys     repeated live keys inside a chain (fn3)
+ *   self_loops, keys_out_of_range (Alg1:L3; Q7)
+ *   owner_mismatch     buckets whose owner word is not their row
+ *   degree_mismatch    rows whose degree differs from their live keys
+ *   broken_chains      chains longer than the pool (a cycle)
+ * and reports what it walked (rows, chains, buckets, live_pairs, tombstones).
+ * Chains longer than 64 buckets are not checked for duplicates (counted in
+ * dup_unchecked_chains).  first_bad_row = lowest local row with a violation, or
+ * UINT64_MAX.  Stream-ordered after every earlier batch; synchronises `stream`.
+ * Local to the calling rank. */
+typedef struct dg_invariants {
+  uint64_t rows, chains, buckets, live_pairs, tombstones;
+  uint64_t empty_not_suffix, misplaced_keys, duplicate_keys, self_loops, keys_out_of_range,
+      owner_mismatch, degree_mismatch, broken_chains, dup_unchecked_chains;
+  uint64_t first_bad_row;
+} dg_invariants;
+DG_API dg_status dg_check_invariants(dg_graph g, dg_invariants* out, void* stream);
 
 /* ------------------------------------------------------------ instrumentation --
  * Off by default; used by bench.py.  While enabled, every probe-kernel launch of an

@@ -24,6 +24,7 @@ DG_FLAG_NO_TOMBSTONE_REUSE = 1
 DG_FLAG_FORCE_ROUTER = 2
 DG_FLAG_SET = 4
 DG_FLAG_ADAPTIVE = 8
+DG_FLAG_COPY_EXCHANGE = 16
 
 VP = ctypes.c_void_p
 U64 = ctypes.c_uint64
@@ -43,6 +44,7 @@ class dg_config(ctypes.Structure):
         ("nranks", ctypes.c_int32),
         ("flags", ctypes.c_uint32),
         ("nccl_unique_id", ctypes.c_void_p),
+        ("group", ctypes.c_void_p),
     ]
 
 
@@ -75,11 +77,20 @@ class dg_profile(ctypes.Structure):
     ]
 
 
+class dg_invariants(ctypes.Structure):
+    _fields_ = [(n, ctypes.c_uint64) for n in (
+        "rows", "chains", "buckets", "live_pairs", "tombstones", "empty_not_suffix",
+        "misplaced_keys", "duplicate_keys", "self_loops", "keys_out_of_range", "owner_mismatch",
+        "degree_mismatch", "broken_chains", "dup_unchecked_chains", "first_bad_row")]
+
+
 # (name, restype, argtypes) — every entry point declared in include/dg.h
 SIGNATURES = [
     ("dg_config_init", None, [ctypes.POINTER(dg_config)]),
     ("dg_status_string", ctypes.c_char_p, [ctypes.c_int]),
     ("dg_get_unique_id", ctypes.c_int, [VP]),
+    ("dg_group_create", ctypes.c_int, [ctypes.c_int32, ctypes.POINTER(VP)]),
+    ("dg_group_destroy", ctypes.c_int, [VP]),
     ("dg_create", ctypes.c_int, [ctypes.POINTER(dg_config), U64, VP, VP, ctypes.POINTER(VP)]),
     ("dg_destroy", ctypes.c_int, [VP]),
     ("dg_num_vertices", ctypes.c_int, [VP, P_U64, P_U64]),
@@ -94,6 +105,7 @@ SIGNATURES = [
     ("dg_batch_status", ctypes.c_int, [VP, VP]),
     ("dg_triangle_count", ctypes.c_int, [VP, U32, U32, P_U64, VP]),
     ("dg_flush_tombstones", ctypes.c_int, [VP, P_U64, VP]),
+    ("dg_check_invariants", ctypes.c_int, [VP, ctypes.POINTER(dg_invariants), VP]),
     ("dg_profile_enable", ctypes.c_int, [VP, ctypes.c_int]),
     ("dg_profile_read", ctypes.c_int, [VP, ctypes.POINTER(dg_profile), VP]),
 ]

@@ -327,6 +327,24 @@ void note_launch(dg_graph g, u64 need, cudaStream_t s) {
 
 }  // namespace
 
+// ops a retry-mode launch records before it runs the whole batch again (128 MB)
+u64 retry_cap_max() {
+  static const u64 v = std::getenv("DG_TEST_RETRY_CAP")
+                           ? std::strtoull(std::getenv("DG_TEST_RETRY_CAP"), nullptr, 10)
+                           : (1ull << 24);
+  return v;
+}
+
+dg_status prepare_insert(dg_graph g, u64 n_ops, cudaStream_t s) {
+  if (n_ops == 0) return DG_OK;
+  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
+  bool retry_mode = false;
+  DG_TRY(plan_capacity(g, n_ops + dg::max_groups(g->G, g->sms), s, &retry_mode));
+  if (retry_mode) DG_TRY(ensure_retry(g, 0, std::min<u64>(n_ops, retry_cap_max())));
+  DG_TRY(ensure_ret(g, n_ops));
+  return DG_OK;
+}
+
 // insert n edges already resident on this GPU (their sources are local rows)
 dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n, bool mirror,
                        u32 epoch, cudaStream_t s) {
@@ -344,10 +362,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   // when more fail, the whole batch runs again after the pool grows (an insert batch
   // is idempotent: re-applied keys are replaced by a weight of the same batch, Q1,
   // and only keys still missing count as added).
-  static const u64 retry_cap_max = std::getenv("DG_TEST_RETRY_CAP")
-                                       ? std::strtoull(std::getenv("DG_TEST_RETRY_CAP"), nullptr, 10)
-                                       : (1ull << 24);
-  const u64 rcap = retry_mode ? std::min<u64>(n_ops, retry_cap_max) : 0;
+  const u64 rcap = retry_mode ? std::min<u64>(n_ops, retry_cap_max()) : 0;
   if (rcap) DG_TRY(ensure_retry(g, 0, rcap));
   DG_TRY(ensure_ret(g, n_ops));
   t = g->tables();
@@ -700,9 +715,9 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
     return DG_ERR_INVALID_ARGUMENT;
   if (!(cfg->load_factor > 0.0f) || !(cfg->load_factor < 1000.0f)) return DG_ERR_INVALID_ARGUMENT;
   if (cfg->nranks < 1 || cfg->rank < 0 || cfg->rank >= cfg->nranks) return DG_ERR_INVALID_ARGUMENT;
-  if (cfg->nranks > 1 && !cfg->nccl_unique_id) return DG_ERR_INVALID_ARGUMENT;
-  if (cfg->flags &
-      ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER | DG_FLAG_SET | DG_FLAG_ADAPTIVE))
+  if (cfg->nranks > 1 && !cfg->nccl_unique_id && !cfg->group) return DG_ERR_INVALID_ARGUMENT;
+  if (cfg->flags & ~(DG_FLAG_NO_TOMBSTONE_REUSE | DG_FLAG_FORCE_ROUTER | DG_FLAG_SET |
+                     DG_FLAG_ADAPTIVE | DG_FLAG_COPY_EXCHANGE))
     return DG_ERR_INVALID_ARGUMENT;
 
   dg_graph g = new (std::nothrow) dg_graph_s();
@@ -763,11 +778,11 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
     return fail(DG_ERR_CUDA);
   if (cudaMalloc(&g->stats_dev, sizeof(dg::StatsOut)) != cudaSuccess) return fail(DG_ERR_CUDA);
 
-  if (g->nranks > 1) {
+  if (g->nranks > 1 || (cfg->group && (cfg->flags & DG_FLAG_FORCE_ROUTER))) {
     dg_status st = dg::router_create(g, cfg->nccl_unique_id, &g->router);
     if (st != DG_OK) return fail(st);
   } else if (cfg->flags & DG_FLAG_FORCE_ROUTER) {
-    // diagnostic: route a single-GPU graph through the NCCL path (1-rank communicator)
+    // diagnostic: route a single-GPU graph through the router (1-rank NCCL communicator)
     char id[128];
     dg_status st = dg::router_unique_id(id);
     if (st == DG_OK) st = dg::router_create(g, id, &g->router);
@@ -1278,6 +1293,20 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   dg::prof_mark(g, dg::PROF_TC, s);
   DG_TRY(read_ctl(g, s));
   *count = g->hctl->count;
+  return DG_OK;
+}
+
+dg_status dg_check_invariants(dg_graph g, dg_invariants* out, void* stream) {
+  DG_TRY(check_handle(g));
+  if (!out) return DG_ERR_INVALID_ARGUMENT;
+  static_assert(sizeof(dg_invariants) == sizeof(dg::InvariantsOut), "dg_invariants layout");
+  cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
+  dg::InvariantsOut* d = nullptr;
+  DG_CK(cudaMallocAsync(&d, sizeof(*d), s));
+  DG_CK(dg::launch_check(g->lay, g->tables(), g->nv, g->rank, d, g->sms, s));
+  DG_CK(cudaMemcpyAsync(out, d, sizeof(*d), cudaMemcpyDeviceToHost, s));
+  DG_CK(cudaFreeAsync(d, s));
+  DG_CK(cudaStreamSynchronize(s));
   return DG_OK;
 }
 

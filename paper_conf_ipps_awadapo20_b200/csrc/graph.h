@@ -131,6 +131,9 @@ dg_status rehash_hot(dg_graph g, cudaStream_t s);
 dg_status rehash_rows(dg_graph g, uint32_t n, bool flush, cudaStream_t s);
 dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
                        uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s);
+// the allocation part of local_insert for n_ops ops, done ahead (the router calls it
+// before the exchange so nothing device-synchronising runs after its scatter)
+dg_status prepare_insert(dg_graph g, uint64_t n_ops, cudaStream_t s);
 dg_status local_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
                        bool mirror, uint32_t epoch, cudaStream_t s);
 dg_status local_query(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,

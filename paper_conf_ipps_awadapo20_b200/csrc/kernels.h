@@ -90,6 +90,16 @@ struct StatsOut {
 };
 cudaError_t launch_stats(int lay, const Tables& t, StatsOut* out, u32* big, int sms, cudaStream_t s);
 
+// structural invariants (kernels_check.cu); field order = dg_invariants (include/dg.h)
+struct InvariantsOut {
+  unsigned long long rows, chains, buckets, live_pairs, tombstones;
+  unsigned long long empty_not_suffix, misplaced_keys, duplicate_keys, self_loops,
+      keys_out_of_range, owner_mismatch, degree_mismatch, broken_chains, dup_unchecked_chains;
+  unsigned long long first_bad_row;
+};
+cudaError_t launch_check(int lay, const Tables& t, u64 nv, u32 rank, InvariantsOut* out, int sms,
+                         cudaStream_t s);
+
 // vertex deletion (kernels_graph.cu)
 // coarse filter of the deleted-vertex bitmap (bit = id >> fshift), kept in shared
 // memory by the purge sweep

@@ -1,44 +1,45 @@
-// router.cu — multi-GPU batch router (a2, a11 of DESIGN.md §2): shards every edge
-// op by source vertex, owner(u) = u mod P, local row = u / P, over NCCL.
+// router.cu — multi-GPU batch router (a2, a11 of DESIGN.md §1): shards every edge
+// op by source vertex, owner(u) = u mod P, local row = u / P.
 //
 // Per routed batch (each rank holds its own slice of the batch):
 //   1. k_route_count: one pass over the slice — range validation (Q7) and a
-//      per-block histogram of owners (block-contiguous op ranges);
+//      per-block histogram of owners over the VALID ops (block-contiguous ranges);
 //   2. k_route_scan: per-block send offsets, grouped by destination rank;
-//   3. k_route_scatter: ops written to the send buffers (SoA) at their offsets;
-//      queries keep pos[i] = send position to put answers back in order;
-//   4. ncclAllGather of each rank's P send counts + its validation flag: every
-//      rank learns its receive counts and the batch-wide verdict (all-or-nothing
-//      before any mutation);
-//   5. grouped ncclSend/ncclRecv of (src, dst[, w]) to the owners;
+//   3. k_route_scatter: valid ops written to the send buffers (SoA) at their
+//      offsets; queries keep pos[i] = send position (or kNoPos for an out-of-range
+//      query) to put answers back in the caller's order;
+//   4. all-gather of each rank's P send counts + its validation flag: every rank
+//      learns its receive counts and the batch-wide verdict (a mutating batch is
+//      all-or-nothing before any mutation; a query batch answers its in-range ops
+//      and reports the batch as rejected, exactly as at P = 1);
+//   5. grouped send/recv of (src, dst[, w]) to the owners;
 //   6. the local probe kernel on the received ops;
 //   7. queries: (found, weight) travel back through the reversed exchange and are
 //      scattered to the caller's order through pos.
-// Fused exchange (default when every peer's memory can be mapped; DG_ROUTER=nccl
-// selects the path above): steps 3 and 5 become ONE kernel.  Each rank owns a
-// receive window (plain device memory exported with CUDA IPC and mapped by every
-// peer over NVLink / NVSwitch); after the counts all-gather every rank knows where
-// its ops land in every owner's window, and k_route_scatter stores each op straight
-// into its owner's window (peer stores) instead of a local send buffer.  The last
-// block of the kernel fences (system scope) and bumps an arrival counter in every
-// peer's window header; a one-thread kernel on the owner waits for P arrivals
-// before the probe kernel reads the window.  Query answers return the same way:
-// the owner's k_route_return stores (found, weight) into each asker's answer window
-// and signals it.  The next batch's counts all-gather orders window reuse (a rank
-// reaches it only after its kernels of the previous batch completed).
-// The paper has a single GPU; this layer is the B200-node extension
-// named by BASELINE.json's north_star.  NCCL is loaded with dlopen (the copy torch
-// already loaded when present), so libdg.so has no link-time NCCL dependency.
-#include <dlfcn.h>
-
+// Fused exchange (default when every peer's memory can be mapped; DG_ROUTER=nccl or
+// DG_FLAG_COPY_EXCHANGE selects the path above): steps 3 and 5 become ONE kernel.
+// Each rank owns a receive window (plain device memory, mapped by every peer over
+// NVLink / NVSwitch: CUDA IPC between processes, plain pointers inside one process);
+// after the counts all-gather every rank knows where its ops land in every owner's
+// window, and k_route_scatter_fused stores each op straight into its owner's window
+// (peer stores) instead of a local send buffer.  The last block of the kernel fences
+// (system scope) and bumps an arrival counter in every peer's window header; a
+// one-thread kernel on the owner waits for P arrivals before the probe kernel reads
+// the window.  Query answers return the same way: the owner's k_route_return stores
+// (found, weight) into each asker's answer window and signals it.  The next batch's
+// counts all-gather orders window reuse (a rank reaches it only after its kernels of
+// the previous batch completed).  A batch larger than the windows triggers a
+// collective window re-setup; if that fails on any rank, every rank moves to the copy
+// exchange for this batch and the rest of the handle's life.
+// The transports (NCCL, or an in-process rank group on one or several GPUs) are in
+// comm.cu.  The paper has a single GPU; this layer is the B200-node
+// extension named by BASELINE.json's north_star.
 #include <algorithm>
 #include <cstdlib>
 #include <cstring>
-#include <mutex>
 #include <vector>
 
-#include <nccl.h>
-
+#include "comm.h"
 #include "graph.h"
 #include "kernels.h"
 #include "router.h"
@@ -46,46 +47,10 @@
 namespace dg {
 namespace {
 
-struct Nccl {
-  decltype(&ncclGetUniqueId) GetUniqueId = nullptr;
-  decltype(&ncclCommInitRank) CommInitRank = nullptr;
-  decltype(&ncclCommDestroy) CommDestroy = nullptr;
-  decltype(&ncclSend) Send = nullptr;
-  decltype(&ncclRecv) Recv = nullptr;
-  decltype(&ncclGroupStart) GroupStart = nullptr;
-  decltype(&ncclGroupEnd) GroupEnd = nullptr;
-  decltype(&ncclAllGather) AllGather = nullptr;
-  decltype(&ncclAllReduce) AllReduce = nullptr;
-  bool ok = false;
-};
-
-template <typename F>
-bool sym(void* h, const char* name, F& f) {
-  f = reinterpret_cast<F>(dlsym(h, name));
-  return f != nullptr;
-}
-
-const Nccl& nccl() {
-  static Nccl n;
-  static std::once_flag once;
-  std::call_once(once, [] {
-    void* h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_NOLOAD);
-    if (!h && std::getenv("DG_NCCL_LIB")) h = dlopen(std::getenv("DG_NCCL_LIB"), RTLD_NOW);
-    if (!h) h = dlopen("libnccl.so.2", RTLD_NOW);
-    if (!h) h = dlopen("libnccl.so", RTLD_NOW);
-    if (!h) return;
-    n.ok = sym(h, "ncclGetUniqueId", n.GetUniqueId) && sym(h, "ncclCommInitRank", n.CommInitRank) &&
-           sym(h, "ncclCommDestroy", n.CommDestroy) && sym(h, "ncclSend", n.Send) &&
-           sym(h, "ncclRecv", n.Recv) && sym(h, "ncclGroupStart", n.GroupStart) &&
-           sym(h, "ncclGroupEnd", n.GroupEnd) && sym(h, "ncclAllGather", n.AllGather) &&
-           sym(h, "ncclAllReduce", n.AllReduce);
-  });
-  return n;
-}
-
 constexpr int kRouteBlocks = 1184;  // 148 SMs x 8
 constexpr int kRouteThreads = 256;
 constexpr int kMaxRanks = 64;
+constexpr u64 kNoPos = ~0ull;       // pos[] of a query that was not routed (out of range)
 
 // ------------------------------------------------------------------ kernels ----
 __device__ __forceinline__ void op_at(const u32* src, const u32* dst, u64 n, u64 j, u32& u,
@@ -142,7 +107,8 @@ __global__ void k_route_scan(const u32* blockcnt, u32 nblocks, u32 P, u64* offs,
 }
 
 __global__ void k_route_scatter(const u32* src, const u32* dst, const u32* w, u64 n, u64 n_ops,
-                                u32 P, const u64* offs, u32* ssrc, u32* sdst, u32* sw, u64* pos) {
+                                u64 nv, u32 P, const u64* offs, u32* ssrc, u32* sdst, u32* sw,
+                                u64* pos) {
   __shared__ unsigned long long cur[kMaxRanks];
   for (u32 p = threadIdx.x; p < P; p += blockDim.x) cur[p] = offs[blockIdx.x * P + p];
   __syncthreads();
@@ -152,6 +118,10 @@ __global__ void k_route_scatter(const u32* src, const u32* dst, const u32* w, u6
     u32 u, v;
     u64 i;
     op_at(src, dst, n, j, u, v, i);
+    if ((u64)u >= nv || (u64)v >= nv) {  // not routed (query batches only get here)
+      if (pos) pos[j] = kNoPos;
+      continue;
+    }
     const u64 slot = atomicAdd(&cur[u % P], 1ull);
     ssrc[slot] = u;
     sdst[slot] = v;
@@ -160,13 +130,15 @@ __global__ void k_route_scatter(const u32* src, const u32* dst, const u32* w, u6
   }
 }
 
+// answers back to the caller's order (Q19: an unrouted out-of-range query answers 0)
 __global__ void k_route_unpermute(const u64* pos, u64 n, const uint8_t* fs, const u32* ws,
                                   uint8_t* found, u32* wout) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
   for (u64 j = (u64)blockIdx.x * blockDim.x + threadIdx.x; j < n; j += stride) {
     const u64 s = pos[j];
-    found[j] = fs[s];
-    if (wout) wout[j] = ws[s];
+    const bool ok = s != kNoPos;
+    found[j] = ok ? fs[s] : 0;
+    if (wout) wout[j] = ok ? ws[s] : 0u;
   }
 }
 
@@ -218,10 +190,11 @@ __device__ __forceinline__ void signal_peers(unsigned int* done, unsigned long l
   }
 }
 
-// steps 3 + 5 in one kernel: ops are stored straight into their owners' windows
+// steps 3 + 5 in one kernel: valid ops are stored straight into their owners' windows
 __global__ void k_route_scatter_fused(const u32* src, const u32* dst, const u32* w, u64 n,
-                                      u64 n_ops, u32 P, const u64* offs, const RouteTable* tb,
-                                      bool with_w, u64* pos, unsigned int* done) {
+                                      u64 n_ops, u64 nv, u32 P, const u64* offs,
+                                      const RouteTable* tb, bool with_w, u64* pos,
+                                      unsigned int* done) {
   __shared__ unsigned long long cur[kMaxRanks];
   for (u32 p = threadIdx.x; p < P; p += blockDim.x) cur[p] = offs[blockIdx.x * P + p];
   __syncthreads();
@@ -231,6 +204,10 @@ __global__ void k_route_scatter_fused(const u32* src, const u32* dst, const u32*
     u32 u, v;
     u64 i;
     op_at(src, dst, n, j, u, v, i);
+    if ((u64)u >= nv || (u64)v >= nv) {
+      if (pos) pos[j] = kNoPos;
+      continue;
+    }
     const u32 p = u % P;
     const u64 slot = atomicAdd(&cur[p], 1ull);
     const u64 at = tb->base[p] + (slot - tb->soff[p]);
@@ -285,29 +262,28 @@ __global__ void k_route_return(const uint8_t* found, const u32* wt, u32 P, const
 }  // namespace
 
 struct Router {
-  ncclComm_t comm = nullptr;
+  Comm* comm = nullptr;
   u32 P = 1, rank = 0;
   struct Buf {
     void* p = nullptr;
     size_t bytes = 0;
   };
   Buf ssrc, sdst, sw, rsrc, rdst, rw, pos, blockcnt, offs, meta_all, flag, rfound, rwt, sfound,
-      swt, ids, ids2, scalar;
+      swt, ids, ids2, scalar, table;
   u64* h_meta = nullptr;  // pinned, P*(P+1)
   u64* h_scalar = nullptr;
   std::vector<u64> scnt, soff, rcnt, roff;
-  // fused exchange: receive window [WinHdr | src | dst | w | found | wt], wcap ops
+  // fused exchange: receive window [WinHdr | src | dst | w | wt | found], wcap ops
   bool fused = false;
+  bool copy_only = false;          // DG_ROUTER=nccl / DG_FLAG_COPY_EXCHANGE, or a failed setup
+  u32 setups = 0;                  // window setups so far
   u64 wcap = 0;
   char* win = nullptr;
   char* peer[kMaxRanks] = {};      // mapped windows of every rank (self: win)
   std::vector<char*> retired;      // outgrown windows (peers may still map them)
   unsigned long long arrive_expected = 0, ans_expected = 0;
-  Buf table;
   RouteTable* h_table = nullptr;   // pinned
 };
-
-dg_status allreduce_u64(dg_graph g, u64* v, ncclRedOp_t op, cudaStream_t s);
 
 namespace {
 
@@ -329,11 +305,13 @@ cudaError_t grow(Router::Buf& b, size_t bytes) {
       return DG_ERR_CUDA;                 \
     }                                     \
   } while (0)
-#define RT_NC(expr)                       \
+// a failed collective leaves the ranks out of step: the handle goes bad
+#define RT_CM(expr)                       \
   do {                                    \
-    if ((expr) != ncclSuccess) {          \
+    const dg_status st_ = (expr);         \
+    if (st_ != DG_OK) {                   \
       g->bad = true;                      \
-      return DG_ERR_NCCL;                 \
+      return st_;                         \
     }                                     \
   } while (0)
 
@@ -343,11 +321,14 @@ T* as(Router::Buf& b) {
 }
 
 // Steps 1-4: partition this rank's slice by owner and agree on counts/validity.
-// Returns DG_ERR_VERTEX_OUT_OF_RANGE (on every rank) if any rank saw a bad ID.
+// Returns DG_ERR_VERTEX_OUT_OF_RANGE (on every rank) if any rank saw a bad ID; the
+// counts then cover the valid ops only (what a query batch still routes).
+// Everything that may synchronise the device (allocation) happens BEFORE the counts
+// exchange: after it, an in-process rank group has ranks spinning on the device for
+// this rank's partition kernel (see the fused exchange).
 dg_status route_partition(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n,
                           bool mirror, bool with_w, bool keep_pos, cudaStream_t s) {
   Router& r = *g->router;
-  const Nccl& N = nccl();
   const u32 P = r.P;
   const u64 n_ops = mirror ? 2 * n : n;
   if (!r.fused) {  // the fused path scatters after the counts exchange, into the windows
@@ -368,14 +349,8 @@ dg_status route_partition(dg_graph g, const u32* src, const u32* dst, const u32*
   k_route_scan<<<1, 64, 0, s>>>(as<u32>(r.blockcnt), kRouteBlocks, P, as<u64>(r.offs), meta_mine,
                                 as<u32>(r.flag));
   note_kernel(1);
-  if (!r.fused) {
-    k_route_scatter<<<kRouteBlocks, kRouteThreads, 0, s>>>(
-        src, dst, w, n, n_ops, P, as<u64>(r.offs), as<u32>(r.ssrc), as<u32>(r.sdst),
-        with_w ? as<u32>(r.sw) : nullptr, keep_pos ? as<u64>(r.pos) : nullptr);
-    note_kernel(1);
-  }
   RT_CK(cudaGetLastError());
-  RT_NC(N.AllGather(meta_mine, r.meta_all.p, P + 1, ncclUint64, r.comm, s));
+  RT_CM(r.comm->allgather(meta_mine, r.meta_all.p, (P + 1) * 8, s));
   RT_CK(cudaMemcpyAsync(r.h_meta, r.meta_all.p, (size_t)P * (P + 1) * 8, cudaMemcpyDeviceToHost, s));
   RT_CK(cudaMemcpyAsync(r.h_scalar + 1, &g->ctl->route_timeout, 4, cudaMemcpyDeviceToHost, s));
   RT_CK(cudaStreamSynchronize(s));
@@ -400,10 +375,25 @@ dg_status route_partition(dg_graph g, const u32* src, const u32* dst, const u32*
   return bad ? DG_ERR_VERTEX_OUT_OF_RANGE : DG_OK;
 }
 
+// Step 3 of the copy exchange: valid ops into the local send buffers.
+dg_status route_scatter_copy(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n,
+                             bool mirror, bool with_w, bool keep_pos, cudaStream_t s) {
+  Router& r = *g->router;
+  const u64 n_ops = mirror ? 2 * n : n;
+  RT_CK(grow(r.ssrc, n_ops * 4 + 4));
+  RT_CK(grow(r.sdst, n_ops * 4 + 4));
+  if (with_w) RT_CK(grow(r.sw, n_ops * 4 + 4));
+  k_route_scatter<<<kRouteBlocks, kRouteThreads, 0, s>>>(
+      src, dst, w, n, n_ops, g->nv, r.P, as<u64>(r.offs), as<u32>(r.ssrc), as<u32>(r.sdst),
+      with_w ? as<u32>(r.sw) : nullptr, keep_pos ? as<u64>(r.pos) : nullptr);
+  note_kernel(1);
+  RT_CK(cudaGetLastError());
+  return DG_OK;
+}
+
 // Step 5: ship the partitioned ops to their owners.
 dg_status route_exchange(dg_graph g, bool with_w, cudaStream_t s) {
   Router& r = *g->router;
-  const Nccl& N = nccl();
   const u64 total = r.roff[r.P];
   RT_CK(grow(r.rsrc, total * 4 + 4));
   RT_CK(grow(r.rdst, total * 4 + 4));
@@ -416,15 +406,15 @@ dg_status route_exchange(dg_graph g, bool with_w, cudaStream_t s) {
     if (r.scnt[r.rank])
       RT_CK(cudaMemcpyAsync(as<u32>(*rb[k]) + r.roff[r.rank], as<u32>(*sb[k]) + r.soff[r.rank],
                             r.scnt[r.rank] * 4, cudaMemcpyDeviceToDevice, s));
-  RT_NC(N.GroupStart());
+  RT_CM(r.comm->group_start());
   for (u32 q = 0; q < r.P; ++q) {
     if (q == r.rank) continue;
     for (int k = 0; k < arrays; ++k) {
-      if (r.scnt[q]) RT_NC(N.Send(as<u32>(*sb[k]) + r.soff[q], r.scnt[q], ncclUint32, q, r.comm, s));
-      if (r.rcnt[q]) RT_NC(N.Recv(as<u32>(*rb[k]) + r.roff[q], r.rcnt[q], ncclUint32, q, r.comm, s));
+      if (r.scnt[q]) RT_CM(r.comm->send(as<u32>(*sb[k]) + r.soff[q], r.scnt[q] * 4, q, s));
+      if (r.rcnt[q]) RT_CM(r.comm->recv(as<u32>(*rb[k]) + r.roff[q], r.rcnt[q] * 4, q, s));
     }
   }
-  RT_NC(N.GroupEnd());
+  RT_CM(r.comm->group_end(s));
   return DG_OK;
 }
 
@@ -447,62 +437,32 @@ WinPtrs win_ptrs(char* base, u64 cap) {
   return x;
 }
 
-void close_peers(Router& r) {
-  for (u32 q = 0; q < r.P; ++q) {
-    if (q != r.rank && r.peer[q]) cudaIpcCloseMemHandle(r.peer[q]);
-    r.peer[q] = nullptr;
-  }
-}
-
-// Collective: every rank allocates a window of `cap` ops and maps every peer's
-// (CUDA IPC handles all-gathered over NCCL).  If any rank cannot map a peer, all
-// ranks fall back to the NCCL exchange.
+// Collective: every rank allocates a window of `cap` ops and maps every peer's.  If
+// any rank cannot map a peer, every rank falls back to the copy exchange for good.
 dg_status window_setup(dg_graph g, u64 cap, cudaStream_t s) {
   Router& r = *g->router;
-  const Nccl& N = nccl();
-  close_peers(r);
+  r.comm->unmap_windows(r.peer);
   if (r.win) r.retired.push_back(r.win);
   r.win = nullptr;
   r.fused = false;
   RT_CK(cudaMalloc(&r.win, kWinHdr + cap * 17 + 64));
   RT_CK(cudaMemsetAsync(r.win, 0, kWinHdr, s));
+  // the owner's answer buffers hold up to a window of ops: sized here, so a fused
+  // query batch allocates nothing after its counts exchange
+  RT_CK(grow(r.rfound, cap + 1));
+  RT_CK(grow(r.rwt, cap * 4 + 4));
+  RT_CK(cudaStreamSynchronize(s));
   r.wcap = cap;
   r.arrive_expected = r.ans_expected = 0;
-  r.peer[r.rank] = r.win;
-  int fail = 0;
-  if (r.P > 1) {
-    static_assert(sizeof(cudaIpcMemHandle_t) == 64, "IPC handle size");
-    cudaIpcMemHandle_t mine;
-    RT_CK(grow(r.scalar, (size_t)(r.P + 1) * 64 + 64));
-    char* hbuf = as<char>(r.scalar);
-    if (cudaIpcGetMemHandle(&mine, r.win) != cudaSuccess) {
-      cudaGetLastError();
-      fail = 1;
-      std::memset(&mine, 0, sizeof(mine));
-    }
-    RT_CK(cudaMemcpyAsync(hbuf + (size_t)r.P * 64, &mine, 64, cudaMemcpyHostToDevice, s));
-    RT_NC(N.AllGather(hbuf + (size_t)r.P * 64, hbuf, 64, ncclUint8, r.comm, s));
-    std::vector<cudaIpcMemHandle_t> all(r.P);
-    RT_CK(cudaMemcpyAsync(all.data(), hbuf, (size_t)r.P * 64, cudaMemcpyDeviceToHost, s));
-    RT_CK(cudaStreamSynchronize(s));
-    for (u32 q = 0; q < r.P && !fail; ++q) {
-      if (q == r.rank) continue;
-      void* p = nullptr;
-      if (cudaIpcOpenMemHandle(&p, all[q], cudaIpcMemLazyEnablePeerAccess) != cudaSuccess) {
-        cudaGetLastError();
-        fail = 1;
-      } else {
-        r.peer[q] = reinterpret_cast<char*>(p);
-      }
-    }
-    u64 v = fail;
-    dg_status st = allreduce_u64(g, &v, ncclMax, s);
-    if (st != DG_OK) return st;
-    fail = v != 0;
-  }
+  bool fail = false;
+  RT_CM(r.comm->map_windows(r.win, r.peer, &fail, s));
+  // test hook: a failed re-setup (every rank reads the same environment)
+  if (r.setups > 0 && std::getenv("DG_TEST_FUSED_REGROW_FAIL")) fail = true;
+  ++r.setups;
   if (fail) {
-    close_peers(r);
-    return DG_OK;  // NCCL exchange from now on
+    r.comm->unmap_windows(r.peer);
+    r.copy_only = true;
+    return DG_OK;  // copy exchange from now on
   }
   r.fused = true;
   return DG_OK;
@@ -510,12 +470,16 @@ dg_status window_setup(dg_graph g, u64 cap, cudaStream_t s) {
 
 // Fused steps 3 + 5 for the counts agreed by route_partition: ops land in their
 // owners' windows; returns once the local window is complete (stream-ordered).
+// *fell_back = the windows had to grow and the re-setup failed on some rank: the
+// caller continues with the copy exchange (route_scatter_copy + route_exchange).
 dg_status route_fused_scatter(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n,
-                              bool mirror, bool with_w, bool keep_pos, cudaStream_t s) {
+                              bool mirror, bool with_w, bool keep_pos, bool* fell_back,
+                              cudaStream_t s) {
   Router& r = *g->router;
   const u32 P = r.P, me = r.rank;
   const u64 n_ops = mirror ? 2 * n : n;
   const u64* M = r.h_meta;  // row q: rank q's send counts per owner
+  *fell_back = false;
   // the same capacity decision on every rank: largest inbound or outbound total
   u64 need = 0;
   for (u32 p = 0; p < P; ++p) {
@@ -529,7 +493,10 @@ dg_status route_fused_scatter(dg_graph g, const u32* src, const u32* dst, const 
   if (need > r.wcap) {
     dg_status st = window_setup(g, std::max<u64>(need + need / 4, 2 * r.wcap), s);
     if (st != DG_OK) return st;
-    if (!r.fused) return DG_ERR_UNSUPPORTED;  // caller retries over NCCL
+    if (!r.fused) {
+      *fell_back = true;
+      return DG_OK;
+    }
   }
   RouteTable& T = *r.h_table;
   for (u32 p = 0; p < P; ++p) {
@@ -550,16 +517,44 @@ dg_status route_fused_scatter(dg_graph g, const u32* src, const u32* dst, const 
     T.roff[p] = r.roff[p];
   }
   T.roff[P] = r.roff[P];
-  RT_CK(grow(r.table, sizeof(RouteTable)));
   RT_CK(cudaMemcpyAsync(r.table.p, r.h_table, sizeof(RouteTable), cudaMemcpyHostToDevice, s));
   const WinPtrs mine = win_ptrs(r.win, r.wcap);
   k_route_scatter_fused<<<kRouteBlocks, kRouteThreads, 0, s>>>(
-      src, dst, w, n, n_ops, P, as<u64>(r.offs), as<RouteTable>(r.table), with_w,
+      src, dst, w, n, n_ops, g->nv, P, as<u64>(r.offs), as<RouteTable>(r.table), with_w,
       keep_pos ? as<u64>(r.pos) : nullptr, &mine.hdr->done);
   r.arrive_expected += P;
   k_route_wait<<<1, 32, 0, s>>>(&mine.hdr->arrive, r.arrive_expected, g->ctl);
   note_kernel(2);
   RT_CK(cudaGetLastError());
+  return DG_OK;
+}
+
+// the ops this rank owns for the current batch, wherever the exchange left them
+struct Received {
+  const u32 *src, *dst, *w;
+};
+
+// Steps 3 + 5 by whichever exchange is active (fused, or copy; fused falls back to
+// copy when its windows cannot grow).
+dg_status route_ops(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n, bool mirror,
+                    bool with_w, bool keep_pos, cudaStream_t s, Received* out, bool* via_window) {
+  Router& r = *g->router;
+  *via_window = false;
+  if (r.fused) {
+    bool fell_back = false;
+    dg_status st = route_fused_scatter(g, src, dst, w, n, mirror, with_w, keep_pos, &fell_back, s);
+    if (st != DG_OK) return st;
+    if (!fell_back) {
+      const WinPtrs x = win_ptrs(r.win, r.wcap);
+      *out = Received{x.src, x.dst, x.w};
+      *via_window = true;
+      return DG_OK;
+    }
+  }
+  dg_status st = route_scatter_copy(g, src, dst, w, n, mirror, with_w, keep_pos, s);
+  if (st != DG_OK) return st;
+  if ((st = route_exchange(g, with_w, s)) != DG_OK) return st;
+  *out = Received{as<u32>(r.rsrc), as<u32>(r.rdst), with_w ? as<u32>(r.rw) : nullptr};
   return DG_OK;
 }
 
@@ -569,34 +564,34 @@ dg_status reset_counters(dg_graph g, cudaStream_t s) {
   return DG_OK;
 }
 
-}  // namespace
-
-dg_status router_unique_id(void* out128) {
-  const Nccl& N = nccl();
-  if (!N.ok) return DG_ERR_UNSUPPORTED;
-  static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId size");
-  ncclUniqueId id;
-  if (N.GetUniqueId(&id) != ncclSuccess) return DG_ERR_NCCL;
-  std::memcpy(out128, &id, sizeof(id));
+// every rank agreed the batch holds an out-of-range ID: record the rejection on the
+// host mirror and the device (read back by dg_batch_status / host-buffer calls)
+dg_status mark_rejected(dg_graph g, u32 epoch, cudaStream_t s) {
+  g->hctl->fail_epoch = std::max(g->hctl->fail_epoch, epoch);
+  g->router->h_scalar[2] = epoch;
+  RT_CK(cudaMemcpyAsync(&g->ctl->fail_epoch, g->router->h_scalar + 2, 4, cudaMemcpyHostToDevice, s));
+  RT_CK(cudaStreamSynchronize(s));  // h_scalar is reused by the next collective
   return DG_OK;
 }
 
+}  // namespace
+
+dg_status router_unique_id(void* out128) { return nccl_unique_id(out128); }
+
 dg_status router_create(dg_graph g, const void* unique_id, Router** out) {
-  const Nccl& N = nccl();
-  if (!N.ok) return DG_ERR_UNSUPPORTED;
   if (g->nranks > (u32)kMaxRanks) return DG_ERR_UNSUPPORTED;
+  Comm* c = nullptr;
+  dg_status st = g->cfg.group ? group_comm_create(g->cfg.group, g->nranks, g->rank, g->device, &c)
+                              : nccl_comm_create(unique_id, g->nranks, g->rank, &c);
+  if (st != DG_OK) return st;
   Router* r = new Router();
+  r->comm = c;
   r->P = g->nranks;
   r->rank = g->rank;
-  ncclUniqueId id;
-  std::memcpy(&id, unique_id, sizeof(id));
-  if (N.CommInitRank(&r->comm, (int)r->P, id, (int)r->rank) != ncclSuccess) {
-    delete r;
-    return DG_ERR_NCCL;
-  }
   if (cudaMallocHost(&r->h_meta, (size_t)(r->P + 1) * (r->P + 1) * 8) != cudaSuccess ||
       cudaMallocHost(&r->h_scalar, 64) != cudaSuccess ||
-      cudaMallocHost(&r->h_table, sizeof(RouteTable)) != cudaSuccess) {
+      cudaMallocHost(&r->h_table, sizeof(RouteTable)) != cudaSuccess ||
+      grow(r->table, sizeof(RouteTable)) != cudaSuccess) {
     router_destroy(r);
     return DG_ERR_CUDA;
   }
@@ -605,21 +600,27 @@ dg_status router_create(dg_graph g, const void* unique_id, Router** out) {
 }
 
 dg_status router_setup_fused(dg_graph g, cudaStream_t s) {
+  Router& r = *g->router;
   const char* mode = std::getenv("DG_ROUTER");
-  if (mode && std::strcmp(mode, "nccl") == 0) return DG_OK;
-  return window_setup(g, 1ull << 20, s);
+  if ((mode && std::strcmp(mode, "nccl") == 0) || (g->cfg.flags & DG_FLAG_COPY_EXCHANGE)) {
+    r.copy_only = true;
+    return DG_OK;
+  }
+  // initial window: 2^20 ops (17 MB); grows collectively with the batches
+  u64 cap = 1ull << 20;
+  if (const char* e = std::getenv("DG_ROUTER_WINDOW_OPS")) cap = std::max<u64>(64, std::strtoull(e, nullptr, 10));
+  return window_setup(g, cap, s);
 }
 
 bool router_fused(const Router* r) { return r && r->fused; }
 
 void router_destroy(Router* r) {
   if (!r) return;
-  const Nccl& N = nccl();
-  close_peers(*r);
+  if (r->comm) r->comm->unmap_windows(r->peer);
   if (r->win) cudaFree(r->win);
   for (char* p : r->retired) cudaFree(p);
   if (r->h_table) cudaFreeHost(r->h_table);
-  if (r->comm && N.ok) N.CommDestroy(r->comm);
+  delete r->comm;
   Router::Buf* all[] = {&r->ssrc, &r->sdst, &r->sw, &r->rsrc, &r->rdst, &r->rw, &r->pos,
                         &r->blockcnt, &r->offs, &r->meta_all, &r->flag, &r->rfound, &r->rwt,
                         &r->sfound, &r->swt, &r->ids, &r->ids2, &r->scalar, &r->table};
@@ -635,117 +636,108 @@ dg_status router_insert(dg_graph g, const u32* src, const u32* dst, const u32* w
   dg_status st = route_partition(g, src, dst, w, n, !g->directed, true, false, s);
   if (st == DG_ERR_VERTEX_OUT_OF_RANGE) {
     // every rank agrees: no mutation; report it like the single-GPU path
-    g->hctl->fail_epoch = epoch;
-    RT_CK(cudaMemcpyAsync(&g->ctl->fail_epoch, &epoch, 4, cudaMemcpyHostToDevice, s));
+    if ((st = mark_rejected(g, epoch, s)) != DG_OK) return st;
     return reset_counters(g, s);
   }
   if (st != DG_OK) return st;
   Router& r = *g->router;
-  if (r.fused) {
-    if ((st = route_fused_scatter(g, src, dst, w, n, !g->directed, true, false, s)) != DG_OK)
-      return st;
-    if ((st = reset_counters(g, s)) != DG_OK) return st;
-    const WinPtrs x = win_ptrs(r.win, r.wcap);
-    return local_insert(g, x.src, x.dst, x.w, r.roff[r.P], false, epoch, s);
-  }
-  if ((st = route_exchange(g, true, s)) != DG_OK) return st;
+  // pool growth for the ops this rank receives happens now, before any rank scatters
+  if ((st = prepare_insert(g, r.roff[r.P], s)) != DG_OK) return st;
+  if (r.fused) RT_CM(r.comm->quiesce());
+  Received rx;
+  bool win = false;
+  if ((st = route_ops(g, src, dst, w, n, !g->directed, true, false, s, &rx, &win)) != DG_OK)
+    return st;
   if ((st = reset_counters(g, s)) != DG_OK) return st;
-  return local_insert(g, as<u32>(r.rsrc), as<u32>(r.rdst), as<u32>(r.rw), r.roff[r.P], false, epoch,
-                      s);
+  return local_insert(g, rx.src, rx.dst, rx.w, r.roff[r.P], false, epoch, s);
 }
 
 dg_status router_delete(dg_graph g, const u32* src, const u32* dst, u64 n, u32 epoch,
                         cudaStream_t s) {
   dg_status st = route_partition(g, src, dst, nullptr, n, !g->directed, false, false, s);
   if (st == DG_ERR_VERTEX_OUT_OF_RANGE) {
-    g->hctl->fail_epoch = epoch;
-    RT_CK(cudaMemcpyAsync(&g->ctl->fail_epoch, &epoch, 4, cudaMemcpyHostToDevice, s));
+    if ((st = mark_rejected(g, epoch, s)) != DG_OK) return st;
     return reset_counters(g, s);
   }
   if (st != DG_OK) return st;
   Router& r = *g->router;
-  if (r.fused) {
-    if ((st = route_fused_scatter(g, src, dst, nullptr, n, !g->directed, false, false, s)) != DG_OK)
-      return st;
-    if ((st = reset_counters(g, s)) != DG_OK) return st;
-    const WinPtrs x = win_ptrs(r.win, r.wcap);
-    return local_delete(g, x.src, x.dst, r.roff[r.P], false, epoch, s);
-  }
-  if ((st = route_exchange(g, false, s)) != DG_OK) return st;
+  Received rx;
+  bool win = false;
+  if ((st = route_ops(g, src, dst, nullptr, n, !g->directed, false, false, s, &rx, &win)) != DG_OK)
+    return st;
   if ((st = reset_counters(g, s)) != DG_OK) return st;
-  return local_delete(g, as<u32>(r.rsrc), as<u32>(r.rdst), r.roff[r.P], false, epoch, s);
+  return local_delete(g, rx.src, rx.dst, r.roff[r.P], false, epoch, s);
 }
 
+// Out-of-range queries (Q7/Q19) behave as at P = 1: they are not routed and answer 0,
+// the in-range queries of the batch are answered, and the batch reports
+// DG_ERR_VERTEX_OUT_OF_RANGE (on every rank).
 dg_status router_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t* found, u32* wout,
                        u32 epoch, cudaStream_t s) {
   Router& r = *g->router;
-  const Nccl& N = nccl();
   dg_status st = route_partition(g, src, dst, nullptr, n, false, false, true, s);
   if (st == DG_ERR_VERTEX_OUT_OF_RANGE) {
-    // answer 0 everywhere and report the batch as rejected (Q7/Q19)
-    if (n) {
-      RT_CK(cudaMemsetAsync(found, 0, n, s));
-      if (wout) RT_CK(cudaMemsetAsync(wout, 0, n * 4, s));
-    }
-    RT_CK(cudaMemcpyAsync(&g->ctl->fail_epoch, &epoch, 4, cudaMemcpyHostToDevice, s));
-    return DG_OK;
+    if ((st = mark_rejected(g, epoch, s)) != DG_OK) return st;
+  } else if (st != DG_OK) {
+    return st;
   }
-  if (st != DG_OK) return st;
   const u64 total = r.roff[r.P];
-  RT_CK(grow(r.rfound, total + 1));
-  RT_CK(grow(r.rwt, total * 4 + 4));
-  if (r.fused) {
-    if ((st = route_fused_scatter(g, src, dst, nullptr, n, false, false, true, s)) != DG_OK)
-      return st;
-    const WinPtrs x = win_ptrs(r.win, r.wcap);
-    if ((st = local_query(g, x.src, x.dst, total, as<uint8_t>(r.rfound), as<u32>(r.rwt), epoch,
-                          s)) != DG_OK)
-      return st;
+  if (!r.fused) {  // (fused: sized with the windows, see window_setup)
+    RT_CK(grow(r.rfound, total + 1));
+    RT_CK(grow(r.rwt, total * 4 + 4));
+  }
+  Received rx;
+  bool win = false;
+  if ((st = route_ops(g, src, dst, nullptr, n, false, false, true, s, &rx, &win)) != DG_OK)
+    return st;
+  if ((st = local_query(g, rx.src, rx.dst, total, as<uint8_t>(r.rfound), as<u32>(r.rwt), epoch,
+                        s)) != DG_OK)
+    return st;
+  const uint8_t* afound = nullptr;
+  const u32* awt = nullptr;
+  if (win) {
     // answers straight into the askers' answer windows, then wait for ours (a11)
+    const WinPtrs x = win_ptrs(r.win, r.wcap);
     k_route_return<<<(unsigned)g->sms * 4, 256, 0, s>>>(as<uint8_t>(r.rfound), as<u32>(r.rwt), r.P,
                                                         as<RouteTable>(r.table), &x.hdr->done_ret);
     r.ans_expected += r.P;
     k_route_wait<<<1, 32, 0, s>>>(&x.hdr->ans_arrive, r.ans_expected, g->ctl);
     note_kernel(2);
-    if (n) {
-      u64 blocks = std::min<u64>((n + 255) / 256, (u64)g->sms * 8);
-      k_route_unpermute<<<(unsigned)blocks, 256, 0, s>>>(as<u64>(r.pos), n, x.found, x.wt, found,
-                                                         wout);
-      note_kernel(1);
-    }
     RT_CK(cudaGetLastError());
-    return DG_OK;
-  }
-  if ((st = route_exchange(g, false, s)) != DG_OK) return st;
-  RT_CK(grow(r.sfound, n + 1));
-  RT_CK(grow(r.swt, n * 4 + 4));
-  if ((st = local_query(g, as<u32>(r.rsrc), as<u32>(r.rdst), total, as<uint8_t>(r.rfound),
-                        as<u32>(r.rwt), epoch, s)) != DG_OK)
-    return st;
-  // answers travel back to the ranks that asked (a11)
-  if (r.rcnt[r.rank]) {
-    RT_CK(cudaMemcpyAsync(as<uint8_t>(r.sfound) + r.soff[r.rank], as<uint8_t>(r.rfound) + r.roff[r.rank],
-                          r.rcnt[r.rank], cudaMemcpyDeviceToDevice, s));
-    RT_CK(cudaMemcpyAsync(as<u32>(r.swt) + r.soff[r.rank], as<u32>(r.rwt) + r.roff[r.rank],
-                          r.rcnt[r.rank] * 4, cudaMemcpyDeviceToDevice, s));
-  }
-  RT_NC(N.GroupStart());
-  for (u32 q = 0; q < r.P; ++q) {
-    if (q == r.rank) continue;
-    if (r.rcnt[q]) {
-      RT_NC(N.Send(as<uint8_t>(r.rfound) + r.roff[q], r.rcnt[q], ncclUint8, q, r.comm, s));
-      RT_NC(N.Send(as<u32>(r.rwt) + r.roff[q], r.rcnt[q], ncclUint32, q, r.comm, s));
+    afound = x.found;
+    awt = x.wt;
+  } else {
+    // answers travel back through the reversed exchange (a11)
+    RT_CK(grow(r.rfound, total + 1));  // (a fused batch that fell back)
+    RT_CK(grow(r.rwt, total * 4 + 4));
+    RT_CK(grow(r.sfound, n + 1));
+    RT_CK(grow(r.swt, n * 4 + 4));
+    if (r.rcnt[r.rank]) {
+      RT_CK(cudaMemcpyAsync(as<uint8_t>(r.sfound) + r.soff[r.rank],
+                            as<uint8_t>(r.rfound) + r.roff[r.rank], r.rcnt[r.rank],
+                            cudaMemcpyDeviceToDevice, s));
+      RT_CK(cudaMemcpyAsync(as<u32>(r.swt) + r.soff[r.rank], as<u32>(r.rwt) + r.roff[r.rank],
+                            r.rcnt[r.rank] * 4, cudaMemcpyDeviceToDevice, s));
     }
-    if (r.scnt[q]) {
-      RT_NC(N.Recv(as<uint8_t>(r.sfound) + r.soff[q], r.scnt[q], ncclUint8, q, r.comm, s));
-      RT_NC(N.Recv(as<u32>(r.swt) + r.soff[q], r.scnt[q], ncclUint32, q, r.comm, s));
+    RT_CM(r.comm->group_start());
+    for (u32 q = 0; q < r.P; ++q) {
+      if (q == r.rank) continue;
+      if (r.rcnt[q]) {
+        RT_CM(r.comm->send(as<uint8_t>(r.rfound) + r.roff[q], r.rcnt[q], q, s));
+        RT_CM(r.comm->send(as<u32>(r.rwt) + r.roff[q], r.rcnt[q] * 4, q, s));
+      }
+      if (r.scnt[q]) {
+        RT_CM(r.comm->recv(as<uint8_t>(r.sfound) + r.soff[q], r.scnt[q], q, s));
+        RT_CM(r.comm->recv(as<u32>(r.swt) + r.soff[q], r.scnt[q] * 4, q, s));
+      }
     }
+    RT_CM(r.comm->group_end(s));
+    afound = as<uint8_t>(r.sfound);
+    awt = as<u32>(r.swt);
   }
-  RT_NC(N.GroupEnd());
   if (n) {
     u64 blocks = std::min<u64>((n + 255) / 256, (u64)g->sms * 8);
-    k_route_unpermute<<<(unsigned)blocks, 256, 0, s>>>(as<u64>(r.pos), n, as<uint8_t>(r.sfound),
-                                                       as<u32>(r.swt), found, wout);
+    k_route_unpermute<<<(unsigned)blocks, 256, 0, s>>>(as<u64>(r.pos), n, afound, awt, found, wout);
     note_kernel(1);
     RT_CK(cudaGetLastError());
   }
@@ -756,11 +748,11 @@ dg_status router_allgather_u32(dg_graph g, const u32* ids, u64 n, int slot, cons
                                u64* all_n, cudaStream_t s) {
   Router& r = *g->router;
   Router::Buf& out = slot ? r.ids2 : r.ids;
-  const Nccl& N = nccl();
   RT_CK(grow(r.scalar, (size_t)(r.P + 1) * 8));
   u64* cnts = as<u64>(r.scalar);
-  RT_CK(cudaMemcpyAsync(cnts + r.P, &n, 8, cudaMemcpyHostToDevice, s));
-  RT_NC(N.AllGather(cnts + r.P, cnts, 1, ncclUint64, r.comm, s));
+  r.h_scalar[3] = n;
+  RT_CK(cudaMemcpyAsync(cnts + r.P, r.h_scalar + 3, 8, cudaMemcpyHostToDevice, s));
+  RT_CM(r.comm->allgather(cnts + r.P, cnts, 8, s));
   RT_CK(cudaMemcpyAsync(r.h_meta, cnts, (size_t)r.P * 8, cudaMemcpyDeviceToHost, s));
   RT_CK(cudaStreamSynchronize(s));
   std::vector<u64> off(r.P + 1, 0);
@@ -768,33 +760,34 @@ dg_status router_allgather_u32(dg_graph g, const u32* ids, u64 n, int slot, cons
   const u64 total = off[r.P];
   RT_CK(grow(out, total * 4 + 4));
   if (n) RT_CK(cudaMemcpyAsync(as<u32>(out) + off[r.rank], ids, n * 4, cudaMemcpyDeviceToDevice, s));
-  RT_NC(N.GroupStart());
+  RT_CM(r.comm->group_start());
   for (u32 q = 0; q < r.P; ++q) {
     if (q == r.rank) continue;
-    if (n) RT_NC(N.Send(ids, n, ncclUint32, q, r.comm, s));
-    if (r.h_meta[q]) RT_NC(N.Recv(as<u32>(out) + off[q], r.h_meta[q], ncclUint32, q, r.comm, s));
+    if (n) RT_CM(r.comm->send(ids, n * 4, q, s));
+    if (r.h_meta[q]) RT_CM(r.comm->recv(as<u32>(out) + off[q], r.h_meta[q] * 4, q, s));
   }
-  RT_NC(N.GroupEnd());
+  RT_CM(r.comm->group_end(s));
   *all = as<u32>(out);
   *all_n = total;
   return DG_OK;
 }
 
-dg_status allreduce_u64(dg_graph g, u64* v, ncclRedOp_t op, cudaStream_t s) {
+namespace {
+dg_status allreduce_u64(dg_graph g, u64* v, bool max, cudaStream_t s) {
   Router& r = *g->router;
-  const Nccl& N = nccl();
   RT_CK(grow(r.scalar, (size_t)(r.P + 1) * 8));
   u64* d = as<u64>(r.scalar);
   r.h_scalar[0] = *v;
   RT_CK(cudaMemcpyAsync(d, r.h_scalar, 8, cudaMemcpyHostToDevice, s));
-  RT_NC(N.AllReduce(d, d, 1, ncclUint64, op, r.comm, s));
+  RT_CM(r.comm->allreduce_u64(d, max, s));
   RT_CK(cudaMemcpyAsync(r.h_scalar, d, 8, cudaMemcpyDeviceToHost, s));
   RT_CK(cudaStreamSynchronize(s));
   *v = r.h_scalar[0];
   return DG_OK;
 }
+}  // namespace
 
-dg_status router_sum_u64(dg_graph g, u64* v, cudaStream_t s) { return allreduce_u64(g, v, ncclSum, s); }
-dg_status router_max_u64(dg_graph g, u64* v, cudaStream_t s) { return allreduce_u64(g, v, ncclMax, s); }
+dg_status router_sum_u64(dg_graph g, u64* v, cudaStream_t s) { return allreduce_u64(g, v, false, s); }
+dg_status router_max_u64(dg_graph g, u64* v, cudaStream_t s) { return allreduce_u64(g, v, true, s); }
 
 }  // namespace dg

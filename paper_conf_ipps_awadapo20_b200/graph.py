@@ -73,7 +73,8 @@ class Graph:
                  device: int | None = None, rank: int = 0, nranks: int = 1,
                  nccl_unique_id: bytes | None = None, reuse_tombstones: bool = True,
                  force_router: bool = False, set_variant: bool = False,
-                 adaptive: bool = False, stream=None):
+                 adaptive: bool = False, group: "RankGroup | None" = None,
+                 copy_exchange: bool = False, stream=None):
         if bucket_bytes == 0:
             adaptive, bucket_bytes = True, 128
         cfg = dg_config()
@@ -90,7 +91,11 @@ class Graph:
         cfg.flags = (0 if reuse_tombstones else _lib.DG_FLAG_NO_TOMBSTONE_REUSE) | \
             (_lib.DG_FLAG_FORCE_ROUTER if force_router else 0) | \
             (_lib.DG_FLAG_SET if set_variant else 0) | \
-            (_lib.DG_FLAG_ADAPTIVE if adaptive else 0)
+            (_lib.DG_FLAG_ADAPTIVE if adaptive else 0) | \
+            (_lib.DG_FLAG_COPY_EXCHANGE if copy_exchange else 0)
+        self._group = group  # keeps the group alive while the handle exists
+        if group is not None:
+            cfg.group = group.handle.value
         self._uid = None
         if nccl_unique_id is not None:
             self._uid = ctypes.create_string_buffer(bytes(nccl_unique_id), 128)
@@ -260,6 +265,19 @@ class Graph:
             check(st, "dg_batch_status")
         return st
 
+    VIOLATIONS = ("empty_not_suffix", "misplaced_keys", "duplicate_keys", "self_loops",
+                  "keys_out_of_range", "owner_mismatch", "degree_mismatch", "broken_chains")
+
+    def check_invariants(self, stream=None) -> dict:
+        """Structural invariants of the tables (dg_check_invariants): violation counts
+        plus what was walked.  ``violations`` sums the violation counters."""
+        r = _lib.dg_invariants()
+        check(lib.dg_check_invariants(self._h, ctypes.byref(r), _stream(stream)),
+              "dg_check_invariants")
+        out = {name: getattr(r, name) for name, _ in _lib.dg_invariants._fields_}
+        out["violations"] = sum(out[k] for k in self.VIOLATIONS)
+        return out
+
     # ------------------------------------------------------- instrumentation --
     PROFILE_KINDS = ("insert", "delete", "query", "vertex_purge", "tc")
 
@@ -289,10 +307,38 @@ class Graph:
         return c.value
 
 
+class RankGroup:
+    """In-process rank group (``dg_group_create``): ``nranks`` host threads of this
+    process act as the ranks of a sharded graph, each creating its own ``Graph(...,
+    rank=r, nranks=nranks, group=grp)`` and calling every collective with its own slice
+    on its own (non-blocking) stream.  ctypes releases the GIL during library calls, so
+    Python threads run the ranks concurrently."""
+
+    def __init__(self, nranks: int):
+        self._h = ctypes.c_void_p()
+        check(lib.dg_group_create(int(nranks), ctypes.byref(self._h)), "dg_group_create")
+        self.nranks = int(nranks)
+
+    @property
+    def handle(self):
+        return self._h
+
+    def close(self):
+        if getattr(self, "_h", None) and self._h.value:
+            lib.dg_group_destroy(self._h)
+            self._h = ctypes.c_void_p()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+
 def get_unique_id() -> bytes:
     buf = ctypes.create_string_buffer(128)
     check(lib.dg_get_unique_id(buf), "dg_get_unique_id")
     return buf.raw
 
 
-__all__ = ["Graph", "DGError", "get_unique_id"]
+__all__ = ["Graph", "RankGroup", "DGError", "get_unique_id"]

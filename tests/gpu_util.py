@@ -64,7 +64,16 @@ def check_against_oracle(g, o: Oracle, where=""):
     assert np.array_equal(deg, o.degrees()), f"{where}: degrees differ"
     errs = check_invariants(ro, d, deg)
     assert not errs, f"{where}: {errs}"
+    assert_table_invariants(g, where)
     return cand
+
+
+def assert_table_invariants(g, where=""):
+    """dg_check_invariants: EMPTY-suffix chains, keys in their hash chain, no duplicate,
+    owner words, degree == live keys, chains end."""
+    inv = g.check_invariants()
+    assert inv["violations"] == 0, f"{where}: table invariants violated: {inv}"
+    return inv
 
 
 def check_queries(g, o: Oracle, qs, qd, cand=None, where=""):

@@ -44,13 +44,15 @@ def test_struct_layout_matches_c(tmp_path):
     from paper_conf_ipps_awadapo20_b200._lib import dg_config, dg_stats
     src = tmp_path / "sz.c"
     src.write_text('#include "dg.h"\n#include <stdio.h>\n#include <stddef.h>\n'
-                   'int main(){printf("%zu %zu %zu %zu\\n", sizeof(dg_config), sizeof(dg_stats),'
-                   ' offsetof(dg_config, nccl_unique_id), offsetof(dg_stats, load_factor));}\n')
+                   'int main(){printf("%zu %zu %zu %zu %zu\\n", sizeof(dg_config), sizeof(dg_stats),'
+                   ' offsetof(dg_config, nccl_unique_id), offsetof(dg_stats, load_factor),'
+                   ' offsetof(dg_config, group));}\n')
     exe = tmp_path / "sz"
     subprocess.check_call(["gcc", "-I", os.path.join(ROOT, "include"), str(src), "-o", str(exe)])
     c = [int(x) for x in subprocess.check_output([str(exe)]).split()]
     assert c == [ctypes.sizeof(dg_config), ctypes.sizeof(dg_stats),
-                 dg_config.nccl_unique_id.offset, dg_stats.load_factor.offset]
+                 dg_config.nccl_unique_id.offset, dg_stats.load_factor.offset,
+                 dg_config.group.offset]
 
 
 def test_config_defaults_and_status_strings():
@@ -103,6 +105,21 @@ def test_flag_values_match_header():
     hdr = open(os.path.join(ROOT, "include", "dg.h")).read()
     flags = dict(re.findall(r"#define (DG_FLAG_\w+) (\d+)u", hdr))
     assert set(flags) == {"DG_FLAG_NO_TOMBSTONE_REUSE", "DG_FLAG_FORCE_ROUTER", "DG_FLAG_SET",
-                          "DG_FLAG_ADAPTIVE"}
+                          "DG_FLAG_ADAPTIVE", "DG_FLAG_COPY_EXCHANGE"}
     for k, v in flags.items():
         assert getattr(_lib, k) == int(v), k
+
+
+def test_rank_group_is_host_only():
+    """dg_group_create / dg_group_destroy need no GPU; a sharded create needs a NCCL id
+    or a group, and a group must have the handle's nranks"""
+    from paper_conf_ipps_awadapo20_b200 import RankGroup, _lib
+    lib = _lib.lib
+    h = ctypes.c_void_p()
+    assert lib.dg_group_create(0, ctypes.byref(h)) == _lib.DG_ERR_INVALID_ARGUMENT
+    assert lib.dg_group_create(65, ctypes.byref(h)) == _lib.DG_ERR_INVALID_ARGUMENT
+    assert lib.dg_group_destroy(None) == _lib.DG_ERR_INVALID_ARGUMENT
+    g = RankGroup(4)
+    assert g.handle.value
+    g.close()
+    assert not g.handle.value

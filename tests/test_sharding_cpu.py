@@ -177,3 +177,150 @@ def test_sharded_query_return_matches_unsharded():
         assert not f[qs == qd].any()  # self-loops are never stored (Alg1:L3)
         hits += int(f.sum())
     assert hits > 0
+
+
+class _ShardedOracleRank:
+    """A CPU stand-in for one rank's ``Graph`` in ``tests/multirank.py``: the rank's
+    shard is an oracle holding only the rows it owns (owner(u) = u mod P); every call
+    is collective over gloo — the slices are all-gathered, each owner applies the ops
+    of its rows, counts are summed and query answers travel back to the askers.  It
+    pins the scenario and its checker (what the GPU router tests assert) on CPU."""
+
+    def __init__(self, nv, rank, P, directed=True):
+        from oracle import Oracle
+        self.rank, self.P, self.directed = rank, P, directed
+        self.o = Oracle(nv, directed=True)
+        self.nv = nv
+        self._status = 0
+
+    def _union(self, *arrs):
+        mine = [np.asarray(a, np.uint32) for a in arrs]
+        allp = [None] * self.P
+        dist.all_gather_object(allp, mine)
+        return [np.concatenate([p[i] for p in allp]) for i in range(len(arrs))], \
+            [p[0].size for p in allp]
+
+    def _sum(self, x):
+        t = torch.tensor([x], dtype=torch.int64)
+        dist.all_reduce(t)
+        return int(t.item())
+
+    def _oob(self, *arrs):
+        return any(bool((a >= self.nv).any()) for a in arrs)
+
+    def _mirror(self, s, d, w=None):
+        if self.directed:
+            return s, d, w
+        return (np.concatenate([s, d]), np.concatenate([d, s]),
+                None if w is None else np.concatenate([w, w]))
+
+    def insert_edges(self, s, d, w, count=True):
+        from paper_conf_ipps_awadapo20_b200 import DGError
+        (s, d, w), _ = self._union(s, d, w)
+        if self._oob(s, d):
+            raise DGError(2, "insert")
+        s, d, w = self._mirror(s, d, w)
+        m = (s % self.P) == self.rank
+        return self._sum(self.o.insert_edges(s[m], d[m], w[m])[1])
+
+    def delete_edges(self, s, d, count=True):
+        from paper_conf_ipps_awadapo20_b200 import DGError
+        (s, d), _ = self._union(s, d)
+        if self._oob(s, d):
+            raise DGError(2, "delete")
+        s, d, _ = self._mirror(s, d)
+        m = (s % self.P) == self.rank
+        return self._sum(self.o.delete_edges(s[m], d[m])[1])
+
+    def query_edges(self, s, d):
+        (us, ud), sizes = self._union(s, d)
+        bad = (us >= self.nv) | (ud >= self.nv)
+        self._status = self._sum(int(bad.any())) and 2
+        m = ((us % self.P) == self.rank) & ~bad
+        f = np.zeros(us.size, np.int64)
+        w = np.zeros(us.size, np.int64)
+        _, f[m], w[m] = self.o.query_edges(us[m], ud[m])
+        ft, wt = torch.from_numpy(f), torch.from_numpy(w)
+        dist.all_reduce(ft)
+        dist.all_reduce(wt)
+        lo = sum(sizes[:self.rank])
+        sl = slice(lo, lo + sizes[self.rank])
+
+        class _T:  # .cpu().numpy() like a tensor
+            def __init__(self, a):
+                self.a = a
+
+            def cpu(self):
+                return self
+
+            def numpy(self):
+                return self.a
+        return _T(ft.numpy()[sl].astype(np.uint8)), _T(wt.numpy()[sl].astype(np.uint32))
+
+    def batch_status(self):
+        st, self._status = self._status, 0
+        return st
+
+    def delete_vertices(self, ids):
+        (ids,), _ = self._union(ids)
+        self._status = 2 if self._oob(ids) else self.o.delete_vertices(ids)
+
+    def insert_vertices(self, ids, hints=None):
+        (ids,), _ = self._union(ids)
+        self.o.insert_vertices(ids)
+        self.nv = self.o.num_vertices
+
+    def export(self, device=False):
+        ro, d, w = self.o.export()
+        rows = np.arange(self.rank, self.nv, self.P)
+        deg = np.diff(ro)[rows].astype(np.int64)
+        sel = (np.concatenate([np.arange(ro[u], ro[u + 1]) for u in rows]).astype(np.int64)
+               if rows.size else np.zeros(0, np.int64))
+        return np.concatenate([[0], np.cumsum(deg)]).astype(np.uint64), d[sel], w[sel]
+
+    def degrees(self, device=False):
+        return np.diff(self.export()[0]).astype(np.uint32)
+
+    def stats(self):
+        return {"exchange": 0}
+
+    @property
+    def num_vertices(self):
+        return self.nv
+
+
+def _scenario_worker(rank, P, port, directed, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=P)
+    try:
+        from tests import multirank
+        g = _ShardedOracleRank(multirank.NV0, rank, P, directed)
+        recs = multirank.run_rank(g, rank, P, lambda a: np.ascontiguousarray(a, np.uint32))
+        out = [None] * P if rank == 0 else None
+        dist.gather_object(recs, out, dst=0)
+        if rank == 0:
+            multirank.check(out, P, directed=directed)
+        q.put((rank, "ok"))
+    except BaseException as e:  # noqa: BLE001
+        q.put((rank, repr(e)))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("P,directed", [(2, True), (3, False)])
+def test_multirank_scenario_on_sharded_oracles(P, directed):
+    """The stream and checker of the GPU router tests (tests/multirank.py), run by P
+    gloo ranks whose shards are oracles: the union of the shards equals the unsharded
+    oracle, rejected batches are rejected on every rank, out-of-range queries answer 0."""
+    port = _free_port()
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    procs = [ctx.Process(target=_scenario_worker, args=(r, P, port, directed, q))
+             for r in range(P)]
+    for p in procs:
+        p.start()
+    res = [q.get(timeout=300) for _ in range(P)]
+    for p in procs:
+        p.join(timeout=60)
+    assert all(r[1] == "ok" for r in res), res
