@@ -46,7 +46,7 @@ constexpr uint64_t kMaxVertices = 0xFFFFFFFEull;
  * write of a key inside one batch from a first one); the graph is A_u : v -> w. */
 struct Entry {
   uint32_t w;
-  uint64_t batch;
+  uint32_t batch;  // (mod 2^32: a stamp only has to differ from the current batch's)
 };
 
 inline uint64_t key_of(uint32_t u, uint32_t v) { return ((uint64_t)u << 32) | v; }
@@ -55,7 +55,7 @@ struct Oracle {
   uint64_t cap = 0;
   bool directed = true;
   unsigned T = 1;        // host threads; thread t owns the vertices u with u % T == t
-  uint64_t batch = 0;    // insert batches applied so far
+  uint32_t batch = 0;    // insert batches applied so far (mod 2^32)
   std::vector<std::unordered_map<uint32_t, Entry>> A;  // A_u : v -> w
   /* Q1: keys (u,v) written >= 2 times by their most recent insert batch, with
    * the weights that batch carried for them (in batch order); any one of them is a
@@ -152,7 +152,7 @@ int orc_insert_edges(void* h, const uint32_t* src, const uint32_t* dst, const ui
   if (!in_range(g, src, n) || !in_range(g, dst, n)) return ORC_ERR_VERTEX_OUT_OF_RANGE;
   std::vector<uint32_t> S, D, W;
   expand(g, src, dst, w, n, S, D, W);
-  const uint64_t b = ++g.batch;
+  const uint32_t b = ++g.batch;
   const unsigned P = threads_for(g, S.size());
   std::vector<uint64_t> added(P, 0);
   parallel(P, [&](unsigned t) {

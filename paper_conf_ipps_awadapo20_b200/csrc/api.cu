@@ -223,11 +223,18 @@ namespace dg {
 
 void prof_mark(dg_graph g, int k, cudaStream_t s) {
   if (!g->prof) return;
-  cudaEvent_t e;
-  if (cudaEventCreate(&e) != cudaSuccess) {
-    cudaGetLastError();
-    return;
+  if (g->prof_pool.empty()) {  // events are created in batches, outside the common path
+    for (int i = 0; i < 64; ++i) {
+      cudaEvent_t e;
+      if (cudaEventCreate(&e) != cudaSuccess) {
+        cudaGetLastError();
+        return;
+      }
+      g->prof_pool.push_back(e);
+    }
   }
+  cudaEvent_t e = g->prof_pool.back();
+  g->prof_pool.pop_back();
   cudaEventRecord(e, s);
   g->prof_ev[k].push_back(e);
 }
@@ -378,6 +385,11 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   a.reuse_tombstones = g->reuse_tombstones ? 1u : 0u;
   a.epoch = epoch;
   a.nv = g->nv;
+  // src-sorted batches (k_validate's verdict for this epoch) take the same-source
+  // grouped path (a3)
+  static const bool no_sorted = std::getenv("DG_NO_SORTED_PATH") != nullptr;
+  // (large batches only: a small batch would pay a second launch for little)
+  a.sorted_path = (!no_sorted && !mirror && epoch == g->validated_epoch && n >= (1u << 18)) ? 1u : 0u;
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
@@ -389,12 +401,8 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
                  (unsigned long long)n_ops, g->hctl->pop_count[0], g->hctl->stack_size[0], b0,
                  g->hctl->bump[0], g->hctl->ret_count);
   }
-  DG_CK(dg::launch_fixup_alloc(t, s));
-  if (g->hot_steps && !g->in_rehash) {  // chain-length metric, read before the next batch
-    DG_CK(cudaMemcpyAsync(g->h_hot, &g->ctl->hot_count, 8, cudaMemcpyDeviceToHost, s));
-    DG_CK(cudaEventRecord(g->hot_event, s));
-    g->hot_pending = true;
-  }
+  // (the fixup kernel also publishes the chain-length metric for the next batch)
+  DG_CK(dg::launch_fixup_alloc(t, (g->hot_steps && !g->in_rehash) ? g->d_hot : nullptr, s));
   if (!retry_mode) {
     note_launch(g, need, s);
     return DG_OK;
@@ -422,10 +430,11 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
     t = g->tables();
     a.idx = whole ? nullptr : g->retry[cur];
     a.n_ops = whole ? n_ops : failed;
+    a.sorted_path = 0;  // re-runs go through k_edges
     a.retry_out = g->retry[cur ^ 1];
     a.retry_cap = next_cap;
     DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
-    DG_CK(dg::launch_fixup_alloc(t, s));
+    DG_CK(dg::launch_fixup_alloc(t, nullptr, s));
     cur ^= 1;
   }
   return DG_OK;
@@ -471,7 +480,8 @@ dg_status local_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_t
 // for twice its degree, and insert the pairs again.  Runs before an insert batch
 // (phase-concurrent: no other batch in flight on the handle).
 dg_status rehash_hot(dg_graph g, cudaStream_t s) {
-  return rehash_rows(g, std::min<u32>(*g->h_hot, g->hot_cap), false, s);
+  DG_TRY(read_ctl(g, s));  // exact count (the published one may lag a batch)
+  return rehash_rows(g, std::min<u32>(g->hctl->hot_count, g->hot_cap), false, s);
 }
 
 // Re-build the n rows of hot_list (flush = false: long chains, sized to double;
@@ -544,6 +554,7 @@ dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
   DG_CK(cudaMemcpyAsync(g->ctl->bump, newbump, 4 * dg::kClasses, cudaMemcpyHostToDevice, s));
   DG_CK(cudaMemsetAsync(g->hot_flags, 0, g->hot_words * 4, s));
   DG_CK(cudaMemsetAsync(&g->ctl->hot_count, 0, 8, s));  // hot_count, hot_pairs
+  g->h_hot[0] = g->h_hot[1] = 0;
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, 4, s));
   for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::max<u64>(g->bump_ub[c], newbump[c]);
@@ -593,7 +604,7 @@ dg_status dg_get_unique_id(void* out128) {
 
 static void prof_clear(dg_graph g) {
   for (auto& v : g->prof_ev) {
-    for (cudaEvent_t e : v) cudaEventDestroy(e);
+    for (cudaEvent_t e : v) g->prof_pool.push_back(e);
     v.clear();
   }
 }
@@ -604,6 +615,8 @@ static void destroy_graph(dg_graph g) {
   cudaDeviceSynchronize();
   cudaGetLastError();
   prof_clear(g);
+  for (cudaEvent_t e : g->prof_pool) cudaEventDestroy(e);
+  g->prof_pool.clear();
   if (g->router) dg::router_destroy(g->router);
   g->dir.release();
   g->degv.release();
@@ -630,7 +643,6 @@ static void destroy_graph(dg_graph g) {
   if (g->hot_flags) cudaFree(g->hot_flags);
   if (g->hot_list) cudaFree(g->hot_list);
   if (g->h_hot) cudaFreeHost(g->h_hot);
-  if (g->hot_event) cudaEventDestroy(g->hot_event);
   for (auto& cs : g->cstream)
     if (cs) cudaStreamDestroy(cs);
   for (cudaEvent_t e : g->slot_ev)
@@ -772,10 +784,10 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   if (cudaMalloc(&g->small_dev, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
   if (const char* hs = std::getenv("DG_HOT_STEPS")) g->hot_steps = (u32)std::atoi(hs);
   if (cudaMalloc(&g->hot_list, (size_t)g->hot_cap * 4) != cudaSuccess) return fail(DG_ERR_CUDA);
-  if (cudaMallocHost(&g->h_hot, 64) != cudaSuccess) return fail(DG_ERR_CUDA);
-  *g->h_hot = 0;
-  if (cudaEventCreateWithFlags(&g->hot_event, cudaEventDisableTiming) != cudaSuccess)
+  if (cudaHostAlloc(reinterpret_cast<void**>(&g->h_hot), 64, cudaHostAllocMapped) != cudaSuccess ||
+      cudaHostGetDevicePointer(reinterpret_cast<void**>(&g->d_hot), g->h_hot, 0) != cudaSuccess)
     return fail(DG_ERR_CUDA);
+  g->h_hot[0] = g->h_hot[1] = 0;
   if (cudaMalloc(&g->stats_dev, sizeof(dg::StatsOut)) != cudaSuccess) return fail(DG_ERR_CUDA);
 
   if (g->nranks > 1 || (cfg->group && (cfg->flags & DG_FLAG_FORCE_ROUTER))) {
@@ -844,18 +856,17 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   if (n_added) *n_added = 0;
   // re-size tables whose chains grew too long in earlier batches
-  if (g->hot_steps && g->hot_pending) {
-    const cudaError_t q = cudaEventQuery(g->hot_event);
-    if (q == cudaSuccess) {
-      g->hot_pending = false;
-      // worth a re-sizing pass (it synchronises): flagged pairs reach 1/1024 of the
-      // table slots (at least 2,048), or the flag list is filling up
+  if (g->hot_steps) {
+    // worth a re-sizing pass (it synchronises): flagged pairs reach 1/1024 of the
+    // table slots (at least 2,048), or the flag list is filling up.  The counters are
+    // the ones the last finished insert published (mapped memory, no copy, no event).
+    const u32 hot_rows = reinterpret_cast<volatile u32*>(g->h_hot)[0];
+    const u32 hot_pairs = reinterpret_cast<volatile u32*>(g->h_hot)[1];
+    if (hot_rows) {
       u64 slots = 0;
       for (int c = 0; c < g->ncls; ++c) slots += g->bump_ub[c] * (g->adaptive ? (4u << c) - 1 : g->BC);
       const u64 thr = std::max<u64>(2048, slots / 1024);
-      if (g->h_hot[1] >= thr || g->h_hot[0] >= g->hot_cap / 2) DG_TRY(dg::rehash_hot(g, s));
-    } else if (q != cudaErrorNotReady) {
-      DG_CK(q);
+      if (hot_pairs >= thr || hot_rows >= g->hot_cap / 2) DG_TRY(dg::rehash_hot(g, s));
     }
   }
   const u32 epoch = ++g->epoch;
@@ -869,6 +880,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     DG_TRY(upload_async(g, 9, dst, n * 4, s, &dd));
     DG_TRY(upload_async(g, 10, weight, weight ? n * 4 : 0, s, &dw));
     DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    g->validated_epoch = epoch;
     DG_TRY(note_validation(g, s));
     DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
                             epoch, s));
@@ -882,6 +894,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
   } else {
     DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+    g->validated_epoch = epoch;
     DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
                             epoch, s));
   }
@@ -1228,8 +1241,7 @@ dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* stream) 
   DG_TRY(check_handle(g));
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   if (rows_rebuilt) *rows_rebuilt = 0;
-  if (g->hot_pending) DG_CK(cudaEventSynchronize(g->hot_event));
-  g->hot_pending = false;  // rows flagged by earlier inserts are rebuilt below too
+  // (rows flagged by earlier inserts are rebuilt below too)
   u64 total = 0;
   for (int pass = 0; pass < 100000; ++pass) {
     dg::Tables t = g->tables();

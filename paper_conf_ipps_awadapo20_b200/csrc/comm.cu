@@ -313,6 +313,18 @@ class GroupComm final : public Comm {
     for (uint32_t q = 0; q < G_->P; ++q) peers[q] = nullptr;
   }
   dg_status quiesce() override { return G_->barrier() ? DG_OK : DG_ERR_NCCL; }
+  bool host_ordered() const override { return true; }
+  dg_status wait_peers(cudaEvent_t ev, cudaStream_t s) override {
+    CM_CK(cudaEventRecord(ev, s));
+    G_->ptr[rank_] = ev;
+    if (!G_->barrier()) return DG_ERR_NCCL;
+    for (uint32_t q = 0; q < G_->P; ++q)
+      if (q != rank_)
+        CM_CK(cudaStreamWaitEvent(s, static_cast<cudaEvent_t>(const_cast<void*>(G_->ptr[q])), 0));
+    // (a peer re-records its event only after everyone has enqueued the wait)
+    if (!G_->barrier()) return DG_ERR_NCCL;
+    return DG_OK;
+  }
 
  private:
   dg_group G_;

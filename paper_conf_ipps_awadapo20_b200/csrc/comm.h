@@ -45,6 +45,14 @@ struct Comm {
   // blocked in a device-wide synchronisation waits for a peer's spin-wait kernel,
   // which waits for this rank's not-yet-launched scatter.
   virtual dg_status quiesce() { return DG_OK; }
+  // How the fused exchange waits for the peers' stores into this rank's window.
+  // false: a one-thread device kernel spins on the window's arrival counter (separate
+  // processes / contexts).  true: in-process groups order the streams with CUDA events
+  // instead (streams of one context can share a hardware queue, where a spinning
+  // kernel would block the very peer kernel it waits for): wait_peers records `ev`
+  // on s after this rank's stores, and makes s wait for every peer's event.
+  virtual bool host_ordered() const { return false; }
+  virtual dg_status wait_peers(cudaEvent_t ev, cudaStream_t s) { return DG_ERR_UNSUPPORTED; }
 };
 
 // NCCL transport (dlopen'ed NCCL; unique_id = 128-byte ncclUniqueId)

@@ -58,6 +58,8 @@ struct DevCtl {
   u32 hot_count;     // rows flagged for re-sizing (long chains), see k_edges / rehash
   u32 hot_pairs;     // sum of their degrees when flagged (saturating): work to re-size
   u32 route_timeout; // a fused-exchange wait gave up on a peer (router.cu)
+  u32 unsorted_epoch; // highest validated batch epoch whose sources were not sorted
+  u32 fixup_done;     // blocks of k_fixup finished (last-block pattern; reset by the last)
 };
 
 struct Tables {

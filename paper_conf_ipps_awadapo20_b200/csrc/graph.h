@@ -60,6 +60,7 @@ struct dg_graph_s {
 
   uint32_t epoch = 0;
   uint32_t checked_epoch = 0;
+  uint32_t validated_epoch = 0;  // batch whose sources k_validate checked (sortedness, a3)
   bool bad = false;
 
   struct Buf {
@@ -80,9 +81,10 @@ struct dg_graph_s {
   uint32_t* hot_list = nullptr;
   uint32_t hot_cap = 65536;
   uint32_t hot_steps = 4;      // 0 = off
-  uint32_t* h_hot = nullptr;   // pinned copy of ctl->hot_count
-  cudaEvent_t hot_event = nullptr;
-  bool hot_pending = false;
+  // mapped pinned {hot_count, hot_pairs}, written by the insert's fixup kernel (read
+  // by the host without a copy; may lag one batch behind, which only delays re-sizing)
+  uint32_t* h_hot = nullptr;
+  uint32_t* d_hot = nullptr;   // its device alias
   bool in_rehash = false;
   cudaStream_t cstream[2] = {nullptr, nullptr};  // host-buffer pipeline: upload, download
   std::vector<cudaEvent_t> pipe_ev;
@@ -93,6 +95,7 @@ struct dg_graph_s {
   bool prof = false;
   uint64_t prof_launch0 = 0;
   std::vector<cudaEvent_t> prof_ev[5];  // start/stop pairs per kernel kind
+  std::vector<cudaEvent_t> prof_pool;   // recycled events (none created on the hot path)
 
   dg::Tables tables() const {
     dg::Tables t;

@@ -32,6 +32,8 @@ struct EdgeBatch {
   u32* wout;          // query, nullable
   u32 reuse_tombstones;  // insert: install new keys in the first tombstone
   u32 chunk;             // insert: buckets per per-warp allocation chunk (set by the launcher)
+  u32 sorted_path;       // insert: k_validate checked this epoch's sources for sortedness;
+                         // a src-sorted batch runs k_insert_sorted (a3), others k_edges
 };
 
 // `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1
@@ -43,7 +45,9 @@ cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 e
 cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
 cudaError_t launch_delete(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
 cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
-cudaError_t launch_fixup_alloc(const Tables& t, cudaStream_t s);
+// after an insert launch: free stack / cursors; hot_out (mapped host, nullable)
+// receives {hot_count, hot_pairs}
+cudaError_t launch_fixup_alloc(const Tables& t, u32* hot_out, cudaStream_t s);
 u64 max_groups(int G, int sms);
 
 // graph structure (kernels_graph.cu)

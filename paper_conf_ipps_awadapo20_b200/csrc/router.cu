@@ -25,7 +25,8 @@
 // (peer stores) instead of a local send buffer.  The last block of the kernel fences
 // (system scope) and bumps an arrival counter in every peer's window header; a
 // one-thread kernel on the owner waits for P arrivals before the probe kernel reads
-// the window.  Query answers return the same way: the owner's k_route_return stores
+// the window (in-process rank groups order the ranks' streams with CUDA events
+// instead, comm.h host_ordered()).  Query answers return the same way: the owner's k_route_return stores
 // (found, weight) into each asker's answer window and signals it.  The next batch's
 // counts all-gather orders window reuse (a rank reaches it only after its kernels of
 // the previous batch completed).  A batch larger than the windows triggers a
@@ -283,6 +284,7 @@ struct Router {
   std::vector<char*> retired;      // outgrown windows (peers may still map them)
   unsigned long long arrive_expected = 0, ans_expected = 0;
   RouteTable* h_table = nullptr;   // pinned
+  cudaEvent_t ev_done = nullptr;   // in-process groups: this rank's stores are issued
 };
 
 namespace {
@@ -522,10 +524,16 @@ dg_status route_fused_scatter(dg_graph g, const u32* src, const u32* dst, const 
   k_route_scatter_fused<<<kRouteBlocks, kRouteThreads, 0, s>>>(
       src, dst, w, n, n_ops, g->nv, P, as<u64>(r.offs), as<RouteTable>(r.table), with_w,
       keep_pos ? as<u64>(r.pos) : nullptr, &mine.hdr->done);
-  r.arrive_expected += P;
-  k_route_wait<<<1, 32, 0, s>>>(&mine.hdr->arrive, r.arrive_expected, g->ctl);
-  note_kernel(2);
+  note_kernel(1);
   RT_CK(cudaGetLastError());
+  r.arrive_expected += P;
+  if (r.comm->host_ordered()) {
+    RT_CM(r.comm->wait_peers(r.ev_done, s));
+  } else {
+    k_route_wait<<<1, 32, 0, s>>>(&mine.hdr->arrive, r.arrive_expected, g->ctl);
+    note_kernel(1);
+    RT_CK(cudaGetLastError());
+  }
   return DG_OK;
 }
 
@@ -591,7 +599,8 @@ dg_status router_create(dg_graph g, const void* unique_id, Router** out) {
   if (cudaMallocHost(&r->h_meta, (size_t)(r->P + 1) * (r->P + 1) * 8) != cudaSuccess ||
       cudaMallocHost(&r->h_scalar, 64) != cudaSuccess ||
       cudaMallocHost(&r->h_table, sizeof(RouteTable)) != cudaSuccess ||
-      grow(r->table, sizeof(RouteTable)) != cudaSuccess) {
+      grow(r->table, sizeof(RouteTable)) != cudaSuccess ||
+      cudaEventCreateWithFlags(&r->ev_done, cudaEventDisableTiming) != cudaSuccess) {
     router_destroy(r);
     return DG_ERR_CUDA;
   }
@@ -620,6 +629,7 @@ void router_destroy(Router* r) {
   if (r->win) cudaFree(r->win);
   for (char* p : r->retired) cudaFree(p);
   if (r->h_table) cudaFreeHost(r->h_table);
+  if (r->ev_done) cudaEventDestroy(r->ev_done);
   delete r->comm;
   Router::Buf* all[] = {&r->ssrc, &r->sdst, &r->sw, &r->rsrc, &r->rdst, &r->rw, &r->pos,
                         &r->blockcnt, &r->offs, &r->meta_all, &r->flag, &r->rfound, &r->rwt,
@@ -700,10 +710,16 @@ dg_status router_query(dg_graph g, const u32* src, const u32* dst, u64 n, uint8_
     const WinPtrs x = win_ptrs(r.win, r.wcap);
     k_route_return<<<(unsigned)g->sms * 4, 256, 0, s>>>(as<uint8_t>(r.rfound), as<u32>(r.rwt), r.P,
                                                         as<RouteTable>(r.table), &x.hdr->done_ret);
-    r.ans_expected += r.P;
-    k_route_wait<<<1, 32, 0, s>>>(&x.hdr->ans_arrive, r.ans_expected, g->ctl);
-    note_kernel(2);
+    note_kernel(1);
     RT_CK(cudaGetLastError());
+    r.ans_expected += r.P;
+    if (r.comm->host_ordered()) {
+      RT_CM(r.comm->wait_peers(r.ev_done, s));
+    } else {
+      k_route_wait<<<1, 32, 0, s>>>(&x.hdr->ans_arrive, r.ans_expected, g->ctl);
+      note_kernel(1);
+      RT_CK(cudaGetLastError());
+    }
     afound = x.found;
     awt = x.wt;
   } else {

@@ -34,8 +34,9 @@ def check(g, o, where):
 def run(nv=600, directed=True, **kw):
     g = Graph(nv, directed=directed, device=0, **kw)
     o = Oracle(nv, directed=directed)
+    keys_only = kw.get("set_variant", False)  # the set variant stores no weights
     for b in range(3):
-        s, d, w = wl.uniform_edges(9, b, 1500, nv)
+        s, d, w = wl.uniform_edges(9, b, 1500, nv, weights=not keys_only)
         s[:300] = 7  # a hub: chain growth and re-sizing
         assert g.insert_edges(s, d, w, count=True) == o.insert_edges(s, d, w)[1]
     check(g, o, f"insert {kw}")
@@ -53,7 +54,7 @@ def run(nv=600, directed=True, **kw):
     g.flush_tombstones()
     g.insert_vertices(np.arange(nv, nv + 40, dtype=np.uint32))
     o.insert_vertices(np.arange(nv, nv + 40, dtype=np.uint32))
-    s, d, w = wl.uniform_edges(9, 12, 800, nv + 40)
+    s, d, w = wl.uniform_edges(9, 12, 800, nv + 40, weights=not keys_only)
     assert g.insert_edges(s, d, w, count=True) == o.insert_edges(s, d, w)[1]
     check(g, o, f"growth {kw}")
     g.stats()

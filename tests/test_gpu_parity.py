@@ -238,33 +238,79 @@ def test_rmat_hubs_without_hints(bb):
 
 @pytest.mark.parametrize("hints", [True, False])
 @pytest.mark.parametrize("reuse", [True, False])
-@pytest.mark.parametrize("bb", [128, 0])
-def test_src_sorted_batches(bb, reuse, hints):
-    """Src-sorted R-MAT batches (the sorted bulk build): the ops of a warp
-    hit the same tables and race for the same free slots; duplicates of one key sit
-    next to each other with different weights (Q1 membership rule)."""
+@pytest.mark.parametrize("bb,set_variant", [(128, False), (0, False), (32, False), (64, True),
+                                            (32, True)])
+def test_src_sorted_batches(bb, set_variant, reuse, hints):
+    """Src-sorted R-MAT batches (the sorted bulk build) take the
+    same-source grouped path (a3, k_insert_sorted): the warp owning a row's first op
+    installs the whole row, a chain's new keys going to its next free slots in one
+    pass; rows with many chains (hubs) stay on the per-op path.  Duplicates of one key
+    sit next to each other with different weights (Q1 membership rule); a third is
+    deleted and re-inserted (tombstones present); every layout incl. the set variant
+    and 32-B buckets (chains overflow into several new buckets per group)."""
     from paper_conf_ipps_awadapo20_b200 import Graph
     scale = 15
     nv = 1 << scale
     s, d = wl.rmat_edges(17, 0, 600_000, scale, wl.GRAPH500)
-    w = wl.weights(17, 0, s.size)
+    w = None if set_variant else wl.weights(17, 0, s.size)
     order = np.lexsort((d, s))
-    s, d, w = s[order], d[order], w[order]
+    s, d = s[order], d[order]
+    if w is not None:
+        w = w[order]
     h = torch.bincount(torch.from_numpy(s.astype(np.int64)), minlength=nv).to(torch.int32)
-    g = Graph(nv, h.cuda() if hints else None, bucket_bytes=bb, reuse_tombstones=reuse)
+    g = Graph(nv, h.cuda() if hints else None, bucket_bytes=bb, reuse_tombstones=reuse,
+              set_variant=set_variant)
     o = Oracle(nv)
     half = s.size // 2
+    W = (lambda x: None) if w is None else (lambda x: w[x])
     for lo, hi in ((0, half), (half, s.size)):
-        assert g.insert_edges(cuda(s[lo:hi]), cuda(d[lo:hi]), cuda(w[lo:hi]), count=True) == \
-            o.insert_edges(s[lo:hi], d[lo:hi], w[lo:hi])[1]
+        sl = slice(lo, hi)
+        assert g.insert_edges(cuda(s[sl]), cuda(d[sl]), cuda(W(sl)), count=True) == \
+            o.insert_edges(s[sl], d[sl], W(sl))[1]
     cand = check_against_oracle(g, o, "sorted insert")
     check_queries(g, o, s[::5], d[::5], cand, "sorted queries")
     # delete a sorted third, re-insert it sorted (tombstone reuse path when enabled)
     m = slice(0, s.size // 3)
     assert g.delete_edges(cuda(s[m]), cuda(d[m]), count=True) == o.delete_edges(s[m], d[m])[1]
-    assert g.insert_edges(cuda(s[m]), cuda(d[m]), cuda(w[m]), count=True) == \
-        o.insert_edges(s[m], d[m], w[m])[1]
+    assert g.insert_edges(cuda(s[m]), cuda(d[m]), cuda(W(m)), count=True) == \
+        o.insert_edges(s[m], d[m], W(m))[1]
     check_against_oracle(g, o, "sorted churn")
+    # a sorted batch of keys that all exist already (replace path) plus new ones
+    m2 = slice(s.size // 4, s.size // 2)
+    assert g.insert_edges(cuda(s[m2]), cuda(d[m2]), cuda(W(m2)), count=True) == \
+        o.insert_edges(s[m2], d[m2], W(m2))[1]
+    check_against_oracle(g, o, "sorted replace")
+    g.close()
+
+
+@pytest.mark.parametrize("retry_cap", [None, 1000])
+def test_src_sorted_pool_exhaustion(retry_cap):
+    """The sorted path in retry mode: groups whose new buckets cannot be allocated
+    hand their overflow ops to the retry list (re-run by k_edges after the pool grows)."""
+    code = r"""
+import numpy as np, sys
+sys.path.insert(0, %r)
+import workloads as wl
+from oracle import Oracle
+from tests.gpu_util import check_against_oracle, cuda
+from paper_conf_ipps_awadapo20_b200 import Graph
+nv = 4096
+g = Graph(nv, pool_bytes=4096, bucket_bytes=32)
+o = Oracle(nv)
+for b in range(3):
+    s, d, w = wl.uniform_edges(2, b, 300_000, nv)
+    order = np.argsort(s, kind="stable")
+    s, d, w = s[order], d[order], w[order]
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+check_against_oracle(g, o, "sorted retry")
+print("OK", g.stats()["pool_buckets"])
+""" % os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, DG_TEST_RETRY_PATH="1", DG_HOT_STEPS="0")
+    if retry_cap:
+        env["DG_TEST_RETRY_CAP"] = str(retry_cap)
+    r = subprocess.run([sys.executable, "-c", code], env=env, capture_output=True, text=True,
+                       timeout=600)
+    assert r.returncode == 0 and "OK" in r.stdout, r.stderr[-3000:]
 
 
 def test_freed_buckets_are_reused():
