@@ -145,8 +145,8 @@ typedef struct dg_stats {
   uint64_t overflow_buckets;  /* chained buckets currently linked into tables */
   uint64_t free_buckets;      /* buckets on the free stack */
   uint64_t pool_buckets;      /* buckets mapped in the pool (sum over size classes) */
-  uint64_t bump_buckets;      /* high-water mark: buckets ever handed out (base + chained;
-                                 sum over size classes) */
+  uint64_t bump_buckets;      /* high-water mark: buckets ever handed out (home, base and
+                                 chained; sum over size classes) */
   uint64_t live_pairs;        /* stored edges (sum of degrees) */
   uint64_t tombstones;        /* deleted-key slots not yet reclaimed */
   uint64_t max_chain;         /* longest bucket chain (in buckets) */
@@ -158,8 +158,8 @@ typedef struct dg_stats {
   uint64_t exchange;          /* batch routing: 0 = none (single GPU), 1 = NCCL all-to-all,
                                  2 = fused partition + peer stores into NVLink-mapped windows */
   uint64_t table_bytes;       /* bytes of the linked (base+overflow) buckets */
-  uint64_t bump_bytes;        /* bytes of all buckets ever handed out (what the streaming
-                                 purge / tombstone sweeps read) */
+  uint64_t bump_bytes;        /* bytes of all buckets ever handed out, home buckets included
+                                 (what the streaming purge / tombstone sweeps read) */
 } dg_stats;
 
 /* Fills defaults: load_factor 0.7, bucket_bytes 128, directed 1, pool_bytes 0,

@@ -390,6 +390,9 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   static const bool no_sorted = std::getenv("DG_NO_SORTED_PATH") != nullptr;
   // (large batches only: a small batch would pay a second launch for little)
   a.sorted_path = (!no_sorted && !mirror && epoch == g->validated_epoch && n >= (1u << 18)) ? 1u : 0u;
+  static const u32 excl_chains = std::getenv("DG_EXCL_CHAINS")
+                                     ? (u32)std::atoi(std::getenv("DG_EXCL_CHAINS")) : 64u;
+  a.excl_chains = excl_chains;
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
@@ -507,7 +510,8 @@ dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
                              g->set ? 1u : 0u, nbnew, nbold, degs, s));
   u64 tot[2 + dg::kClasses] = {};
   for (int c = 0; c < g->ncls; ++c) {
-    DG_CK(dg::scan_class_offsets(nbnew, n, (u32)c, nboff + c * m, &g->scan_temp, &g->scan_bytes, s));
+    DG_CK(dg::scan_class_offsets(nbnew, n, (u32)c, g->adaptive ? 0u : 1u, nboff + c * m,
+                                 &g->scan_temp, &g->scan_bytes, s));
     DG_CK(cudaMemcpyAsync(&tot[2 + c], nboff + c * m + n, 8, cudaMemcpyDeviceToHost, s));
   }
   DG_CK(dg::scan_exclusive_u64(nbold, obo, m, &g->scan_temp, &g->scan_bytes, s));
@@ -620,6 +624,8 @@ static void destroy_graph(dg_graph g) {
   if (g->router) dg::router_destroy(g->router);
   g->dir.release();
   g->degv.release();
+  g->home.release();  // (a view into pool[0]'s reservation: before the pools)
+  g->nbsv.release();
   for (auto& p : g->pool) p.release();
   for (auto& p : g->stack) p.release();
   if (g->ctl) cudaFree(g->ctl);
@@ -659,6 +665,9 @@ static void destroy_graph(dg_graph g) {
 static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_global,
                           const u32* hints_local, u64 slack_buckets, cudaStream_t s) {
   if (count == 0) return DG_OK;
+  // uniform layouts address home buckets by row in 30 bits (2^30 rows of 128 B are
+  // 128 GiB: more than the tables could hold anyway)
+  if (!g->adaptive && row0 + count > dg::kMaxHomeRows) return DG_ERR_UNSUPPORTED;
   u64* nb = nullptr;   // #buckets | class << 40
   u64* off = nullptr;  // per class: count + 1 offsets
   DG_CK(cudaMallocAsync(&nb, (count + 1) * 8, s));
@@ -667,7 +676,8 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
                                    g->lf_milli, g->BC, g->adaptive ? 1u : 0u, g->set ? 1u : 0u, s));
   u64 total[dg::kClasses] = {0, 0, 0};
   for (int c = 0; c < g->ncls; ++c) {
-    DG_CK(dg::scan_class_offsets(nb, count, (u32)c, off + c * (count + 1), &g->scan_temp,
+    DG_CK(dg::scan_class_offsets(nb, count, (u32)c, g->adaptive ? 0u : 1u, off + c * (count + 1),
+                                 &g->scan_temp,
                                  &g->scan_bytes, s));
     DG_CK(cudaMemcpyAsync(&total[c], off + c * (count + 1) + count, 8, cudaMemcpyDeviceToHost, s));
   }
@@ -695,6 +705,14 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
   e = g->degv.ensure((row0 + count) * sizeof(u32), 0, s);
   if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
   DG_CK(e);
+  if (!g->adaptive) {  // (k_init_rows writes every new home bucket and chain-count byte)
+    e = g->home.ensure((row0 + count) * g->bucket_bytes, -1, s);
+    if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
+    DG_CK(e);
+    e = g->nbsv.ensure(row0 + count, -1, s);
+    if (e == cudaErrorMemoryAllocation) return DG_ERR_OUT_OF_MEMORY;
+    DG_CK(e);
+  }
   g->rows = row0 + count;
   {  // re-sizing flags: one bit per row (transient: a growth simply clears them)
     const u64 words = (g->rows + 31) / 32 + 1;
@@ -765,15 +783,27 @@ dg_status dg_create(const dg_config* cfg, uint64_t num_vertices, const uint32_t*
   g->nv = num_vertices;
 
   const size_t total_mem = prop.totalGlobalMem;
+  const u64 max_rows = (kMaxVertices + g->nranks - 1) / g->nranks + 1;
   for (int c = 0; c < g->ncls; ++c) {
-    if (g->pool[c].reserve(g->device, total_mem) != cudaSuccess) return fail(DG_ERR_CUDA);
+    if (!g->adaptive) {
+      // the pool (bucket ids < 2^30) and, 2^31 buckets after its base, the home buckets
+      const u64 bb = g->bucket_bytes;
+      if (g->pool[c].reserve_pair(g->device, std::min<u64>(total_mem, bb << 30), bb << 31,
+                                  std::min<u64>(max_rows, dg::kMaxHomeRows) * bb,
+                                  g->home) != cudaSuccess)
+        return fail(DG_ERR_CUDA);
+    } else if (g->pool[c].reserve(g->device, total_mem) != cudaSuccess) {
+      return fail(DG_ERR_CUDA);
+    }
     if (g->stack[c].reserve(g->device, total_mem / g->cbytes(c) * 4 + (2u << 20)) != cudaSuccess)
       return fail(DG_ERR_CUDA);
   }
-  const u64 max_rows = (kMaxVertices + g->nranks - 1) / g->nranks + 1;
   if (g->dir.reserve(g->device, max_rows * sizeof(dg::DirEntry)) != cudaSuccess ||
-      g->degv.reserve(g->device, max_rows * sizeof(u32)) != cudaSuccess)
+      g->degv.reserve(g->device, max_rows * sizeof(u32)) != cudaSuccess ||
+      (!g->adaptive && g->nbsv.reserve(g->device, std::min<u64>(max_rows, dg::kMaxHomeRows)) !=
+                           cudaSuccess))
     return fail(DG_ERR_CUDA);
+
   if (cudaMalloc(&g->ctl, sizeof(dg::DevCtl)) != cudaSuccess) return fail(DG_ERR_CUDA);
   if (cudaMemsetAsync(g->ctl, 0, sizeof(dg::DevCtl), s) != cudaSuccess) return fail(DG_ERR_CUDA);
   if (cudaMallocHost(&g->hctl, sizeof(dg::DevCtl)) != cudaSuccess) return fail(DG_ERR_CUDA);
@@ -1207,13 +1237,17 @@ dg_status dg_get_stats(dg_graph g, dg_stats* out, void* stream) {
   out->exchange = !g->router ? 0 : dg::router_fused(g->router) ? 2 : 1;
   out->base_buckets = h.base_buckets;
   out->overflow_buckets = h.linked_buckets - h.base_buckets;
-  out->pool_bytes = g->dir.mapped() + g->degv.mapped();
+  out->pool_bytes = g->dir.mapped() + g->degv.mapped() + g->home.mapped() + g->nbsv.mapped();
   for (int c = 0; c < g->ncls; ++c) {
     out->free_buckets += g->hctl->stack_size[c];
     out->pool_buckets += g->cap[c];
     out->bump_buckets += g->hctl->bump[c];
     out->bump_bytes += (u64)g->hctl->bump[c] * g->cbytes(c);
     out->pool_bytes += g->pool[c].mapped() + g->stack[c].mapped();
+  }
+  if (!g->adaptive) {  // the home buckets (one per row) are handed out and swept too
+    out->bump_buckets += g->rows;
+    out->bump_bytes += g->rows * g->bucket_bytes;
   }
   out->live_pairs = h.live;
   out->tombstones = h.tombs;

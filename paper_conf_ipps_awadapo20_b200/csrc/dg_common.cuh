@@ -15,9 +15,18 @@
 //   free stack : u32[pool capacity] of reclaimed bucket indices + bump cursor
 //   ctl        : DevCtl (allocator cursors, counters, validation epochs)
 //
+// Home buckets (uniform layouts): chain 0 of row r is bucket r of a
+// separate HOME pool indexed by row, mapped exactly 2^31 buckets after the bucket
+// pool's base (so `pool + id * W` addresses both; home ids = kHomeBit | row).  Home
+// buckets are ordinary buckets (same slots, next, owner = row).  A probe reads the
+// row's chain count from a 1-byte-per-row array (`nbs`, min(nb, 255): L2-resident,
+// 4.8 MB on cfg2): a key that hashes to chain 0 goes straight to the home bucket
+// without the directory; the others read the directory {xbase, nb} for chain j >= 1,
+// which starts at pool bucket xbase + j - 1.
+//
 // Bucket ids: bits 31..30 = size class (index of the pool the bucket lives in),
 // bits 29..0 = index in that pool.  Uniform layouts use class 0 only (one pool of
-// `bucket_bytes` buckets).  The degree-adaptive layout (DG_FLAG_ADAPTIVE, SURVEY
+// `bucket_bytes` buckets) plus home ids.  The degree-adaptive layout (DG_FLAG_ADAPTIVE, SURVEY
 // §8(f) row 4, "hash tables with varying slab sizes") keeps three pools:
 // class c holds 32 << c byte buckets (32 / 64 / 128 B), and every bucket of a row
 // (base and chained) has the row's class, so a bucket id alone fixes its geometry.
@@ -38,6 +47,8 @@ constexpr u32 kClassShift = 30;           // bucket id = class << 30 | index
 constexpr u32 kIdxMask = (1u << kClassShift) - 1u;
 constexpr int kClasses = 3;               // adaptive size classes: 32, 64, 128 B
 constexpr u64 kNbMask = (1ull << 40) - 1; // packed (#buckets | class << 40) entries
+constexpr u32 kHomeBit = 1u << 31;        // uniform layouts: home bucket id = kHomeBit | row
+constexpr u64 kMaxHomeRows = 1ull << 30;  // rows per rank of a uniform layout
 
 struct __align__(8) DirEntry {
   u32 base;    // first base bucket
@@ -63,7 +74,9 @@ struct DevCtl {
 };
 
 struct Tables {
-  DirEntry* dir;
+  DirEntry* dir;     // uniform layouts: {xbase, nb}; adaptive: {first base bucket, nb}
+  u32* home;         // uniform layouts: home bucket of every row (chain 0), W words each
+  uint8_t* nbs;      // uniform layouts: min(nb, 255) per row
   u32* deg;          // exact degree per local row
   u32* pool[kClasses];   // bucket pool per size class
   u32* stack[kClasses];  // free stack per size class (bucket ids)
@@ -213,13 +226,18 @@ struct Geo {
   typedef Lay<G, S> LY;
   u32* p;     // first word of the bucket
   u32 units;  // 16-B units
+  bool home;  // a home bucket (uniform layouts): not on the free stack
   __device__ __forceinline__ Geo(const Tables& t, u32 id) {
     if constexpr (A) {
       const u32 c = id >> kClassShift;
       units = 2u << c;
       p = by_class(t.pool, c) + (u64)(id & kIdxMask) * (8u << c);
+      home = false;
     } else {
+      // home bucket r (id 2^31 | r) lies 2^31 buckets after the pool base
+      // (VmmArray::reserve_pair), so one formula addresses both
       units = G;
+      home = (id & kHomeBit) != 0;
       p = t.pool[0] + (u64)id * LY::W;
     }
   }
@@ -238,6 +256,14 @@ struct Geo {
     else return LY::BC;
   }
 };
+
+// Head of chain j of a row from its directory entry: uniform layouts start chain 0 in
+// the row's home bucket and chain j >= 1 at xbase + j - 1; adaptive: base + j.
+template <bool A>
+__device__ __forceinline__ u32 chain_head(u32 base, u32 row, u32 j) {
+  if constexpr (A) return base + j;
+  else return j == 0 ? (kHomeBit | row) : base + j - 1;
+}
 
 // units of a bucket id (no pool access)
 template <int G, bool A>

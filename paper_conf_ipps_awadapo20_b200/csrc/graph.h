@@ -35,6 +35,8 @@ struct dg_graph_s {
   uint64_t rows = 0;      // local rows
 
   dg::VmmArray dir, degv;
+  dg::VmmArray home;  // uniform layouts: one home bucket per row (chain 0)
+  dg::VmmArray nbsv;  // uniform layouts: min(nb, 255) per row (the probe's chain count)
   dg::VmmArray pool[dg::kClasses], stack[dg::kClasses];  // per size class
   uint32_t cap[dg::kClasses] = {0, 0, 0};      // buckets mapped in each pool
   uint64_t bump_ub[dg::kClasses] = {0, 0, 0};  // host upper bounds of the device bump cursors
@@ -100,6 +102,8 @@ struct dg_graph_s {
   dg::Tables tables() const {
     dg::Tables t;
     t.dir = reinterpret_cast<dg::DirEntry*>(dir.ptr());
+    t.home = adaptive ? nullptr : reinterpret_cast<uint32_t*>(home.ptr());
+    t.nbs = adaptive ? nullptr : reinterpret_cast<uint8_t*>(nbsv.ptr());
     t.deg = reinterpret_cast<uint32_t*>(degv.ptr());
     for (int c = 0; c < dg::kClasses; ++c) {
       t.pool[c] = c < ncls ? reinterpret_cast<uint32_t*>(pool[c].ptr()) : nullptr;

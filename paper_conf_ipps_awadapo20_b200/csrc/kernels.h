@@ -34,6 +34,7 @@ struct EdgeBatch {
   u32 chunk;             // insert: buckets per per-warp allocation chunk (set by the launcher)
   u32 sorted_path;       // insert: k_validate checked this epoch's sources for sortedness;
                          // a src-sorted batch runs k_insert_sorted (a3), others k_edges
+  u32 excl_chains;       // k_insert_sorted: rows with at most this many chains are owned
 };
 
 // `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1
@@ -60,7 +61,8 @@ cudaError_t launch_initial_buckets(u64* nb, u64 count, u64 row0, const u32* hint
                                    const u32* hints_local, u32 nranks, u32 rank, u32 lf_milli,
                                    u32 bc, u32 adaptive, u32 set, cudaStream_t s);
 // off[r] = sum over r' < r of the class-c buckets of nbc[r'] (count + 1 entries)
-cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u64* off, void** temp,
+// (home = 1: uniform layouts, chain 0 in the home bucket: nb - 1 pool buckets per row)
+cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u32 home, u64* off, void** temp,
                                size_t* temp_bytes, cudaStream_t s);
 // out[i] = sum of in[0..i) for i < count (temp storage grows as needed)
 cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,

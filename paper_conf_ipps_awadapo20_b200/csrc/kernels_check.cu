@@ -38,10 +38,13 @@ __global__ void __launch_bounds__(256) k_check(Tables t, u64 nv, u32 rank, Invar
   for (u64 row = warp; row < t.rows; row += nwarps) {
     const DirEntry de = t.dir[row];
     const u64 gid = row * t.nranks + rank;  // global vertex id of the row
+    // uniform layouts: the probe's chain-count byte must agree with the directory
+    if (!A && lane == 0 && t.nbs[row] != (de.nb < 255u ? de.nb : 255u))
+      bump(&out->owner_mismatch);
     unsigned long long live = 0, tombs = 0, buckets = 0;
     bool bad = false;
     for (u32 j = lane; j < de.nb; j += 32) {
-      u32 b = de.base + j;
+      u32 b = chain_head<A>(de.base, (u32)row, j);
       u64 len = 0;
       bool seen_empty = false, not_suffix = false;
       while (b != kNil) {
@@ -55,6 +58,7 @@ __global__ void __launch_bounds__(256) k_check(Tables t, u64 nv, u32 rank, Invar
           bump(&out->owner_mismatch);
           bad = true;
         }
+
         for (u32 uu = 0; uu < gb.units; ++uu) {
 #pragma unroll
           for (int k = 0; k < LY::SPU; ++k) {
@@ -87,7 +91,7 @@ __global__ void __launch_bounds__(256) k_check(Tables t, u64 nv, u32 rank, Invar
         bump(&out->dup_unchecked_chains);
         continue;
       }
-      for (u32 b1 = de.base + j; b1 != kNil;) {
+      for (u32 b1 = chain_head<A>(de.base, (u32)row, j); b1 != kNil;) {
         const GEO g1(t, b1);
         for (u32 uu = 0; uu < g1.units; ++uu) {
           for (int k = 0; k < LY::SPU; ++k) {

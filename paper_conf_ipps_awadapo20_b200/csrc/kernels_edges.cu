@@ -13,15 +13,21 @@
 // WCWS):
 //   * a warp stages 32 consecutive ops of the batch with one coalesced load per
 //     input array;
-//   * every lane loads the directory entry of ITS op and issues an L2 prefetch of
-//     the op's first bucket, so 32 directory gathers and 32 bucket gathers per
-//     warp are in flight at once (memory-level parallelism is the bound);
+//   * uniform layouts: lane L reads its row's chain count from an L2-resident byte
+//     array; a key that hashes to chain 0 goes straight to the row's HOME bucket
+//     (addressed by row) without a directory access, the others read
+//     the directory entry for their chain's first bucket; the degree-adaptive layout
+//     reads the directory entry first;
 //   * a "group" of G = bucket_bytes/16 lanes then probes the G ops of its lanes one
 //     after another, each lane holding 16 B of the bucket (one 128-B bucket = one
 //     coalesced request of 8 lanes); 32/G groups per warp probe independently;
-//   * a new pair is installed with one 64-bit CAS on (key, value); a deletion is a
-//     32-bit CAS key -> tombstone, so exactly one of several racing deleters wins
-//     and degrees stay exact (Alg1:L9-10);
+//   * a new pair is installed with one 64-bit CAS on (key, value) into the chain's
+//     first free slot; after a lost CAS on an EMPTY slot the next slot of the bucket
+//     is tried with a 32-bit key CAS (EMPTY -> key) followed by a plain value store
+//     (legal under phase concurrency: no reader runs during an insert phase;
+//     DESIGN.md §4.2).  The set variant always installs with a 32-bit key CAS.  A
+//     deletion is a 32-bit CAS key -> tombstone, so exactly one of several racing
+//     deleters wins and degrees stay exact (Alg1:L9-10);
 //   * degree updates are one fire-and-forget atomic per added/removed key; batch
 //     counters are reduced per warp.
 #include <atomic>
@@ -50,6 +56,7 @@ enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 #ifndef DG_SLOT_WALK_MAIN
 #define DG_SLOT_WALK_MAIN 1
 #endif
+
 
 // ----------------------------------------------------------- allocator (a8) ----
 // Phase-concurrent free stack + bump cursor: during an insert
@@ -236,9 +243,25 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
   u32 nbase = 0;
   if (pend) {
     // base/nb never change during an edge phase; only deg is written (atomics)
-    const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
-    head = de.x + bucket_of(v, de.y);
-    nbase = de.y;
+    if constexpr (A) {
+      const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
+      head = de.x + bucket_of(v, de.y);
+      nbase = de.y;
+    } else {
+      // uniform layouts: the row's chain count from the L2-resident byte array; a key
+      // of chain 0 goes straight to the row's home bucket, the others read the
+      // directory for the chain's first bucket
+      const u32 nbb = __ldg(t.nbs + row);
+      const u32 j0 = nbb < 255u ? bucket_of(v, nbb) : 1u;
+      if (j0 == 0) {
+        head = kHomeBit | row;
+        nbase = nbb;
+      } else {
+        const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
+        head = chain_head<false>(de.x, row, bucket_of(v, de.y));
+        nbase = de.y;
+      }
+    }
   }
   u32 cur = head;
   bool found = false;
@@ -337,7 +360,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
               // metric + rehash)
               if (++steps == t.hot_steps && t.hot_flags) {
                 const u32 dr = ld_relaxed_u32(t.deg + row);
-                if (dr > nbase * GEO::bc_u(units)) {
+                if (dr > nbase * GEO::bc_u(units)) {  // (home chains hold one less)
                   const u32 bit = 1u << (row & 31);
                   if (!(atomicOr(&t.hot_flags[row >> 5], bit) & bit)) {
                     const u32 k = atomicAdd(&t.ctl->hot_count, 1u);
@@ -383,14 +406,16 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
         if (DG_SLOT_WALK_MAIN || !MAIN) {
           if ((u32)ffo == kEmpty) {
             // word index of the slot in its bucket from the address (pools are aligned
-            // to the bucket size), so no bucket pointer is kept live
+            // to the bucket size), so no bucket pointer is kept live; the slots end
+            // before the (next, owner) words, or before the header of a home bucket
             const u32 nw = 4 * units_of<G, A>(cur);
+            const u32 lim = nw - 2u;
             u32 off = (u32)(reinterpret_cast<uintptr_t>(ff) >> 2) & (nw - 1u);
             u32* p = ff;
 #if DG_SLOT_WALK_ONCE
-            if ((off += (S ? 1u : 2u)) < nw - 2u) {  // one further slot, then re-scan
+            if ((off += (S ? 1u : 2u)) < lim) {  // one further slot, then re-scan
 #else
-            while ((off += (S ? 1u : 2u)) < nw - 2u) {
+            while ((off += (S ? 1u : 2u)) < lim) {
 #endif
               p += S ? 1 : 2;
               const u32 k2 = atomicCAS(p, kEmpty, v);
@@ -576,11 +601,13 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
 // and linked for the overflow in the same pass.  Chains stay prefix-filled (EMPTY
 // slots only at the tail) because every group fills from the first free
 // slot on, in order, before the next group of that chain runs.  Rows with many
-// chains (nb > kExclChains: hubs, whose ops spread over many chains and would make
+// chains (nb > a.excl_chains: hubs, whose ops spread over many chains and would make
 // one warp walk a long run alone) go through the lock-free per-op path of k_edges
 // (run_ops) in every chunk, as in unsorted batches.
 //
-constexpr u32 kExclChains = 16;
+#ifndef DG_SORTED_MINB
+#define DG_SORTED_MINB 2
+#endif
 
 // position of the n-th (0-based) set bit of m
 __device__ __forceinline__ u32 nth_bit(u32 m, u32 n) {
@@ -607,7 +634,7 @@ __device__ __forceinline__ void install_owned(const Tables& t, const EdgeBatch& 
   u32 j = 0, b = kNil, hit_word = kNil, tail = kNil, e = 0;
   if (writer) {
     j = bucket_of(v, nb);
-    b = base + j;
+    b = chain_head<A>(base, row, j);
     while (true) {
       const GEO gb(t, b);
       u32 first_empty = kNil;
@@ -639,18 +666,19 @@ __device__ __forceinline__ void install_owned(const Tables& t, const EdgeBatch& 
   const u32 bct = fresh ? GEO(t, tail).bc() : 0u;
   const u32 cls = A ? (tail >> kClassShift) : 0u;
   const u32 avail = fresh ? bct - e : 0u;
-  // overflow: ranks >= avail go to new buckets of bct slots (same class as the row)
+  // overflow: ranks >= avail go to new pool buckets of bcn slots (the row's class)
+  const u32 bcn = bct;
   const bool over = fresh && r >= avail;
   const u32 q = over ? r - avail : 0u;
-  const bool want = over && q % bct == 0;  // the first key of each new bucket allocates it
+  const bool want = over && q % bcn == 0;  // the first key of each new bucket allocates it
   u32 got = kNil;
   if (__any_sync(FULL, want)) got = alloc_bucket_chunk<A>(t, want, cls, a.chunk);
-  // the new buckets of the group, k-th held by the lane of rank avail + k*bct
-  const u32 kb = q / bct;
+  // the new buckets of the group, k-th held by the lane of rank avail + k*bcn
+  const u32 kb = over ? q / bcn : 0u;
   u32 mine = kNil, pred = tail;
   {
-    const u32 src_mine = over ? nth_bit(gm, avail + kb * bct) : lane;
-    const u32 src_pred = (over && kb > 0) ? nth_bit(gm, avail + (kb - 1) * bct) : lane;
+    const u32 src_mine = over ? nth_bit(gm, avail + kb * bcn) : lane;
+    const u32 src_pred = (over && kb > 0) ? nth_bit(gm, avail + (kb - 1) * bcn) : lane;
     const u32 m1 = __shfl_sync(FULL, got, src_mine);
     const u32 m2 = __shfl_sync(FULL, got, src_pred);
     if (over) {
@@ -678,7 +706,7 @@ __device__ __forceinline__ void install_owned(const Tables& t, const EdgeBatch& 
   const bool store = fresh && !group_failed;
   if (store) {
     const u32 bk = over ? mine : tail;
-    const u32 slot = over ? q % bct : e + r;
+    const u32 slot = over ? q % bcn : e + r;
     u32* p = GEO(t, bk).p + (S ? slot : 2 * slot);
     if (S) *p = v;
     else *reinterpret_cast<unsigned long long*>(p) = pack_pair(v, w);
@@ -691,7 +719,7 @@ __device__ __forceinline__ void install_owned(const Tables& t, const EdgeBatch& 
 }
 
 template <int G, int S, bool A>
-__global__ void __launch_bounds__(kEdgeBlock, 2) k_insert_sorted(Tables t, EdgeBatch a) {
+__global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<Lanes<G, OP_INSERT>::L> g;
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;      // rejected (Q7)
@@ -715,9 +743,9 @@ __global__ void __launch_bounds__(kEdgeBlock, 2) k_insert_sorted(Tables t, EdgeB
     const u32 w = (valid && a.w) ? a.w[i] : 0u;
     const u32 prev = lo ? a.src[lo - 1] : kNil;  // the row of the op before the chunk
     const u32 row = (t.nranks == 1) ? u : u / t.nranks;
-    uint2 de = make_uint2(0, 0);
+    uint2 de = make_uint2(0, 0);  // {base (uniform: xbase), nb}
     if (valid) de = ld_dir(t.dir + row);
-    const bool excl = valid && de.y <= kExclChains;
+    const bool excl = valid && de.y <= a.excl_chains;
     // 1. rows with many chains: the per-op lock-free path, every chunk its own ops
     const bool cas = valid && !excl;
     if (__any_sync(FULL, cas))

@@ -63,21 +63,24 @@ cudaError_t scan_exclusive_u64(const u64* in, u64* out, u64 count, void** temp,
 }
 
 // buckets of class c in a packed (#buckets | class << 40) entry
+// (home: uniform layouts keep chain 0 in the row's home bucket, so a row takes
+// #buckets - 1 buckets from the pool)
 struct ClassCount {
   const u64* nbc;
   u64 n;
   u32 c;
+  u32 home;
   __host__ __device__ u64 operator()(u64 i) const {
     if (i >= n) return 0ull;
     const u64 v = nbc[i];
-    return (u32)(v >> 40) == c ? (v & kNbMask) : 0ull;
+    return (u32)(v >> 40) == c ? (v & kNbMask) - home : 0ull;
   }
 };
 
-cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u64* off, void** temp,
+cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u32 home, u64* off, void** temp,
                                size_t* temp_bytes, cudaStream_t s) {
   auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0),
-                                            ClassCount{nbc, count, c});
+                                            ClassCount{nbc, count, c, home});
   size_t need = 0;
   cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, off, (int64_t)(count + 1), s);
   if (e != cudaSuccess) return e;
@@ -96,9 +99,13 @@ cudaError_t scan_class_offsets(const u64* nbc, u64 count, u32 c, u64* off, void*
 // Row r gets nbc[r] consecutive base buckets of its class c, starting at
 // cb.base0[c] + cb.off[c][r]; each base bucket records its owner row.  `rows`
 // (nullable) maps r to a directory row (re-sizing), else row = row0 + r.
+// Uniform layouts (t.home set): chain 0 lives in the row's home bucket (all slots
+// EMPTY, next NIL, owner = row), the other nb - 1 base buckets are consecutive from
+// xbase in the pool, and the probe's chain-count byte nbs[row] = min(nb, 255).
 __global__ void k_init_rows(Tables t, u64 row0, u64 count, const u32* rows, const u64* nbc,
                             ClassBases cb) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
+  const u32 home = t.home ? 1u : 0u;
   for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < count; r += stride) {
     const u64 v = nbc[r];
     const u32 c = (u32)(v >> 40);
@@ -112,7 +119,14 @@ __global__ void k_init_rows(Tables t, u64 row0, u64 count, const u32* rows, cons
     t.deg[row] = 0;
     const u32 wc = by_class(cb.words, c);
     u32* pool = by_class(t.pool, c);
-    for (u32 k = 0; k < n; ++k) pool[(u64)(idx + k) * wc + wc - 1] = row;
+    for (u32 k = 0; k + home < n; ++k) pool[(u64)(idx + k) * wc + wc - 1] = row;
+    if (home) {
+      uint4* hb = reinterpret_cast<uint4*>(t.home + (u64)row * wc);
+      const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
+      for (u32 uu = 0; uu + 1 < wc / 4; ++uu) hb[uu] = empty4;
+      hb[wc / 4 - 1] = make_uint4(kEmpty, kEmpty, kNil, row);
+      t.nbs[row] = (uint8_t)(n < 255u ? n : 255u);
+    }
     if (rows && t.hot_flags) atomicAnd(&t.hot_flags[row >> 5], ~(1u << (row & 31)));
   }
 }
@@ -257,7 +271,7 @@ __global__ void __launch_bounds__(256) k_export_fill(Tables t, const u64* ro, u3
     }
     u64 pos = ro[row];
     for (u32 k = 0; k < de.nb; ++k) {
-      u32 b = de.base + k;
+      u32 b = chain_head<A>(de.base, (u32)row, k);
       while (b != kNil) {
         const Geo<G, S, A> gb(t, b);
         const uint4 q = ld_unit(gb, g.gl);
@@ -282,7 +296,7 @@ __global__ void __launch_bounds__(256) k_export_big(Tables t, const u64* ro, u32
     if (threadIdx.x == 0) cursor = ro[row];
     __syncthreads();
     for (u32 k = gib; k < de.nb; k += ngb) {
-      u32 b = de.base + k;
+      u32 b = chain_head<A>(de.base, row, k);
       while (b != kNil) {
         const Geo<G, S, A> gb(t, b);
         const uint4 q = ld_unit(gb, g.gl);
@@ -378,7 +392,7 @@ __global__ void __launch_bounds__(256) k_stats(Tables t, StatsOut* out, u32* big
       if (g.gl == 0) big[1 + atomicAdd(big, 1u)] = (u32)row;
       continue;
     }
-    for (u32 k = 0; k < de.nb; ++k) stats_chain<G, S, A>(t, g, de.base + k, a);
+    for (u32 k = 0; k < de.nb; ++k) stats_chain<G, S, A>(t, g, chain_head<A>(de.base, (u32)row, k), a);
   }
   if (g.gl == 0) {
     if (nbase) atomicAdd(&out->base_buckets, nbase);
@@ -393,8 +407,9 @@ __global__ void __launch_bounds__(256) k_stats_big(Tables t, StatsOut* out, cons
   StatsAcc a;
   const u32 nbig = big[0];
   for (u32 i = blockIdx.x; i < nbig; i += gridDim.x) {
-    const DirEntry de = t.dir[big[1 + i]];
-    for (u32 k = gib; k < de.nb; k += ngb) stats_chain<G, S, A>(t, g, de.base + k, a);
+    const u32 row = big[1 + i];
+    const DirEntry de = t.dir[row];
+    for (u32 k = gib; k < de.nb; k += ngb) stats_chain<G, S, A>(t, g, chain_head<A>(de.base, row, k), a);
   }
   if (g.gl == 0) stats_flush(out, a);
 }
@@ -464,7 +479,9 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // of the pool (coalesced, G lanes per bucket); every live key in D becomes a
 // tombstone and the owner row's degree drops by one.
 // One launch per size class c: the pool of class c holds buckets of G units.
-template <int G, int S>
+// H: the home pool (uniform layouts; bucket r = row r's chain 0, header in the last
+// unit) instead of pool `cls`.
+template <int G, int S, bool H = false>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     const u32* __restrict__ filter, u32 fshift,
                                                     u32 epoch, u32 cls) {
@@ -482,8 +499,8 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   for (u32 i = threadIdx.x; i < kVdelFilterBits / 32; i += blockDim.x) sf[i] = filter[i];
   __syncthreads();
-  const u32 nbk = ld_relaxed_u32(&t.ctl->bump[cls]);
-  u32* const pool = by_class(t.pool, cls);
+  const u32 nbk = H ? (u32)t.rows : ld_relaxed_u32(&t.ctl->bump[cls]);
+  u32* const pool = H ? t.home : by_class(t.pool, cls);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b0 = gid; b0 < nbk; b0 += ng * U) {
@@ -551,16 +568,17 @@ cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const
     note_kernel(3);
     return cudaGetLastError();
   }
-  switch (lay) {
-#define DG_CASE(G_, S_)                                                                    \
-  case DG_LAY(G_, S_):                                                                     \
-    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);      \
+  switch (lay) {  // uniform layouts: the pool, then the home buckets
+#define DG_CASE(G_, S_)                                                                      \
+  case DG_LAY(G_, S_):                                                                       \
+    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);        \
+    k_vdel_sweep<G_, S_, true><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);  \
     break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
+  note_kernel(2);
   return cudaGetLastError();
 }
 
@@ -644,7 +662,7 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
   for (u64 x = gid; x < total; x += ng) {
     const u32 k = owner_of(boff, cnt, x);
     const u32 u = dedup[k];
-    u32 b = t.dir[u].base + (u32)(x - boff[k]);
+    u32 b = chain_head<A>(t.dir[u].base, u, (u32)(x - boff[k]));
     while (b != kNil) {
       const Geo<G, S, A> gb(t, b);
       const uint4 q = (A && g.gl >= gb.units) ? make_uint4(kEmpty, kEmpty, kEmpty, kEmpty)
@@ -657,7 +675,8 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
           lm &= lm - 1;
           const u32 v = g.shfl(LY::key(q, j), l);
           const DirEntry dv = t.dir[v];
-          if (purge_delete<G, S, A>(t, g, dv.base + bucket_of(u, dv.nb), u) && g.gl == 0)
+          if (purge_delete<G, S, A>(t, g, chain_head<A>(dv.base, v, bucket_of(u, dv.nb)), u) &&
+              g.gl == 0)
             atomicSub(&t.deg[v], 1u);
         }
       }
@@ -701,7 +720,7 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
     const u32 k = owner_of(boff, cnt, x);
     const u32 row = dedup[k] / t.nranks;
     const u32 j = (u32)(x - boff[k]);
-    u32 b = t.dir[row].base + j;
+    u32 b = chain_head<A>(t.dir[row].base, row, j);
     bool base_bucket = true;
     while (b != kNil) {
       const Geo<G, 0, A> gb(t, b);

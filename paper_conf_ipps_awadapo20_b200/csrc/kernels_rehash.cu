@@ -80,7 +80,7 @@ __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* 
     const u32 k = seg_of(obo, n, x);
     const u32 row = t.hot_list[k];
     const u32 gid_u = row * t.nranks + rank;  // global source id
-    u32 b = t.dir[row].base + (u32)(x - obo[k]);
+    u32 b = chain_head<A>(t.dir[row].base, row, (u32)(x - obo[k]));
     while (b != kNil) {
       const Geo<G, S, A> gb(t, b);
       const uint4 q = (A && g.gl >= gb.units) ? make_uint4(kEmpty, kEmpty, kEmpty, kEmpty)
@@ -110,7 +110,7 @@ __global__ void __launch_bounds__(256) k_hot_export(Tables t, u32 n, const u64* 
 }
 
 // every bucket of the old tables -> EMPTY, onto the free stack (base ones too: the
-// row moves to a new base range)
+// row moves to a new base range); a home bucket stays the row's (emptied here)
 template <int G, bool A>
 __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64* obo) {
   const Group<G> g;
@@ -121,7 +121,7 @@ __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64*
   for (u64 x = gid; x < total; x += ng) {
     const u32 k = seg_of(obo, n, x);
     const u32 row = t.hot_list[k];
-    u32 b = t.dir[row].base + (u32)(x - obo[k]);
+    u32 b = chain_head<A>(t.dir[row].base, row, (u32)(x - obo[k]));
     while (b != kNil) {
       const Geo<G, 0, A> gb(t, b);
       const bool in = !A || g.gl < gb.units;
@@ -129,7 +129,7 @@ __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64*
       const uint4 q = in ? ld_relaxed_v4(bp) : empty4;
       const u32 next = g.shfl(q.z, gb.units - 1);
       if (in) st_v4(bp, empty4);
-      if (g.gl == 0) {
+      if (g.gl == 0 && !gb.home) {
         const u32 c = b >> kClassShift;
         by_class(t.stack, c)[atomicAdd(&t.ctl->stack_size[c], 1u)] = b;
       }
@@ -142,12 +142,13 @@ __global__ void __launch_bounds__(256) k_hot_release(Tables t, u32 n, const u64*
 // the data structure"): one streaming pass over every allocated bucket; a bucket
 // holding a tombstone flags its owner row (bucket word W-1) for a compacting
 // re-build (the rows are then re-sized with flush = 1).
-template <int G, int S>
+// (H: the home pool of a uniform layout)
+template <int G, int S, bool H = false>
 __global__ void __launch_bounds__(256) k_tomb_sweep(Tables t, u32 cls) {
   typedef Lay<G, S> LY;
   const Group<G> g;
-  const u32 nbk = ld_relaxed_u32(&t.ctl->bump[cls]);
-  const u32* const pool = by_class(t.pool, cls);
+  const u32 nbk = H ? (u32)t.rows : ld_relaxed_u32(&t.ctl->bump[cls]);
+  const u32* const pool = H ? t.home : by_class(t.pool, cls);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b = gid; b < nbk; b += ng) {
@@ -182,13 +183,16 @@ cudaError_t launch_tomb_sweep(int lay, const Tables& t, int sms, cudaStream_t s)
     return cudaGetLastError();
   }
   switch (lay) {
-#define DG_CASE(G_, S_) \
-  case DG_LAY(G_, S_): k_tomb_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, 0); break;
+#define DG_CASE(G_, S_)                                       \
+  case DG_LAY(G_, S_):                                        \
+    k_tomb_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, 0);        \
+    k_tomb_sweep<G_, S_, true><<<blocks, 256, 0, s>>>(t, 0);  \
+    break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
+  note_kernel(2);
   return cudaGetLastError();
 }
 

@@ -176,7 +176,7 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
     for (u32 k0 = 0; k0 < maxc; k0 += G) {
       const bool act = k0 + g.gl < ncand;
       const u32 w = act ? __ldg(oadj + e + 1 + k0 + g.gl) : kEmpty;
-      const u32 head = dv.x + bucket_of(w, dv.y);
+      const u32 head = chain_head<A>(dv.x, v, bucket_of(w, dv.y));
       const u32 amask = __ballot_sync(FULL, act);
       uint4 q[G];
 #pragma unroll

@@ -68,6 +68,32 @@ cudaError_t VmmArray::reserve(int device, size_t max_bytes) {
     reserved_ = 0;
     return cudaErrorMemoryAllocation;
   }
+  va_bytes_ = reserved_;
+  return cudaSuccess;
+}
+
+cudaError_t VmmArray::reserve_pair(int device, size_t max_bytes, size_t hi_offset,
+                                   size_t hi_bytes, VmmArray& hi) {
+  const Driver& d = driver();
+  if (!d.ok) return cudaErrorNotSupported;
+  device_ = hi.device_ = device;
+  CUmemAllocationProp p = prop_for(device);
+  size_t g = 0;
+  if (d.GetGranularity(&g, &p, CU_MEM_ALLOC_GRANULARITY_RECOMMENDED) != CUDA_SUCCESS || !g)
+    return cudaErrorMemoryAllocation;
+  gran_ = hi.gran_ = g;
+  reserved_ = (std::max<size_t>(max_bytes, g) + g - 1) / g * g;
+  hi.reserved_ = (std::max<size_t>(hi_bytes, g) + g - 1) / g * g;
+  if (hi_offset % g || reserved_ > hi_offset) return cudaErrorInvalidValue;
+  const size_t total = hi_offset + hi.reserved_;
+  if (d.AddressReserve(&base_, total, g, 0, 0) != CUDA_SUCCESS) {
+    base_ = 0;
+    reserved_ = hi.reserved_ = 0;
+    return cudaErrorMemoryAllocation;
+  }
+  va_bytes_ = total;
+  hi.base_ = base_ + hi_offset;
+  hi.va_bytes_ = 0;
   return cudaSuccess;
 }
 
@@ -115,11 +141,11 @@ void VmmArray::release() {
     d.Release(handles_[i]);
     off += sizes_[i];
   }
-  d.AddressFree(base_, reserved_);
+  if (va_bytes_) d.AddressFree(base_, va_bytes_);
   handles_.clear();
   sizes_.clear();
   base_ = 0;
-  reserved_ = mapped_ = 0;
+  reserved_ = mapped_ = va_bytes_ = 0;
 }
 
 }  // namespace dg

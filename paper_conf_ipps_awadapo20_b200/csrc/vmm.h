@@ -26,6 +26,12 @@ class VmmArray {
 
   // Reserve `max_bytes` of virtual address space on `device`.
   cudaError_t reserve(int device, size_t max_bytes);
+  // One reservation for two arrays: this one at its start (`max_bytes`) and `hi` at
+  // byte offset `hi_offset` (`hi_bytes`), so that hi.ptr() - ptr() == hi_offset
+  // exactly (the home buckets sit 2^31 buckets after the pool: one address formula
+  // serves both, dg_common.cuh Geo).  Release `hi` before this array.
+  cudaError_t reserve_pair(int device, size_t max_bytes, size_t hi_offset, size_t hi_bytes,
+                           VmmArray& hi);
   // Ensure at least `bytes` are mapped; new memory is filled with `fill` (a byte
   // value, or -1 for no fill) on `stream`.
   cudaError_t ensure(size_t bytes, int fill, cudaStream_t stream);
@@ -39,6 +45,7 @@ class VmmArray {
  private:
   CUdeviceptr base_ = 0;
   size_t reserved_ = 0;
+  size_t va_bytes_ = 0;  // bytes of the reservation this array frees (0: a view into another's)
   size_t mapped_ = 0;
   size_t gran_ = 0;
   int device_ = 0;

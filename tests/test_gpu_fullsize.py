@@ -87,7 +87,7 @@ def _bench_step(g, o, nv, B, seed, base, where):
     us, ud, _ = wl.uniform_edges(seed, 7000, B // 2, nv, weights=False)
     qs, qd = np.concatenate([bs[idx], us]), np.concatenate([bd[idx], ud])
     hits = assert_same_answers(g, o, qs, qd, f"{where} queries")
-    assert hits >= B // 2 - 64
+    assert hits >= int((bs[idx] != bd[idx]).sum())  # every sampled base edge but self-loops
     ys, yd, _ = wl.uniform_edges(seed, 8000, B // 2, nv, weights=False)
     xs, xd = np.concatenate([s[: B // 2], ys]), np.concatenate([d[: B // 2], yd])
     got = g.delete_edges(_cu(xs), _cu(xd), count=True)

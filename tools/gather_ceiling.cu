@@ -52,6 +52,104 @@ __global__ void gather(uint4* __restrict__ buf, uint64_t nblocks, uint64_t iters
   if (acc == 0x12345678u) atomicAdd(sink, 1ull);
 }
 
+// ---------------------------------------------------- cp.async.bulk mode ----
+// Blackwell data movement instead of register loads: each warp keeps 2 x D random
+// 128-B buckets in flight as 1-D bulk copies (cp.async.bulk, SASS UBLKCP) into a
+// shared-memory ring, completion tracked by one mbarrier per stage (expect_tx),
+// double-buffered: while stage s is consumed the other stage's copies are in
+// flight.  In-flight requests per SM = warps x 2D, bounded by shared memory rather
+// than registers x occupancy.
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return (uint32_t)__cvta_generic_to_shared(p);
+}
+
+template <int D>
+__global__ void gather_bulk(const uint4* __restrict__ buf, uint64_t nblocks, uint64_t iters,
+                            unsigned long long* sink) {
+  extern __shared__ __align__(128) unsigned char smem[];
+  __shared__ __align__(8) unsigned long long bars[32][2];
+  const uint32_t w = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  uint4* ring = reinterpret_cast<uint4*>(smem) + (size_t)w * 2 * D * 8;  // [stage][D][8]
+  const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+  const uint32_t b0 = smem_u32(&bars[w][0]), b1 = smem_u32(&bars[w][1]);
+  if (lane == 0) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b0));
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], 1;" ::"r"(b1));
+    asm volatile("fence.mbarrier_init.release.cluster;");
+  }
+  __syncwarp();
+  auto issue = [&](int st, uint64_t it) {
+    const uint32_t bar = st ? b1 : b0;
+    if (lane == 0)
+      asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(bar),
+                   "r"(D * 128) : "memory");
+    __syncwarp();
+    for (int k = lane; k < D; k += 32) {
+      const uint64_t b = ((mix(gw * 2654435761ULL + it * D + k) & 0xFFFFFFFFull) * nblocks) >> 32;
+      const uint32_t dst = smem_u32(ring + ((size_t)st * D + k) * 8);
+      asm volatile(
+          "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], 128, [%2];"
+          ::"r"(dst), "l"(buf + b * 8), "r"(bar) : "memory");
+    }
+  };
+  auto wait = [&](int st, uint32_t parity) {
+    const uint32_t bar = st ? b1 : b0;
+    asm volatile(
+        "{\n .reg .pred p;\n WAIT_%=:\n"
+        " mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+        " @!p bra WAIT_%=;\n}" ::"r"(bar), "r"(parity) : "memory");
+  };
+  uint32_t acc = 0;
+  issue(0, 0);
+  issue(1, 1);
+  for (uint64_t it = 0; it < iters; ++it) {
+    const int st = (int)(it & 1);
+    wait(st, (uint32_t)((it >> 1) & 1));
+    for (int k = lane; k < D; k += 32) {
+      const uint4 x = ring[((size_t)st * D + k) * 8 + (it & 7)];
+      acc += x.x ^ x.w;
+    }
+    __syncwarp();
+    if (it + 2 < iters + 2) issue(st, it + 2);
+  }
+  wait(0, (uint32_t)(((iters) >> 1) & 1));
+  wait(1, (uint32_t)(((iters + 1) >> 1) & 1));
+  if (acc == 0x12345678u) atomicAdd(sink, 1ull);
+}
+
+// G ops/s of the bulk-copy gather: D buckets per stage, `warps` warps per block
+template <int D>
+double run_bulk(const uint4* buf, uint64_t bytes, int sms, int bps, int warps) {
+  const uint64_t nblocks = bytes / 128;
+  const int threads = 32 * warps;
+  const size_t smem = (size_t)warps * 2 * D * 128;
+  if (cudaFuncSetAttribute(gather_bulk<D>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                           (int)smem) != cudaSuccess)
+    return 0.0;
+  unsigned long long* sink;
+  cudaMalloc(&sink, 8);
+  const uint64_t iters = 64;
+  gather_bulk<D><<<sms * bps, threads, smem>>>(buf, nblocks, 4, sink);
+  cudaEvent_t a, b;
+  cudaEventCreate(&a);
+  cudaEventCreate(&b);
+  cudaEventRecord(a);
+  gather_bulk<D><<<sms * bps, threads, smem>>>(buf, nblocks, iters, sink);
+  const cudaError_t le = cudaGetLastError();  // e.g. more shared memory than an SM has
+  cudaEventRecord(b);
+  if (le != cudaSuccess || cudaEventSynchronize(b) != cudaSuccess) {
+    cudaGetLastError();
+    cudaFree(sink);
+    return 0.0;
+  }
+  float ms = 0;
+  cudaEventElapsedTime(&ms, a, b);
+  cudaFree(sink);
+  // every iteration consumes one stage of D buckets (the two issued past the end are
+  // waited for but not counted)
+  return (double)sms * bps * warps * iters * D / (ms * 1e-3) / 1e9;
+}
+
 template <int G, int U, int M = 0>
 double run(uint4* buf, uint64_t bytes, int sms, uint32_t* cnt = nullptr, uint32_t ncnt = 1,
            double* gops = nullptr, int bps = 8) {
@@ -111,7 +209,22 @@ int main() {
 #undef DG_TRY
   }
   printf("\"G_ops_s_S128\": {\"read\": %.2f, \"read_store8\": %.2f, \"read_cas8\": %.2f, "
-         "\"read_cas8_counter\": %.2f}}\n", best[0], best[1], best[2], best[3]);
+         "\"read_cas8_counter\": %.2f}, ", best[0], best[1], best[2], best[3]);
+  // cp.async.bulk + mbarrier gather (128-B buckets into shared memory): best over
+  // buckets per stage D, warps per block and blocks per SM
+  double bb = 0;
+  char cfgs[64] = "";
+  for (int bps : {1, 2, 4}) {
+    for (int warps : {4, 8}) {
+      double g;
+#define DG_TRYB(D_)                                                                    \
+      g = run_bulk<D_>(buf, bytes, sm, bps, warps);                                    \
+      if (g > bb) { bb = g; snprintf(cfgs, sizeof cfgs, "D%d_w%d_b%d", D_, warps, bps); }
+      DG_TRYB(8) DG_TRYB(16) DG_TRYB(32) DG_TRYB(64)
+#undef DG_TRYB
+    }
+  }
+  printf("\"G_ops_s_S128_bulk\": {\"read\": %.2f, \"best\": \"%s\"}}\n", bb, cfgs);
   cudaFree(cnt);
   cudaFree(buf);
   return 0;
