@@ -62,9 +62,10 @@ cudaError_t ensure_buf(dg_graph_s::Buf& b, size_t bytes) {
 
 // Input buffer: device pointers pass through; host memory is copied to a staging
 // buffer (the call then becomes synchronous).
+// (is_dev: the caller already knows p is device memory; -1 = ask the runtime)
 dg_status stage_in(dg_graph g, int slot, const void* p, size_t bytes, cudaStream_t s,
-                   const void** out, bool* host) {
-  if (!p || bytes == 0 || is_device_ptr(p)) {
+                   const void** out, bool* host, int is_dev = -1) {
+  if (!p || bytes == 0 || (is_dev >= 0 ? is_dev != 0 : is_device_ptr(p))) {
     *out = p;
     return DG_OK;
   }
@@ -275,19 +276,47 @@ namespace {
 // failed ops after the launch and re-run them after growing the pool).
 // (every size class must be able to absorb the worst case: all ops of the launch
 // may extend chains of one class)
+// The host's bound on the bump cursors, tightened from what the insert fixup kernels
+// published to mapped memory (no copy, no event): launches up to the published epoch
+// are done, so bump <= published bump + the worst case of the launches after it.
+void refresh_bound(dg_graph g) {
+  if (g->pending_need.empty()) return;
+  volatile const u32* h = g->h_hot;
+  const u32 pe = h[5];
+  if (pe == 0 || pe < g->pub_floor) return;  // nothing newer than the last exact read
+  bool dropped = false;
+  while (!g->pending_need.empty() && g->pending_need.front().first <= pe) {
+    g->pending_need.pop_front();
+    dropped = true;
+  }
+  if (!dropped) return;
+  u64 rest = 0;
+  for (const auto& p : g->pending_need) rest += p.second;
+  for (int c = 0; c < g->ncls; ++c)
+    g->bump_ub[c] = std::min<u64>(g->bump_ub[c], (u64)h[2 + c] + rest);
+}
+
+// after an exact read of the cursors (read_ctl): nothing older is pending
+void bound_exact(dg_graph g) {
+  for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = g->hctl->bump[c];
+  g->pending_need.clear();
+  g->pub_floor = g->epoch;
+}
+
 dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) {
   *retry_mode = false;
-  if (g->snap_pending && cudaEventQuery(g->snap_event) == cudaSuccess) {
-    g->snap_pending = false;
-    for (int c = 0; c < g->ncls; ++c)  // exact as of the snapshot; nothing launched since
-      g->bump_ub[c] = g->hctl->bump[c];
-  }
+  refresh_bound(g);
   bool ok = true;
   for (int c = 0; c < g->ncls; ++c) ok = ok && (u64)g->cap[c] >= g->bump_ub[c] + need;
   if (ok) return DG_OK;
+  static const bool trace = std::getenv("DG_TRACE_PLAN") != nullptr;
+  if (trace)
+    std::fprintf(stderr, "dg: plan sync epoch %u need %llu cap %u bump_ub %llu pending %zu pub %u floor %u\n",
+                 g->epoch, (unsigned long long)need, g->cap[0], (unsigned long long)g->bump_ub[0],
+                 g->pending_need.size(), reinterpret_cast<volatile u32*>(g->h_hot)[5], g->pub_floor);
   // exact free counts
   DG_TRY(read_ctl(g, s));
-  g->snap_pending = false;
+  bound_exact(g);
   static const bool no_upfront = std::getenv("DG_TEST_RETRY_PATH") != nullptr;
   // Reserve the worst case (one new bucket per op) up front when it is bounded
   // (<= 4 GB and half of free device memory): steady-state batches then never
@@ -295,17 +324,28 @@ dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) 
   // actually failed.
   u64 limit = 0;  // cudaMemGetInfo is slow: query it only when a pool must grow
   for (int c = 0; c < g->ncls; ++c) {
-    g->bump_ub[c] = g->hctl->bump[c];
     const u64 free_exact = (u64)g->cap[c] - g->hctl->bump[c] + g->hctl->stack_size[c];
-    // pops come from the stack first; the bump cursor moves by at most need - stack
-    if (free_exact >= need) continue;
+    // pops come from the stack first; the bump cursor moves by at most need - stack.
+    // Beyond the batch's own worst case, keep headroom for several more batches of this
+    // size, so that back-to-back calls do not come back here (a synchronisation)
+    // before the cursors published by earlier launches catch up (refresh_bound).
+    if (!limit) limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
+    const u64 room = std::max<u64>(
+        std::min<u64>(8 * need, std::min<u64>(limit, 2ull << 30) / g->cbytes(c)), 65536);
+    if (free_exact >= need + room) continue;
+    if (free_exact >= need) {  // enough for this batch: top up the headroom if cheap
+      if (!no_upfront) {
+        dg_status st = grow_pool(g, c, (u64)g->cap[c] + need + room - free_exact, s);
+        if (st != DG_OK && st != DG_ERR_OUT_OF_MEMORY) return st;
+      }
+      continue;
+    }
     const u64 missing = need - free_exact;
     // (adaptive layout: the worst case is reserved in every class pool — mapped
     // capacity, not table bytes; retry mode instead made every batch synchronise and
     // grow inside the step: cfg3 insert 2.4 -> 18 ms per 2^24)
-    if (!limit) limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
     if (!no_upfront && missing * g->cbytes(c) <= limit) {
-      const u64 want = (u64)g->cap[c] + missing + std::max<u64>(missing / 4, 65536);
+      const u64 want = (u64)g->cap[c] + missing + std::max<u64>(missing / 4, room);
       dg_status st = grow_pool(g, c, want, s);
       if (st == DG_OK) continue;
       if (st != DG_ERR_OUT_OF_MEMORY) return st;
@@ -315,21 +355,9 @@ dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) 
   return DG_OK;
 }
 
-void note_launch(dg_graph g, u64 need, cudaStream_t s) {
-  bool tight = false;
-  for (int c = 0; c < g->ncls; ++c) {
-    g->bump_ub[c] = std::min<u64>(g->cap[c], g->bump_ub[c] + need);
-    tight = tight || (u64)g->cap[c] < g->bump_ub[c] + need;
-  }
-  // snapshot the allocator cursors asynchronously when the bound gets tight
-  if (tight && !g->snap_pending) {
-    if (cudaMemcpyAsync(g->hctl, g->ctl, sizeof(dg::DevCtl), cudaMemcpyDeviceToHost, s) ==
-            cudaSuccess &&
-        cudaEventRecord(g->snap_event, s) == cudaSuccess)
-      g->snap_pending = true;
-    else
-      cudaGetLastError();
-  }
+void note_launch(dg_graph g, u64 need, u32 epoch) {
+  for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::min<u64>(g->cap[c], g->bump_ub[c] + need);
+  g->pending_need.emplace_back(epoch, need);
 }
 
 }  // namespace
@@ -344,9 +372,8 @@ u64 retry_cap_max() {
 
 dg_status prepare_insert(dg_graph g, u64 n_ops, cudaStream_t s) {
   if (n_ops == 0) return DG_OK;
-  if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));
   bool retry_mode = false;
-  DG_TRY(plan_capacity(g, n_ops + dg::max_groups(g->G, g->sms), s, &retry_mode));
+  DG_TRY(plan_capacity(g, n_ops + dg::spare_bound(n_ops, g->ncls, g->G, g->sms), s, &retry_mode));
   if (retry_mode) DG_TRY(ensure_retry(g, 0, std::min<u64>(n_ops, retry_cap_max())));
   DG_TRY(ensure_ret(g, n_ops));
   return DG_OK;
@@ -358,12 +385,8 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   dg::Tables t = g->tables();
   const u64 n_ops = mirror ? 2 * n : n;
   if (n_ops == 0) return DG_OK;
-  const u64 need = n_ops + dg::max_groups(g->G, g->sms);
+  const u64 need = n_ops + dg::spare_bound(n_ops, g->ncls, g->G, g->sms);
   bool retry_mode = false;
-  // the snapshot must not be in flight while read_ctl rewrites hctl
-  if (g->snap_pending) {
-    DG_CK(cudaEventSynchronize(g->snap_event));
-  }
   DG_TRY(plan_capacity(g, need, s, &retry_mode));
   // Retry mode records the ops that found no bucket, up to a bounded list (128 MB);
   // when more fail, the whole batch runs again after the pool grows (an insert batch
@@ -391,8 +414,12 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   // (large batches only: a small batch would pay a second launch for little)
   a.sorted_path = (!no_sorted && !mirror && epoch == g->validated_epoch && n >= (1u << 18)) ? 1u : 0u;
   static const u32 excl_chains = std::getenv("DG_EXCL_CHAINS")
-                                     ? (u32)std::atoi(std::getenv("DG_EXCL_CHAINS")) : 64u;
+                                     ? (u32)std::atoi(std::getenv("DG_EXCL_CHAINS")) : 256u;
   a.excl_chains = excl_chains;
+  // small batches: the insert kernel's last block does the allocator fixup (one launch
+  // instead of two; a large batch returns more spare buckets than one block copies fast)
+  const bool fused = !g->adaptive && !retry_mode && !a.sorted_path && n_ops <= (1u << 18);
+  a.pub = fused ? g->d_hot : nullptr;
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
@@ -404,17 +431,17 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
                  (unsigned long long)n_ops, g->hctl->pop_count[0], g->hctl->stack_size[0], b0,
                  g->hctl->bump[0], g->hctl->ret_count);
   }
-  // (the fixup kernel also publishes the chain-length metric for the next batch)
-  DG_CK(dg::launch_fixup_alloc(t, (g->hot_steps && !g->in_rehash) ? g->d_hot : nullptr, s));
+  // (the fixup also publishes the chain-length metric and the cursors)
+  if (!fused) DG_CK(dg::launch_fixup_alloc(t, g->d_hot, epoch, s));
   if (!retry_mode) {
-    note_launch(g, need, s);
+    note_launch(g, need, epoch);
     return DG_OK;
   }
   // retry mode: re-run the ops that found no free bucket after growing the pool
   int cur = 0;
   for (int round = 0;; ++round) {
     DG_TRY(read_ctl(g, s));
-    for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = g->hctl->bump[c];
+    bound_exact(g);
     const u64 failed = g->hctl->retry_count;
     if (failed == 0) break;
     if (round > 64) return DG_ERR_OUT_OF_MEMORY;
@@ -434,10 +461,11 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
     a.idx = whole ? nullptr : g->retry[cur];
     a.n_ops = whole ? n_ops : failed;
     a.sorted_path = 0;  // re-runs go through k_edges
+    a.pub = nullptr;
     a.retry_out = g->retry[cur ^ 1];
     a.retry_cap = next_cap;
     DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
-    DG_CK(dg::launch_fixup_alloc(t, nullptr, s));
+    DG_CK(dg::launch_fixup_alloc(t, g->d_hot, epoch, s));
     cur ^= 1;
   }
   return DG_OK;
@@ -562,6 +590,8 @@ dg_status rehash_rows(dg_graph g, u32 n, bool flush, cudaStream_t s) {
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   DG_CK(cudaMemsetAsync(&g->ctl->retry_count, 0, 4, s));
   for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::max<u64>(g->bump_ub[c], newbump[c]);
+  g->pending_need.clear();  // (synchronised above: every earlier launch is done)
+  g->pub_floor = g->epoch + 1;
   // the pairs go back through the ordinary insert kernel (all keys distinct)
   DG_TRY(local_insert(g, osrc, odst, ow, total_deg, false, ++g->epoch, s));
   DG_CK(cudaStreamSynchronize(s));
@@ -732,6 +762,8 @@ static dg_status add_rows(dg_graph g, u64 row0, u64 count, const u32* hints_glob
   DG_CK(cudaFreeAsync(off, s));
   DG_CK(cudaStreamSynchronize(s));
   for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = std::max<u64>(g->bump_ub[c], newbump[c]);
+  g->pending_need.clear();  // (synchronised: every earlier launch is done)
+  g->pub_floor = g->epoch + 1;
   return DG_OK;
 }
 
@@ -871,6 +903,8 @@ dg_status dg_num_vertices(dg_graph g, uint64_t* num_vertices, uint64_t* local_ro
 static dg_status check_handle(dg_graph g) {
   if (!g) return DG_ERR_INVALID_ARGUMENT;
   if (g->bad) return DG_ERR_BAD_STATE;
+  int cur = -1;
+  if (cudaGetDevice(&cur) == cudaSuccess && cur == g->device) return DG_OK;
   if (cudaSetDevice(g->device) != cudaSuccess) {
     g->bad = true;
     return DG_ERR_CUDA;
@@ -902,8 +936,9 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   const u32 epoch = ++g->epoch;
   bool host = false;
   const void *ds = nullptr, *dd = nullptr, *dw = nullptr;
-  if (!g->router && !n_added && n && !is_device_ptr(src) && !is_device_ptr(dst) &&
-      (!weight || !is_device_ptr(weight))) {
+  const bool dev_src = is_device_ptr(src), dev_dst = is_device_ptr(dst);
+  const bool dev_w = weight && is_device_ptr(weight);
+  if (!g->router && !n_added && n && !dev_src && !dev_dst && (!weight || !dev_w)) {
     // host inputs, no count requested: return once the batch is uploaded and
     // validated; the insert kernel runs behind the caller's next upload
     DG_TRY(upload_async(g, 8, src, n * 4, s, &ds));
@@ -917,9 +952,9 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     DG_TRY(release_slots(g, 8, 11, s));
     return validation_status(g, epoch);
   }
-  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
-  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
-  DG_TRY(stage_in(g, 2, weight, weight ? n * 4 : 0, s, &dw, &host));
+  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host, dev_src));
+  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host, dev_dst));
+  DG_TRY(stage_in(g, 2, weight, weight ? n * 4 : 0, s, &dw, &host, dev_w));
   if (g->router) {
     DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
   } else {
@@ -934,7 +969,7 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     if (g->router) DG_TRY(dg::router_sum_u64(g, &cnt, s));
     if (n_added) *n_added = cnt;
     g->snap_pending = false;
-    for (int c = 0; c < g->ncls; ++c) g->bump_ub[c] = g->hctl->bump[c];
+    dg::bound_exact(g);
     return status_of(g, epoch);
   }
   return DG_OK;
@@ -950,7 +985,8 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
   const u32 epoch = ++g->epoch;
   bool host = false;
   const void *ds = nullptr, *dd = nullptr;
-  if (!g->router && !n_removed && n && !is_device_ptr(src) && !is_device_ptr(dst)) {
+  const bool dev_src = is_device_ptr(src), dev_dst = is_device_ptr(dst);
+  if (!g->router && !n_removed && n && !dev_src && !dev_dst) {
     // host inputs, no count requested: as in dg_insert_edges
     DG_TRY(upload_async(g, 11, src, n * 4, s, &ds));
     DG_TRY(upload_async(g, 12, dst, n * 4, s, &dd));
@@ -960,8 +996,8 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
     DG_TRY(release_slots(g, 11, 13, s));
     return validation_status(g, epoch);
   }
-  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host));
-  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host));
+  DG_TRY(stage_in(g, 0, src, n * 4, s, &ds, &host, dev_src));
+  DG_TRY(stage_in(g, 1, dst, n * 4, s, &dd, &host, dev_dst));
   if (g->router) {
     DG_TRY(dg::router_delete(g, (const u32*)ds, (const u32*)dd, n, epoch, s));
   } else {

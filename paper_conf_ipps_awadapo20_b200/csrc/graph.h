@@ -2,6 +2,8 @@
 #pragma once
 #include <cstddef>
 #include <cstdint>
+#include <deque>
+#include <utility>
 #include <vector>
 
 #include <cuda_runtime.h>
@@ -40,6 +42,10 @@ struct dg_graph_s {
   dg::VmmArray pool[dg::kClasses], stack[dg::kClasses];  // per size class
   uint32_t cap[dg::kClasses] = {0, 0, 0};      // buckets mapped in each pool
   uint64_t bump_ub[dg::kClasses] = {0, 0, 0};  // host upper bounds of the device bump cursors
+  // insert launches whose cursors the fixup kernel has not published yet: (epoch,
+  // worst-case buckets); the bound is published bump + their sum (api.cu refresh_bound)
+  std::deque<std::pair<uint32_t, uint64_t>> pending_need;
+  uint32_t pub_floor = 0;  // publications older than this epoch predate an exact read
   // bytes of one bucket of class c
   uint32_t cbytes(int c) const { return adaptive ? (32u << c) : bucket_bytes; }
 
@@ -83,8 +89,9 @@ struct dg_graph_s {
   uint32_t* hot_list = nullptr;
   uint32_t hot_cap = 65536;
   uint32_t hot_steps = 4;      // 0 = off
-  // mapped pinned {hot_count, hot_pairs}, written by the insert's fixup kernel (read
-  // by the host without a copy; may lag one batch behind, which only delays re-sizing)
+  // mapped pinned {hot_count, hot_pairs, bump[3], epoch}, written by the insert's fixup
+  // kernel (read by the host without a copy; it may lag behind the stream, which only
+  // delays re-sizing and keeps the cursor bound conservative)
   uint32_t* h_hot = nullptr;
   uint32_t* d_hot = nullptr;   // its device alias
   bool in_rehash = false;

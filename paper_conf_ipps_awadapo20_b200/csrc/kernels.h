@@ -35,6 +35,9 @@ struct EdgeBatch {
   u32 sorted_path;       // insert: k_validate checked this epoch's sources for sortedness;
                          // a src-sorted batch runs k_insert_sorted (a3), others k_edges
   u32 excl_chains;       // k_insert_sorted: rows with at most this many chains are owned
+  u32* pub;              // insert, uniform layouts: when set, the last block of k_edges
+                         // does the allocator fixup and publishes to pub (small batches:
+                         // one launch instead of two)
 };
 
 // `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1
@@ -47,9 +50,11 @@ cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms,
 cudaError_t launch_delete(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
 cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);
 // after an insert launch: free stack / cursors; hot_out (mapped host, nullable)
-// receives {hot_count, hot_pairs}
-cudaError_t launch_fixup_alloc(const Tables& t, u32* hot_out, cudaStream_t s);
+// receives {hot_count, hot_pairs, bump[3], epoch} (kernels_edges.cu publish())
+cudaError_t launch_fixup_alloc(const Tables& t, u32* hot_out, u32 epoch, cudaStream_t s);
 u64 max_groups(int G, int sms);
+// buckets an insert launch of n_ops ops may take beyond those it links
+u64 spare_bound(u64 n_ops, int ncls, int G, int sms);
 
 // graph structure (kernels_graph.cu)
 // nb[r] for rows r in [0, count): initial bucket count from a hint,

@@ -516,15 +516,23 @@ template <int OP>
 struct MinBlocks {
   static constexpr int v = OP == OP_INSERT ? DG_MINB_INS : OP == OP_QUERY ? DG_MINB_QRY : DG_MINB_DEL;
 };
+// the allocator fixup of k_fixup by ONE block (the last of k_edges, small batches)
+__device__ __forceinline__ void fixup_block(const Tables& t, u32* pub, u32 epoch);
+
 template <int G, int S, int OP, bool A>
 __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<Lanes<G, OP>::L> g;
+  bool skip = false;
   if (OP != OP_QUERY) {
-    if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) return;  // batch rejected (Q7)
+    if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) skip = true;  // batch rejected (Q7)
   }
   if (OP == OP_INSERT && a.sorted_path && ld_relaxed_u32(&t.ctl->unsorted_epoch) != a.epoch)
-    return;  // src-sorted batch: k_insert_sorted installs it
+    skip = true;  // src-sorted batch: k_insert_sorted installs it
+  if (skip) {
+    if (OP == OP_INSERT && !A && a.pub) fixup_block(t, a.pub, a.epoch);  // (every block: a no-op
+    return;                                                            //  but for the last)
+  }
   const bool reuse = a.reuse_tombstones != 0;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
@@ -587,6 +595,7 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
     if (g.lane == 0 && tot)
       atomicAdd(reinterpret_cast<unsigned long long*>(&t.ctl->count), (unsigned long long)tot);
   }
+  if (OP == OP_INSERT && !A && a.pub) fixup_block(t, a.pub, a.epoch);
 }
 
 // ------------------------------------------------- src-sorted batches (a3) ----
@@ -606,7 +615,7 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
 // (run_ops) in every chunk, as in unsorted batches.
 //
 #ifndef DG_SORTED_MINB
-#define DG_SORTED_MINB 2
+#define DG_SORTED_MINB 3
 #endif
 
 // position of the n-th (0-based) set bit of m
@@ -908,6 +917,16 @@ cudaError_t launch_query(int lay, const Tables& t, const EdgeBatch& a, int sms, 
   return launch_op<OP_QUERY>(lay, t, a, sms, s);
 }
 
+u64 spare_bound(u64 n_ops, int ncls, int G, int sms) {
+  // a launch of n_ops ops takes at most one bucket per extending op (linked or kept
+  // as its lane's spare) plus, per warp and size class, the unused rest of its last
+  // chunk (< one bucket per op of the warp): small batches need far less than the
+  // machine-wide bound
+  const u64 small = n_ops * (1 + (u64)ncls) + 4096;
+  const u64 big = max_groups(G, sms);
+  return small < big ? small : big;
+}
+
 u64 max_groups(int G, int sms) {
   // upper bound on the buckets an insert launch takes beyond the ones it links: each
   // resident thread may hold one spare bucket, each resident warp the unused rest of
@@ -925,12 +944,54 @@ cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 e
   return cudaGetLastError();
 }
 
+// What the host reads from mapped memory after an insert (no copy, no event; it may
+// lag behind the stream): the re-sizing counters and, tagged with the batch's epoch,
+// the allocator cursors (the host bounds the cursors of launches not yet published).
+// Layout (u32): [0] hot_count, [1] hot_pairs, [2..4] bump per class, [5] epoch
+// (written last, after a fence, so a host that sees the epoch sees the cursors).
+__device__ __forceinline__ void publish(const DevCtl* c, u32* out, u32 epoch) {
+  volatile u32* o = out;
+  o[0] = c->hot_count;
+  o[1] = c->hot_pairs;
+  for (int k = 0; k < kClasses; ++k) o[2 + k] = c->bump[k];
+  __threadfence_system();
+  o[5] = epoch;
+}
+
+// Every block of the launch calls this at its end; the last one to arrive (a fenced
+// counter) pushes the returned spare buckets onto the free stack, moves the cursors
+// and publishes them (uniform layouts; the launcher uses it for small batches, where
+// one block copies the few returned buckets quickly).
+__device__ __forceinline__ void fixup_block(const Tables& t, u32* pub, u32 epoch) {
+  __shared__ bool last;
+  __threadfence();
+  __syncthreads();
+  if (threadIdx.x == 0) last = atomicAdd(&t.ctl->fixup_done, 1u) == gridDim.x - 1;
+  __syncthreads();
+  if (!last) return;
+  __threadfence();
+  DevCtl* c = t.ctl;
+  const u32 pc = ld_relaxed_u32(&c->pop_count[0]), ss = ld_relaxed_u32(&c->stack_size[0]);
+  const u32 rc = ld_relaxed_u32(&c->ret_count);
+  const u32 base = pc >= ss ? 0u : ss - pc;
+  for (u32 k = threadIdx.x; k < rc; k += blockDim.x) t.stack[0][base + k] = t.ret_list[k];
+  __syncthreads();
+  if (threadIdx.x != 0) return;
+  __threadfence();
+  c->stack_size[0] = base + rc;
+  c->pop_count[0] = 0;
+  c->ret_count = 0;
+  if (c->bump[0] > t.cap[0]) c->bump[0] = t.cap[0];
+  publish(c, pub, epoch);
+  c->fixup_done = 0;
+}
+
 // Uniform layouts, ONE launch: every block copies its share of the returned spare
 // buckets onto the free stack (k_fixup_copy's work); the last block to finish (a
 // fenced counter) moves the cursors (k_fixup_alloc's work) and publishes the
 // re-sizing counters to `hot_out` (mapped host memory, nullable), so the host reads
 // them without a copy or an event per insert batch.
-__global__ void k_fixup(Tables t, u32* hot_out) {
+__global__ void k_fixup(Tables t, u32* hot_out, u32 epoch) {
   DevCtl* c = t.ctl;
   const u32 pc = c->pop_count[0], ss = c->stack_size[0], rc = c->ret_count;
   const u32 base = pc >= ss ? 0u : ss - pc;
@@ -948,28 +1009,24 @@ __global__ void k_fixup(Tables t, u32* hot_out) {
   c->pop_count[0] = 0;
   c->ret_count = 0;
   if (c->bump[0] > t.cap[0]) c->bump[0] = t.cap[0];
-  if (hot_out) {
-    hot_out[0] = c->hot_count;
-    hot_out[1] = c->hot_pairs;
-  }
+  if (hot_out) publish(c, hot_out, epoch);
   c->fixup_done = 0;
 }
 
-__global__ void k_hot_publish(const DevCtl* c, u32* hot_out) {
-  hot_out[0] = c->hot_count;
-  hot_out[1] = c->hot_pairs;
+__global__ void k_hot_publish(const DevCtl* c, u32* hot_out, u32 epoch) {
+  publish(c, hot_out, epoch);
 }
 
-cudaError_t launch_fixup_alloc(const Tables& t, u32* hot_out, cudaStream_t s) {
+cudaError_t launch_fixup_alloc(const Tables& t, u32* hot_out, u32 epoch, cudaStream_t s) {
   const bool uniform = t.cap[1] == 0;
   if (uniform) {
-    k_fixup<<<148, 256, 0, s>>>(t, hot_out);
+    k_fixup<<<148, 256, 0, s>>>(t, hot_out, epoch);
     note_kernel(1);
     return cudaGetLastError();
   }
   k_fixup_alloc<<<1, 256, 0, s>>>(t, false); note_kernel(1);
   if (hot_out) {
-    k_hot_publish<<<1, 1, 0, s>>>(t.ctl, hot_out);
+    k_hot_publish<<<1, 1, 0, s>>>(t.ctl, hot_out, epoch);
     note_kernel(1);
   }
   return cudaGetLastError();

@@ -23,14 +23,13 @@ def _ptr(a, n_expected=None, dtype_bytes=4, what="array"):
     """-> (pointer int, length, is_cuda)"""
     if a is None:
         return None, 0, False
-    if isinstance(a, torch.Tensor):
+    if type(a) is torch.Tensor or isinstance(a, torch.Tensor):
         if a.element_size() != dtype_bytes:
             raise TypeError(f"{what}: expected {dtype_bytes}-byte elements, got {a.dtype}")
         if not a.is_contiguous():
             raise ValueError(f"{what}: tensor must be contiguous")
         n = a.numel()
-        p = a.data_ptr() if n else None
-        return p, n, a.is_cuda
+        return (a.data_ptr() if n else None), n, a.is_cuda
     arr = np.asarray(a)
     if arr.dtype.itemsize != dtype_bytes or not arr.flags.c_contiguous:
         raise TypeError(f"{what}: expected a contiguous {dtype_bytes}-byte numpy array")
@@ -42,19 +41,30 @@ def _as_u32(a):
     """torch tensors pass through (int32/uint32); anything else becomes contiguous uint32 numpy."""
     if a is None:
         return None
-    if isinstance(a, torch.Tensor):
+    if type(a) is torch.Tensor or isinstance(a, torch.Tensor):
         if a.dtype not in _U32_OK:
             raise TypeError(f"expected int32/uint32 tensor, got {a.dtype}")
-        return a.contiguous()
+        return a if a.is_contiguous() else a.contiguous()
     return np.ascontiguousarray(np.asarray(a).astype(np.uint32, copy=False))
 
 
+_HAS_CUDA = None
+_raw_stream = getattr(torch._C, "_cuda_getCurrentRawStream", None)
+_cur_dev = getattr(torch._C, "_cuda_getDevice", None) or torch.cuda.current_device
+
+
 def _stream(stream):
+    """cudaStream_t handle of `stream`, else of torch's current stream (legacy 0 without CUDA)."""
+    global _HAS_CUDA
     if stream is not None:
         return stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
-    if torch.cuda.is_available():
-        return torch.cuda.current_stream().cuda_stream
-    return 0
+    if _HAS_CUDA is None:
+        _HAS_CUDA = torch.cuda.is_available()
+    if not _HAS_CUDA:
+        return 0
+    if _raw_stream is not None:  # (the current stream without building a Stream object)
+        return _raw_stream(_cur_dev())
+    return torch.cuda.current_stream().cuda_stream
 
 
 class Graph:
