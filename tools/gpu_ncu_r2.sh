@@ -12,3 +12,5 @@ timeout 900 ncu --set full --clock-control none -k regex:"k_tc_wedges" -c 1 \
 for f in cfg2 cfg3 cfg5; do python tools/ncu_summary.py $D/$f.ncu-rep > $D/summary_$f.txt 2>&1; done
 python tools/launch_share.py $D/launches_bench_cfg2.csv > $D/launches_summary.txt 2>&1
 ls -la $D
+timeout 1500 python bench.py --config cfg5 > $D/bench_cfg5.json 2> $D/bench_cfg5.err; echo cfg5 rc=$?
+python -c "import json; d=json.loads(open('$D/bench_cfg5.json').read().strip().splitlines()[-1]); print('cfg5', d['value'], d['tc']['insert_ms_per_step'], d['tc']['tc_ms_per_step'], d['clocks'])"
