@@ -504,8 +504,8 @@ struct Prefetch {
 // 2^24 batches: insert 1.41 -> 1.35 ms and query 0.625 -> 0.603 ms at 3 blocks of
 // 256 threads, 85 registers, no spills; delete is faster at 4: 1.07 vs 1.12 ms)
 #ifndef DG_MINB_INS
-#define DG_MINB_INS 3
-#endif
+#define DG_MINB_INS 4  // round 2 (home buckets): 4 blocks with a 148-B spill beat 3 blocks
+#endif                 // at 80 registers, cfg2 insert 1.242 -> 1.206 ms (profiles/r02/ab)
 #ifndef DG_MINB_QRY
 #define DG_MINB_QRY 3
 #endif
