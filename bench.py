@@ -33,12 +33,15 @@ import os
 import statistics
 import subprocess
 import sys
+import threading
 import time
 
 import numpy as np
 
 ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
+if __name__ == "__main__":  # bench_stream imports `bench`: the same module, not a copy
+    sys.modules.setdefault("bench", sys.modules[__name__])
 
 import workloads as wl  # noqa: E402
 
@@ -66,11 +69,119 @@ def in_sample(u):
 
 
 # ----------------------------------------------------------------- helpers --
+_RANK = threading.local()  # --inproc: (world, rank, local) of this rank thread
+
+
 def dist_env():
+    if getattr(_RANK, "env", None):
+        return _RANK.env
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     return world, rank, local
+
+
+class DistColl:
+    """The bench's own collectives over torch.distributed (one process per GPU, the
+    layout the driver launches); the library's rank communicator is NCCL."""
+
+    def __init__(self, dev, rank):
+        import torch.distributed as dist
+        from paper_conf_ipps_awadapo20_b200 import get_unique_id
+        dist.init_process_group("nccl", device_id=dev)
+        self.dist = dist
+        obj = [get_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(obj, src=0)
+        self.uid = obj[0]
+
+    def graph_kwargs(self):
+        return {"nccl_unique_id": self.uid}
+
+    def barrier(self):
+        self.dist.barrier()
+
+    def all_reduce(self, t, op="sum"):
+        self.dist.all_reduce(t, op=self.dist.ReduceOp.MAX if op == "max" else self.dist.ReduceOp.SUM)
+
+    def close(self):
+        self.dist.barrier()
+        self.dist.destroy_process_group()
+
+
+class ThreadColl:
+    """Dry run of the N > 1 path without N GPUs (`--inproc N`): the ranks are threads
+    of this process over an in-process rank group (`RankGroup`), spread round-robin
+    over the visible GPUs; the bench's collectives meet at a thread barrier.  It
+    exercises the sharded bench and library code paths (slices, routing, answers,
+    max-over-ranks timing); its rates are not a scaling measurement."""
+
+    def __init__(self, shared, rank):
+        self.s, self.rank = shared, rank
+
+    def graph_kwargs(self):
+        return {"group": self.s["group"]}
+
+    def barrier(self):
+        self.s["barrier"].wait()
+
+    def all_reduce(self, t, op="sum"):
+        import torch
+        slots = self.s["slots"]
+        slots[self.rank] = t.detach().cpu().clone()
+        self.barrier()
+        acc = slots[0].clone()
+        for x in slots[1:]:
+            acc = torch.maximum(acc, x) if op == "max" else acc + x
+        self.barrier()
+        t.copy_(acc.to(t.device))
+
+    def close(self):
+        self.barrier()
+
+
+def parallelism_label(world, what="source-vertex sharding"):
+    lab = f"{what} x{world}" if world > 1 else "single GPU"
+    if getattr(_RANK, "shared", None):
+        lab += " (in-process rank group dry run: --inproc)"
+    return lab
+
+
+def make_coll(world, rank, dev):
+    if world == 1:
+        return None
+    shared = getattr(_RANK, "shared", None)
+    return ThreadColl(shared, rank) if shared else DistColl(dev, rank)
+
+
+def run_inproc(args, fn):
+    """--inproc N: N rank threads, each with its own stream (dry run, see ThreadColl)."""
+    import torch
+    from paper_conf_ipps_awadapo20_b200 import RankGroup
+    n = args.inproc
+    ndev = max(1, torch.cuda.device_count())
+    shared = {"group": RankGroup(n), "barrier": threading.Barrier(n), "slots": [None] * n}
+    errors = []
+
+    def rank_main(r):
+        try:
+            _RANK.env = (n, r, r % ndev)
+            _RANK.shared = shared
+            torch.cuda.set_device(r % ndev)
+            with torch.cuda.stream(torch.cuda.Stream()):
+                fn(args, CONFIGS[args.config])
+        except BaseException as e:  # noqa: BLE001
+            errors.append((r, repr(e)))
+            shared["barrier"].abort()
+
+    th = [threading.Thread(target=rank_main, args=(r,)) for r in range(n)]
+    for t in th:
+        t.start()
+    for t in th:
+        t.join()
+    if errors:
+        print(json.dumps({"inproc_errors": errors}), file=sys.stderr)
+        return 1
+    return 0
 
 
 def slice_of(n, rank, world):
@@ -315,7 +426,7 @@ def config_block(cfg, args, nv, m, B, world):
             "bucket_bytes": args.bucket_bytes, "load_factor": args.load_factor,
             "variant": args.variant or "map",
             "l2": "flushed (256 MiB write) before every timed op; tables >> L2",
-            "parallelism": f"source-vertex sharding x{world}" if world > 1 else "single GPU"}
+            "parallelism": parallelism_label(world)}
 
 
 # -------------------------------------------------------------------- ours --
@@ -324,16 +435,9 @@ def run_ours(args, cfg):
     world, rank, local = dist_env()
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
-    from paper_conf_ipps_awadapo20_b200 import Graph, get_unique_id
-    pg = None
-    uid = None
-    if world > 1:
-        import torch.distributed as dist
-        dist.init_process_group("nccl", device_id=dev)
-        pg = dist
-        obj = [get_unique_id() if rank == 0 else None]
-        dist.broadcast_object_list(obj, src=0)
-        uid = obj[0]
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    pg = make_coll(world, rank, dev)
+    gkw = pg.graph_kwargs() if pg else {}
 
     B = 1 << args.batch_log2
     S = args.bucket_bytes
@@ -342,7 +446,7 @@ def run_ours(args, cfg):
     # global degree hints (connectivity information known in advance)
     hints_t = torch.bincount(torch.from_numpy(base_s.astype(np.int64)).to(dev), minlength=nv)
     if pg:
-        pg.all_reduce(hints_t)
+        pg.all_reduce(hints_t, "sum")
     hints = hints_t.to(torch.int32).contiguous()
     del hints_t
     gen_s = time.perf_counter() - t_gen
@@ -366,8 +470,7 @@ def run_ours(args, cfg):
     c0, c1, c2 = ev(), ev(), ev()
     c0.record()
     g = Graph(nv, hints, bucket_bytes=S, load_factor=args.load_factor, rank=rank, nranks=world,
-              set_variant=args.variant == "set",
-              nccl_unique_id=uid)
+              set_variant=args.variant == "set", **gkw)
     c1.record()
     bs = torch.from_numpy(base_s).to(dev)
     bd = torch.from_numpy(base_d).to(dev)
@@ -508,8 +611,8 @@ def run_ours(args, cfg):
     kms = torch.tensor([prof["kernel_ms"]["insert"], prof["kernel_ms"]["query"],
                         prof["kernel_ms"]["delete"]], dtype=torch.float64, device=dev)
     if pg:
-        pg.all_reduce(times, op=pg.ReduceOp.MAX)
-        pg.all_reduce(kms, op=pg.ReduceOp.MAX)
+        pg.all_reduce(times, "max")
+        pg.all_reduce(kms, "max")
     t_ins, t_q, t_del = times.tolist()
     total_ms = t_ins + t_q + t_del
     K = args.steps
@@ -612,7 +715,7 @@ def run_ours(args, cfg):
                     e2e_wall[k] = e2e_wall.get(k, 0.0) + 1e3 * dt
         t = torch.tensor([e2e_ms], dtype=torch.float64, device=dev)
         if pg:
-            pg.all_reduce(t, op=pg.ReduceOp.MAX)
+            pg.all_reduce(t, "max")
         e2e_ms = t.item()
         e2e = {"value": 3 * B * E * world / (e2e_ms * 1e3), "unit": UNIT,
                "h2d_bytes_per_step": B * (12 + 8 + 8), "d2h_bytes_per_step": B * 5 + 3 * 64,
@@ -684,8 +787,7 @@ def run_ours(args, cfg):
         print(json.dumps(line), flush=True)
     g.close()
     if pg:
-        pg.barrier()
-        pg.destroy_process_group()
+        pg.close()
     return 0
 
 
@@ -707,6 +809,9 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-sorted-build", action="store_true",
                     help="skip the second bulk build from src-sorted input")
+    ap.add_argument("--inproc", type=int, default=0,
+                    help="dry run of the N-rank path: N rank threads of this process over an "
+                         "in-process rank group on the visible GPUs (not a scaling measurement)")
     args = ap.parse_args()
     cfg = CONFIGS[args.config]
     if args.bucket_bytes is None:  # TC probes whole buckets: 64-B set buckets (14 keys) move half the bytes
@@ -715,11 +820,15 @@ def main():
         return run_reference(args, cfg)
     if cfg.get("stream"):
         import bench_stream
-        return bench_stream.run_mixed(args, cfg)
-    if cfg.get("tc"):
+        fn = bench_stream.run_mixed
+    elif cfg.get("tc"):
         import bench_stream
-        return bench_stream.run_tc(args, cfg)
-    return run_ours(args, cfg)
+        fn = bench_stream.run_tc
+    else:
+        fn = run_ours
+    if args.inproc > 1:
+        return run_inproc(args, fn)
+    return fn(args, cfg)
 
 
 if __name__ == "__main__":

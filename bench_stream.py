@@ -21,8 +21,8 @@ import time
 import numpy as np
 
 import workloads as wl
-from bench import (METRIC, UNIT, ClockSampler, config_block, dist_env, load_peaks, model_bytes,
-                   slice_of)
+from bench import (METRIC, UNIT, ClockSampler, config_block, dist_env, load_peaks, make_coll,
+                   model_bytes, parallelism_label, slice_of)
 
 
 def _setup(args):
@@ -30,12 +30,7 @@ def _setup(args):
     world, rank, local = dist_env()
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
-    pg = None
-    if world > 1:
-        import torch.distributed as dist
-        dist.init_process_group("nccl", device_id=dev)
-        pg = dist
-    return torch, world, rank, local, dev, pg
+    return torch, world, rank, local, dev, make_coll(world, rank, dev)
 
 
 def _clock(local):
@@ -46,26 +41,22 @@ def _clock(local):
 def _max(torch, pg, dev, vals):
     t = torch.tensor(vals, dtype=torch.float64, device=dev)
     if pg:
-        pg.all_reduce(t, op=pg.ReduceOp.MAX)
+        pg.all_reduce(t, "max")
     return t.tolist()
 
 
 def _sum(torch, pg, dev, vals):
     t = torch.tensor(vals, dtype=torch.float64, device=dev)
     if pg:
-        pg.all_reduce(t)
+        pg.all_reduce(t, "sum")
     return t.tolist()
 
 
 # ------------------------------------------------------------------ cfg4 ----
 def run_mixed(args, cfg):
     torch, world, rank, local, dev, pg = _setup(args)
-    from paper_conf_ipps_awadapo20_b200 import Graph, get_unique_id
-    uid = None
-    if pg:
-        obj = [get_unique_id() if rank == 0 else None]
-        pg.broadcast_object_list(obj, src=0)
-        uid = obj[0]
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    gkw = pg.graph_kwargs() if pg else {}
     nv, m, seed, scale, abc = cfg["nv"], cfg["m"], cfg["seed"], cfg["scale"], cfg["abc"]
     S = args.bucket_bytes
     t0 = time.perf_counter()
@@ -74,7 +65,7 @@ def run_mixed(args, cfg):
     bw = wl.weights(seed, 0, cnt, offset=off)
     deg = torch.bincount(torch.from_numpy(bs.astype(np.int64)).to(dev), minlength=nv)
     if pg:
-        pg.all_reduce(deg)
+        pg.all_reduce(deg, "sum")
     hints = deg.to(torch.int32).contiguous()
     top = torch.topk(deg, nv // 100).indices.to(torch.int64).cpu().numpy().astype(np.uint32)
     gen_s = time.perf_counter() - t0
@@ -85,8 +76,7 @@ def run_mixed(args, cfg):
         pg.barrier()
     a0, a1 = ev(), ev()
     g = Graph(nv, hints, bucket_bytes=S, load_factor=args.load_factor, rank=rank, nranks=world,
-              set_variant=args.variant == "set",
-              nccl_unique_id=uid)
+              set_variant=args.variant == "set", **gkw)
     BS, BD, BW = cu(bs), cu(bd), cu(bw)
     torch.cuda.synchronize()
     a0.record()
@@ -198,7 +188,7 @@ def run_mixed(args, cfg):
                                f"{VB:,} vertices + re-insert {RB:,} edges (global)",
                    "bucket_bytes": S, "load_factor": args.load_factor,
                    "l2": "flushed (256 MiB write) before every timed op; tables >> L2",
-                   "parallelism": f"source-vertex sharding x{world}" if world > 1 else "single GPU"},
+                   "parallelism": parallelism_label(world)},
         "ops": ops, "bulk_build": {"insert_ms": bulk_ms, "unique_added": int(added0)},
         "roofline": roofline, "gpu_launches": prof["launches"], "clocks": clocks,
         "graph": {k: st_[k] for k in ("live_pairs", "tombstones", "max_chain", "pool_bytes")},
@@ -208,8 +198,7 @@ def run_mixed(args, cfg):
         print(json.dumps(line), flush=True)
     g.close()
     if pg:
-        pg.barrier()
-        pg.destroy_process_group()
+        pg.close()
     return 0
 
 
@@ -327,8 +316,7 @@ def run_tc(args, cfg):
                                f"per wedge)",
                    "bucket_bytes": S, "load_factor": args.load_factor, "variant": variant,
                    "l2": "flushed (256 MiB write) before every step",
-                   "parallelism": f"replicas x{world}, wedges split by u mod {world}"
-                   if world > 1 else "single GPU"},
+                   "parallelism": parallelism_label(world, f"replicas, wedges split by u mod {world},")},
         "tc": {"triangles_per_step": tri, "tc_ms_per_step": t_tc / K,
                "insert_ms_per_step": t_ins / K, "wedges_per_tc": wedges,
                "wedge_G_per_s": sum(wedges) / (t_tc * 1e-3) / 1e9,
@@ -342,8 +330,7 @@ def run_tc(args, cfg):
         print(json.dumps(line), flush=True)
     g.close()
     if pg:
-        pg.barrier()
-        pg.destroy_process_group()
+        pg.close()
     return 0
 
 
