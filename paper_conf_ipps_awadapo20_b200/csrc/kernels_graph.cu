@@ -479,8 +479,8 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // of the pool (coalesced, G lanes per bucket); every live key in D becomes a
 // tombstone and the owner row's degree drops by one.
 // One launch per size class c: the pool of class c holds buckets of G units.
-// H (uniform layouts): one pass over the pool's allocated buckets and then the home
-// buckets (bucket r = row r's chain 0), as one range of bump + rows buckets.
+// H: the home pool (uniform layouts; bucket r = row r's chain 0, header in the last
+// unit) instead of pool `cls`.
 template <int G, int S, bool H = false>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     const u32* __restrict__ filter, u32 fshift,
@@ -499,13 +499,8 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
   if (ld_relaxed_u32(&t.ctl->fail_epoch) == epoch) return;
   for (u32 i = threadIdx.x; i < kVdelFilterBits / 32; i += blockDim.x) sf[i] = filter[i];
   __syncthreads();
-  const u32 npool = ld_relaxed_u32(&t.ctl->bump[cls]);
-  const u64 nbk = H ? (u64)npool + t.rows : (u64)npool;
-  u32* const pool = by_class(t.pool, cls);
-  // bucket b of the range: pool bucket b, or (H) home bucket b - npool
-  auto at = [&](u64 b) -> u32* {
-    return (H && b >= npool) ? t.home + (b - npool) * W : pool + b * W;
-  };
+  const u32 nbk = H ? (u32)t.rows : ld_relaxed_u32(&t.ctl->bump[cls]);
+  u32* const pool = H ? t.home : by_class(t.pool, cls);
   const u64 gid = ((u64)blockIdx.x * blockDim.x + threadIdx.x) / G;
   const u64 ng = ((u64)gridDim.x * blockDim.x) / G;
   for (u64 b0 = gid; b0 < nbk; b0 += ng * U) {
@@ -518,7 +513,7 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
     for (int k0 = 0; k0 < U; k0 += G) {
       const u32 k = k0 + g.gl;
       const u64 b = b0 + (u64)k * ng;
-      const bool l = k < (u32)U && b < nbk && *at(b) != kEmpty;
+      const bool l = k < (u32)U && b < nbk && pool[b * W] != kEmpty;
       live |= g.ballot(l) << k0;
     }
 #else
@@ -529,17 +524,17 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
     for (int k = 0; k < U; ++k) {
       const u64 b = (live >> k) & 1u ? b0 + (u64)k * ng : nbk;
 #ifdef DG_SWEEP_LDCS
-      q[k] = b < nbk ? __ldcs(reinterpret_cast<const uint4*>(at(b) + 4 * g.gl))
+      q[k] = b < nbk ? __ldcs(reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl))
                      : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
 #else
-      q[k] = b < nbk ? *reinterpret_cast<const uint4*>(at(b) + 4 * g.gl)
+      q[k] = b < nbk ? *reinterpret_cast<const uint4*>(pool + b * W + 4 * g.gl)
                      : make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
 #endif
     }
 #pragma unroll
     for (int k = 0; k < U; ++k) {
       const u64 b = b0 + (u64)k * ng;
-      u32* bp = at(b < nbk ? b : 0);
+      u32* bp = pool + b * W;
       const uint4 x = q[k];
       const u32 owner = g.shfl(x.w, G - 1);
       u32 dec = 0;
@@ -573,16 +568,17 @@ cudaError_t launch_vdel_sweep(int lay, const Tables& t, const u32* bitmap, const
     note_kernel(3);
     return cudaGetLastError();
   }
-  switch (lay) {  // uniform layouts: the pool and the home buckets in one pass
+  switch (lay) {  // uniform layouts: the pool, then the home buckets
 #define DG_CASE(G_, S_)                                                                      \
   case DG_LAY(G_, S_):                                                                       \
+    k_vdel_sweep<G_, S_><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);        \
     k_vdel_sweep<G_, S_, true><<<blocks, 256, 0, s>>>(t, bitmap, filter, fshift, epoch, 0);  \
     break;
     DG_FOR_LAYOUTS(DG_CASE)
 #undef DG_CASE
     default: return cudaErrorInvalidValue;
   }
-  note_kernel(1);
+  note_kernel(2);
   return cudaGetLastError();
 }
 
