@@ -479,8 +479,8 @@ cudaError_t launch_vdel_mark(const u32* ids, u64 n, u64 nv, u32 epoch, u32* bitm
 // of the pool (coalesced, G lanes per bucket); every live key in D becomes a
 // tombstone and the owner row's degree drops by one.
 // One launch per size class c: the pool of class c holds buckets of G units.
-// H: the home pool (uniform layouts; bucket r = row r's chain 0, header in the last
-// unit) instead of pool `cls`.
+// H: the home pool (uniform layouts; bucket r = row r's chain 0) instead of pool
+// `cls` (a second launch; one merged pass over both measured slower).
 template <int G, int S, bool H = false>
 __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restrict__ bitmap,
                                                     const u32* __restrict__ filter, u32 fshift,
