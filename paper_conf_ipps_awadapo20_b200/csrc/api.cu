@@ -415,7 +415,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   a.sorted_path = (!no_sorted && !mirror && epoch == g->validated_epoch && n >= (1u << 18)) ? 1u : 0u;
   static const u32 excl_chains = std::getenv("DG_EXCL_CHAINS")
                                      ? (u32)std::atoi(std::getenv("DG_EXCL_CHAINS")) : 256u;
-  a.excl_chains = excl_chains;
+  a.excl_chains = std::min<u32>(excl_chains, 256u);  // (k_insert_sorted packs chain < 256)
   // small batches: the insert kernel's last block does the allocator fixup (one launch
   // instead of two; a large batch returns more spare buckets than one block copies fast)
   const bool fused = !g->adaptive && !retry_mode && !a.sorted_path && n_ops <= (1u << 18);
