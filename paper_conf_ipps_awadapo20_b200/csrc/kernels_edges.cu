@@ -484,6 +484,9 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
   return deferred;
 }
 
+#ifndef DG_INPUT_PF
+#define DG_INPUT_PF 0  // (measured: no gain on cfg2, -1% on cfg3)
+#endif
 #ifndef DG_QUERY_PREFETCH
 #define DG_QUERY_PREFETCH 0
 #endif
@@ -549,6 +552,17 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
   for (u64 chunk = warp; chunk * 32 < a.n_ops; chunk += nwarps) {
     const u64 j = chunk * 32 + g.lane;
     const bool valid = j < a.n_ops;
+#if DG_INPUT_PF
+    // the next chunk's input lines (32 ops = one 128-B line per array) into L2 now, so
+    // its staging loads do not wait on DRAM (no registers held across the iteration)
+    if (!a.idx && g.lane < 3) {
+      const u64 nx = (chunk + nwarps) * 32;
+      if (nx < a.n) {
+        const u32* arr = g.lane == 0 ? a.src : g.lane == 1 ? a.dst : a.w;
+        if (arr) prefetch_l2(arr + nx);
+      }
+    }
+#endif
     const u64 opid = valid ? (a.idx ? a.idx[j] : j) : 0;
     // (off by default) load the NEXT chunk's sources now and prefetch their directory
     // entries into L2 after this chunk is probed, so the next chunk's directory gather
