@@ -830,3 +830,25 @@ def test_adaptive_promotion_and_memory():
     assert sa["table_bytes"] <= su["table_bytes"] // 2
     a.close()
     u.close()
+
+
+def test_src_sorted_batch_beyond_2_24_rows():
+    """The sorted path's chain groups use a 32-bit (row, chain) key below 2^24 rows and
+    the exact 64-bit key above: a src-sorted batch on a graph of 2^24 + 4096 vertices,
+    rows on both sides of the boundary, with hub rows (> 256 chains: per-op path)."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = (1 << 24) + 4096
+    rs = np.random.RandomState(24)
+    rows = np.concatenate([rs.randint(0, nv, 300_000), np.full(60_000, nv - 7),
+                           np.full(40_000, 5)]).astype(np.uint32)
+    dst = rs.randint(0, nv, rows.size).astype(np.uint32)
+    w = rs.randint(0, 1 << 32, rows.size, dtype=np.uint64).astype(np.uint32)
+    order = np.argsort(rows, kind="stable")
+    s, d, w = rows[order], dst[order], w[order]
+    hints = np.zeros(nv, np.uint32)
+    hints[nv - 7] = 60_000  # > 256 chains: the per-op path inside the sorted kernel
+    g = Graph(nv, hints)
+    o = Oracle(nv)
+    assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
+    check_against_oracle(g, o, "sorted batch, 2^24+ rows")
+    g.close()
