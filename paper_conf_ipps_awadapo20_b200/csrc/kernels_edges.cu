@@ -637,6 +637,19 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
 #ifndef DG_SORTED_PF  // load the next chunk's inputs while the current one is installed
 #define DG_SORTED_PF 0    // (measured: 4.41 -> 4.51 ms on the cfg2 sorted build: registers)
 #endif
+#ifndef DG_SORTED_TMA  // stage the next chunk's inputs in shared memory with bulk copies
+#define DG_SORTED_TMA 0   // (measured: 3.87 -> 3.99 ms on the cfg2 sorted build)
+#endif
+#ifndef DG_SORTED_DENSE  // owned rows in dense passes (else: chunk pass + tail-row passes)
+#define DG_SORTED_DENSE 2
+#endif
+
+// one warp's staged 32-op chunk: src (with the 4 ops before the chunk), dst, weight
+struct alignas(16) SortedStage {
+  u32 src[36];
+  u32 dst[32];
+  u32 w[32];
+};
 
 // position of the n-th (0-based) set bit of m
 __device__ __forceinline__ u32 nth_bit(u32 m, u32 n) {
@@ -792,17 +805,67 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Ta
   };
   u32 nu = 0, nv = 0, nw = 0, np = 0;
   if (DG_SORTED_PF) load_in(warp, nu, nv, nw, np);
+#if DG_SORTED_TMA
+  // Double-buffered per-warp staging: while chunk c is installed, the TMA engine
+  // copies chunk c + nwarps into the other stage (full 32-op chunks of 16-B aligned
+  // arrays; other chunks load directly).
+  __shared__ SortedStage s_stage[kEdgeBlock / 32][2];
+  __shared__ unsigned long long s_bar[kEdgeBlock / 32][2];
+  const u32 wib = threadIdx.x >> 5;
+  const bool tma_ok =
+      ((reinterpret_cast<uintptr_t>(a.src) | reinterpret_cast<uintptr_t>(a.dst) |
+        reinterpret_cast<uintptr_t>(a.w)) & 15u) == 0;
+  if (tma_ok && lane == 0) {
+    mbar_init(&s_bar[wib][0], 1);
+    mbar_init(&s_bar[wib][1], 1);
+  }
+  __syncwarp();
+  // warp-uniform: stage chunk c into stage st; false = not staged (load it directly)
+  auto stage_in = [&](u64 c, u32 st) -> bool {
+    if (!tma_ok || (c + 1) * 32 > n) return false;
+    if (lane == 0) {
+      const u32 pre = c ? 4u : 0u;  // the 4 ops before the chunk (for `prev`)
+      SortedStage& sg = s_stage[wib][st];
+      fence_proxy_async_smem();  // this warp's earlier reads of the stage come first
+      mbar_expect_tx(&s_bar[wib][st], (32u + pre) * 4u + 128u + (a.w ? 128u : 0u));
+      bulk_g2s(sg.src + 4 - pre, a.src + c * 32 - pre, (32u + pre) * 4u, &s_bar[wib][st]);
+      bulk_g2s(sg.dst, a.dst + c * 32, 128u, &s_bar[wib][st]);
+      if (a.w) bulk_g2s(sg.w, a.w + c * 32, 128u, &s_bar[wib][st]);
+    }
+    return true;
+  };
+  u32 st = 0, parity = 0;  // parity bit s: the phase to wait for on stage s
+  bool staged = stage_in(warp, 0);
+#endif
   for (u64 chunk = warp; chunk * 32 < n; chunk += nwarps) {
     const u64 lo = chunk * 32;
     const u64 i = lo + lane;
     const bool valid = i < n;
     u32 u, v, w, prev;  // (prev: the row of the op before the chunk)
+#if DG_SORTED_TMA
+    __syncwarp();  // every lane has read the other stage (previous iteration)
+    const bool staged_next = stage_in(chunk + nwarps, st ^ 1u);
+    if (staged) {
+      mbar_wait(&s_bar[wib][st], (parity >> st) & 1u);
+      parity ^= 1u << st;
+      const SortedStage& sg = s_stage[wib][st];
+      u = sg.src[4 + lane];
+      v = sg.dst[lane];
+      w = a.w ? sg.w[lane] : 0u;
+      prev = lo ? sg.src[3] : kNil;
+    } else {
+      load_in(chunk, u, v, w, prev);
+    }
+    staged = staged_next;
+    st ^= 1u;
+#else
     if (DG_SORTED_PF) {
       u = nu; v = nv; w = nw; prev = np;
       load_in(chunk + nwarps, nu, nv, nw, np);  // consumed next iteration
     } else {
       load_in(chunk, u, v, w, prev);
     }
+#endif
     const u32 row = (t.nranks == 1) ? u : u / t.nranks;
     uint2 de = make_uint2(0, 0);  // {base (uniform: xbase), nb}
     if (valid) de = ld_dir(t.dir + row);
@@ -811,6 +874,65 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Ta
     const bool cas = valid && !excl;
     if (__any_sync(FULL, cas))
       run_ops<G, S, OP_INSERT, false, A>(t, a, g, cas, i, i, reuse, my_count, spare, bad_range);
+#if DG_SORTED_DENSE == 2
+    // 2. rows that start in this chunk: all their ops, in dense passes of 32
+    //    consecutive ops from the first row start on (a pass holds several rows; the
+    //    last row may run past the chunk).  Pass 0 takes the chunk's ops from the
+    //    registers (shifted by shuffles) and the tail row's next ops from memory.
+    const u32 starts = __ballot_sync(FULL, valid && (lo == 0 || u != prev));
+    if (starts) {
+      const u32 off = __ffs(starts) - 1;
+      const u32 tail_row = __shfl_sync(FULL, u, 31);  // started here (sorted), or kNil
+      const u32 trow = __shfl_sync(FULL, row, 31);
+      const uint2 tde = make_uint2(__shfl_sync(FULL, de.x, 31), __shfl_sync(FULL, de.y, 31));
+      const bool tail_ex = tail_row != kNil && tde.y <= a.excl_chains;
+      const u32 sl = (lane + off) & 31u;
+      u32 s2 = __shfl_sync(FULL, u, sl), v2 = __shfl_sync(FULL, v, sl);
+      u32 w2 = __shfl_sync(FULL, w, sl), r2 = __shfl_sync(FULL, row, sl);
+      uint2 de2 = make_uint2(__shfl_sync(FULL, de.x, sl), __shfl_sync(FULL, de.y, sl));
+      bool in = __shfl_sync(FULL, valid ? 1 : 0, sl) != 0;
+      u64 i2 = lo + off + lane;
+      for (bool first = true;; first = false) {
+        if (!first || lane + off >= 32) {  // beyond the chunk: the tail row's next ops
+          const bool ok2 = tail_ex && i2 < n;  // (the three loads in parallel)
+          s2 = ok2 ? a.src[i2] : kNil;
+          v2 = ok2 ? a.dst[i2] : 0u;
+          w2 = (ok2 && a.w) ? a.w[i2] : 0u;
+          in = ok2 && s2 == tail_row;
+          r2 = trow;
+          de2 = tde;
+        }
+        install_owned<G, S, A>(t, a, in && de2.y <= a.excl_chains && v2 != s2, i2, r2, v2, w2,
+                               de2.x, de2.y, my_count);
+        if (!tail_ex || !__shfl_sync(FULL, in ? 1 : 0, 31) || i2 - lane + 32 >= n) break;
+        i2 += 32;
+      }
+    }
+#elif DG_SORTED_DENSE
+    // 2. rows that start in this chunk: all their ops, in dense passes of 32
+    //    consecutive ops from the first row start on (the last row may run past the
+    //    chunk; a pass holds several rows)
+    const u32 starts = __ballot_sync(FULL, valid && (lo == 0 || u != prev));
+    if (starts) {
+      const u32 tail_row = __shfl_sync(FULL, u, 31);  // started here (sorted), or kNil
+      const u32 tail_nb = __shfl_sync(FULL, de.y, 31);
+      for (u64 p0 = lo + (__ffs(starts) - 1);; p0 += 32) {
+        const u64 i2 = p0 + lane;
+        const bool ok2 = i2 < n;  // (the three loads in parallel: one round trip)
+        const u32 s2 = ok2 ? a.src[i2] : kNil;
+        const u32 v2 = ok2 ? a.dst[i2] : 0u;
+        const u32 w2 = (ok2 && a.w) ? a.w[i2] : 0u;
+        const bool in = ok2 && (i2 < lo + 32 || s2 == tail_row);
+        const u32 r2 = (t.nranks == 1) ? s2 : s2 / t.nranks;
+        uint2 de2 = make_uint2(0, 0);
+        if (in) de2 = ld_dir(t.dir + r2);
+        install_owned<G, S, A>(t, a, in && de2.y <= a.excl_chains && v2 != s2, i2, r2, v2, w2,
+                               de2.x, de2.y, my_count);
+        if (!__shfl_sync(FULL, in ? 1 : 0, 31) || p0 + 32 >= n || tail_nb > a.excl_chains)
+          break;  // the last row ended (or is not owned)
+      }
+    }
+#else
     // 2. rows this chunk owns (started in it): the whole row, 32 ops at a time
     const bool owned = excl && (lo == 0 || u != prev);
     install_owned<G, S, A>(t, a, owned && u != v, i, row, v, w, de.x, de.y, my_count);
@@ -822,14 +944,19 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Ta
       const u32 trow = (t.nranks == 1) ? tail_row : tail_row / t.nranks;
       for (u64 lo2 = lo + 32; lo2 < n; lo2 += 32) {
         const u64 i2 = lo2 + lane;
-        const bool in = i2 < n && a.src[i2] == tail_row;
-        const u32 v2 = in ? a.dst[i2] : 0u;
-        const u32 w2 = (in && a.w) ? a.w[i2] : 0u;
+        const bool ok2 = i2 < n;  // (the three loads in parallel: one round trip)
+        const u32 s2 = ok2 ? a.src[i2] : kNil;
+        const u32 v2r = ok2 ? a.dst[i2] : 0u;
+        const u32 w2r = (ok2 && a.w) ? a.w[i2] : 0u;
+        const bool in = ok2 && s2 == tail_row;
+        const u32 v2 = in ? v2r : 0u;
+        const u32 w2 = in ? w2r : 0u;
         install_owned<G, S, A>(t, a, in && v2 != tail_row, i2, trow, v2, w2, tde.x, tde.y,
                                my_count);
         if (__ballot_sync(FULL, in) != FULL) break;  // the run ended in this sub-chunk
       }
     }
+#endif
   }
   if (spare != kNil) t.ret_list[atomicAdd(&t.ctl->ret_count, 1u)] = spare;
   __syncwarp();
