@@ -2,9 +2,9 @@
 //
 // Data layout in HBM:
 //   directory  : DirEntry[local_rows], 8 B per row {base bucket, #base buckets} and
-//   degree     : u32[local_rows], the exact neighbour count (the paper's vertex
-//                dictionary holds both; split so the
-//                read-mostly 8-B entries and the 4-B counters stay L2-resident)
+//   degree     : the exact neighbour count (the paper's vertex dictionary holds it,
+//                P:L316-322, L399-407, L426-428): u32[local_rows] (L2-resident),
+//                or, with DG_HOME_DEG=1, the last word of the row's HOME bucket
 //   pool       : bucket array; bucket b occupies words [b*W, (b+1)*W), W = bucket_bytes/4.
 //                words 2i, 2i+1 = (key, value) of pair i, i < BC = W/2 - 1
 //                (set variant: word i = key i, i < BC = W - 2; see Lay below)
@@ -18,7 +18,12 @@
 // Home buckets (uniform layouts): chain 0 of row r is bucket r of a
 // separate HOME pool indexed by row, mapped exactly 2^31 buckets after the bucket
 // pool's base (so `pool + id * W` addresses both; home ids = kHomeBit | row).  Home
-// buckets are ordinary buckets (same slots, next, owner = row).  A probe reads the
+// buckets are ordinary buckets (same slots, next) whose owner is implied by their
+// index; with DG_HOME_DEG=1 their last word holds the row's DEGREE, so the degree
+// update of an op on chain 0 lands on the line its probe and CAS already hold (the
+// gather ceiling favours it: 15.7 G ops/s with a separate counter array, 18.4 G with
+// the counter in the gathered line, tools/gather_ceiling.cu; the insert kernel does
+// not: see DG_HOME_DEG below).  A probe reads the
 // row's chain count from a 1-byte-per-row array (`nbs`, min(nb, 255): L2-resident,
 // 4.8 MB on cfg2): a key that hashes to chain 0 goes straight to the home bucket
 // without the directory; the others read the directory {xbase, nb} for chain j >= 1,
@@ -77,7 +82,9 @@ struct Tables {
   DirEntry* dir;     // uniform layouts: {xbase, nb}; adaptive: {first base bucket, nb}
   u32* home;         // uniform layouts: home bucket of every row (chain 0), W words each
   uint8_t* nbs;      // uniform layouts: min(nb, 255) per row
-  u32* deg;          // exact degree per local row
+  u32* deg;          // adaptive layout: exact degree per local row; uniform layouts: a
+                     // snapshot written by launch_degrees for the TC orientation
+  u32 hw;            // uniform layouts: words per home bucket (the degree is word hw-1)
   u32* pool[kClasses];   // bucket pool per size class
   u32* stack[kClasses];  // free stack per size class (bucket ids)
   DevCtl* ctl;
@@ -90,6 +97,23 @@ struct Tables {
   u32 hot_cap;       // capacity of hot_list
   u32 hot_steps;     // chain buckets an insert may walk before flagging its row
 };
+
+// The degree counter of a local row: the last word of its home bucket (uniform
+// layouts) or deg[row] (adaptive layout; uniform layouts too with DG_HOME_DEG=0).
+// (measured on B200, cfg2 2^24 batches, profiles/r02/ab/homedeg_*: the degree word
+// dirties a second sector of the home line, DRAM writes per insert launch 0.75 ->
+// 1.00 GB, insert 1.207 -> 1.413 ms, delete 0.810 -> 0.926 ms: off)
+#ifndef DG_HOME_DEG
+#define DG_HOME_DEG 0
+#endif
+__device__ __forceinline__ u32* deg_at(const Tables& t, u64 row) {
+  return t.hw ? t.home + row * t.hw + (t.hw - 1) : t.deg + row;
+}
+template <int G, bool A>
+__device__ __forceinline__ u32* deg_ptr(const Tables& t, u64 row) {
+  if constexpr (A || !DG_HOME_DEG) return t.deg + row;
+  else return t.home + row * (4 * G) + (4 * G - 1);
+}
 
 // ------------------------------------------------------------------ hashing ----
 // Q16: murmur3 fmix32, then multiply-shift onto [0, nb).  The paper defers the

@@ -112,6 +112,7 @@ struct dg_graph_s {
     t.home = adaptive ? nullptr : reinterpret_cast<uint32_t*>(home.ptr());
     t.nbs = adaptive ? nullptr : reinterpret_cast<uint8_t*>(nbsv.ptr());
     t.deg = reinterpret_cast<uint32_t*>(degv.ptr());
+    t.hw = (adaptive || !DG_HOME_DEG) ? 0u : (uint32_t)(bucket_bytes / 4);
     for (int c = 0; c < dg::kClasses; ++c) {
       t.pool[c] = c < ncls ? reinterpret_cast<uint32_t*>(pool[c].ptr()) : nullptr;
       t.stack[c] = c < ncls ? reinterpret_cast<uint32_t*>(stack[c].ptr()) : nullptr;

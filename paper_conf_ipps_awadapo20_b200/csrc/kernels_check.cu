@@ -54,7 +54,8 @@ __global__ void __launch_bounds__(256) k_check(Tables t, u64 nv, u32 rank, Invar
           break;
         }
         const GEO gb(t, b);
-        if (gb.p[gb.owner_word()] != (u32)row) {
+        // (a home bucket's owner is its index: its last word is the row's degree)
+        if (!gb.home && gb.p[gb.owner_word()] != (u32)row) {
           bump(&out->owner_mismatch);
           bad = true;
         }
@@ -125,7 +126,7 @@ __global__ void __launch_bounds__(256) k_check(Tables t, u64 nv, u32 rank, Invar
     }
     bad = __any_sync(0xFFFFFFFFu, bad);
     if (lane == 0) {
-      if (live != t.deg[row]) {
+      if (live != *deg_at(t, row)) {
         bump(&out->degree_mismatch);
         bad = true;
       }

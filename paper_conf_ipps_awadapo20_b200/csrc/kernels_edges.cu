@@ -359,7 +359,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
               // flag the row for re-sizing before the next batch (per-vertex chain
               // metric + rehash)
               if (++steps == t.hot_steps && t.hot_flags) {
-                const u32 dr = ld_relaxed_u32(t.deg + row);
+                const u32 dr = ld_relaxed_u32(deg_ptr<G, A>(t, row));
                 if (dr > nbase * GEO::bc_u(units)) {  // (home chains hold one less)
                   const u32 bit = 1u << (row & 31);
                   if (!(atomicOr(&t.hot_flags[row >> 5], bit) & bit)) {
@@ -377,7 +377,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
     // c. one atomic per lane, all in flight together
     if (OP == OP_DELETE && act == ACT_CAS_DEL) {
       if (atomicCAS(ff, v, kTomb) == v) {
-        atomicSub(&t.deg[row], 1u);
+        atomicSub(deg_ptr<G, A>(t, row), 1u);
         ++my_count;
       }
       pend = false;  // a lost CAS means another op deleted the key (Q5)
@@ -388,7 +388,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
                          : (u32)atomicCAS(reinterpret_cast<unsigned long long*>(ff), ffo,
                                           (unsigned long long)pack_pair(v, w));
       if (okey == (u32)ffo) {
-        atomicAdd(&t.deg[row], 1u);
+        atomicAdd(deg_ptr<G, A>(t, row), 1u);
         ++my_count;
         pend = false;
       } else if (okey == v) {  // a racing op installed the same key: replace
@@ -420,7 +420,7 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
               p += S ? 1 : 2;
               const u32 k2 = atomicCAS(p, kEmpty, v);
               if (k2 == kEmpty) {
-                atomicAdd(&t.deg[row], 1u);
+                atomicAdd(deg_ptr<G, A>(t, row), 1u);
                 ++my_count;
               }
               if (k2 == kEmpty || k2 == v) {  // installed, or a racing op's v: replace
@@ -774,7 +774,7 @@ __device__ __forceinline__ void install_owned(const Tables& t, const EdgeBatch& 
   }
   // one degree update per group (Alg1:L9-10): its leader adds the group's installs
   const u32 sm = __ballot_sync(FULL, store) & gm;
-  if (store && (sm & below) == 0) atomicAdd(&t.deg[row], __popc(sm));
+  if (store && (sm & below) == 0) atomicAdd(deg_ptr<G, A>(t, row), __popc(sm));
   __syncwarp();  // the stores are visible to the warp's next walk
 }
 

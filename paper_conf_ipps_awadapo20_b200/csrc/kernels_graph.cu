@@ -116,7 +116,7 @@ __global__ void k_init_rows(Tables t, u64 row0, u64 count, const u32* rows, cons
     e.base = (c << kClassShift) | idx;
     e.nb = n;
     t.dir[row] = e;
-    t.deg[row] = 0;
+    *deg_at(t, row) = 0;
     const u32 wc = by_class(cb.words, c);
     u32* pool = by_class(t.pool, c);
     for (u32 k = 0; k + home < n; ++k) pool[(u64)(idx + k) * wc + wc - 1] = row;
@@ -124,7 +124,7 @@ __global__ void k_init_rows(Tables t, u64 row0, u64 count, const u32* rows, cons
       uint4* hb = reinterpret_cast<uint4*>(t.home + (u64)row * wc);
       const uint4 empty4 = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
       for (u32 uu = 0; uu + 1 < wc / 4; ++uu) hb[uu] = empty4;
-      hb[wc / 4 - 1] = make_uint4(kEmpty, kEmpty, kNil, row);
+      hb[wc / 4 - 1] = make_uint4(kEmpty, kEmpty, kNil, 0u);  // (degree 0)
       t.nbs[row] = (uint8_t)(n < 255u ? n : 255u);
     }
     if (rows && t.hot_flags) atomicAnd(&t.hot_flags[row >> 5], ~(1u << (row & 31)));
@@ -181,30 +181,36 @@ cudaError_t launch_max_id(const u32* ids, u64 n, u32* out, cudaStream_t s) {
 }
 
 // ------------------------------------------------------------------ degrees ----
-__global__ void k_degrees(const u32* deg, u64 rows, u32* out) {
+// (uniform layouts: the last word of every home bucket, one 32-B sector per row)
+__global__ void k_degrees(Tables t, u32* out) {
   const u64 stride = (u64)gridDim.x * blockDim.x;
-  for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < rows; r += stride)
-    out[r] = deg[r];
+  for (u64 r = (u64)blockIdx.x * blockDim.x + threadIdx.x; r < t.rows; r += stride)
+    out[r] = *deg_at(t, r);
 }
 
 cudaError_t launch_degrees(const Tables& t, u32* out, cudaStream_t s) {
   if (t.rows == 0) return cudaSuccess;
   u64 blocks = (t.rows + 255) / 256;
   if (blocks > 65535) blocks = 65535;
-  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t.deg, t.rows, out); note_kernel(1);
+  k_degrees<<<(unsigned)blocks, 256, 0, s>>>(t, out); note_kernel(1);
   return cudaGetLastError();
 }
 
 // ------------------------------------------------------------ export (a12) ----
 struct DegAt {
-  const u32* deg;
+  const u32* deg;   // adaptive layout
+  const u32* home;  // uniform layouts: degree = word hw-1 of home bucket i
+  u32 hw;
   u64 rows;
-  __host__ __device__ u64 operator()(u64 i) const { return i < rows ? (u64)deg[i] : 0ull; }
+  __host__ __device__ u64 operator()(u64 i) const {
+    if (i >= rows) return 0ull;
+    return hw ? (u64)home[i * hw + hw - 1] : (u64)deg[i];
+  }
 };
 
 cudaError_t launch_export_offsets(const Tables& t, u64* ro, void** temp, size_t* temp_bytes,
                                   cudaStream_t s) {
-  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0), DegAt{t.deg, t.rows});
+  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0), DegAt{t.deg, t.home, t.hw, t.rows});
   size_t need = 0;
   cudaError_t e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, ro, (int64_t)(t.rows + 1), s);
   if (e != cudaSuccess) return e;
@@ -536,7 +542,7 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
       const u64 b = b0 + (u64)k * ng;
       u32* bp = pool + b * W;
       const uint4 x = q[k];
-      const u32 owner = g.shfl(x.w, G - 1);
+      const u32 owner = H ? (u32)b : g.shfl(x.w, G - 1);  // (home: word W-1 = degree)
       u32 dec = 0;
 #pragma unroll
       for (int j = 0; j < LY::SPU; ++j) {
@@ -547,7 +553,7 @@ __global__ void __launch_bounds__(256) k_vdel_sweep(Tables t, const u32* __restr
             atomicCAS(bp + LY::word(g.gl, j), kk, kTomb) == kk)
           ++dec;
       }
-      if (dec) atomicSub(&t.deg[owner], dec);
+      if (dec) atomicSub(deg_at(t, owner), dec);
     }
   }
 }
@@ -677,7 +683,7 @@ __global__ void __launch_bounds__(256) k_vdel_neighbors(Tables t, const u32* ded
           const DirEntry dv = t.dir[v];
           if (purge_delete<G, S, A>(t, g, chain_head<A>(dv.base, v, bucket_of(u, dv.nb)), u) &&
               g.gl == 0)
-            atomicSub(&t.deg[v], 1u);
+            atomicSub(deg_at(t, v), 1u);
         }
       }
       b = g.shfl(q.z, gb.units - 1);
@@ -728,7 +734,8 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
       u32* bp = gb.p + 4 * g.gl;
       const uint4 q = in ? ld_relaxed_v4(bp) : empty4;
       const u32 next = g.shfl(q.z, gb.units - 1);
-      if (g.gl == gb.units - 1) st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, base_bucket ? row : kNil));
+      if (g.gl == gb.units - 1)  // (a home bucket's last word is the degree := 0)
+        st_v4(bp, make_uint4(kEmpty, kEmpty, kNil, gb.home ? 0u : base_bucket ? row : kNil));
       else if (in) st_v4(bp, empty4);
       if (!base_bucket && g.gl == 0) {
         const u32 c = b >> kClassShift;
@@ -737,7 +744,7 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
       base_bucket = false;
       b = next;
     }
-    if (j == 0 && g.gl == 0) t.deg[row] = 0;
+    if (A && j == 0 && g.gl == 0) t.deg[row] = 0;
   }
 }
 

@@ -29,7 +29,7 @@ __global__ void k_hot_sizes(Tables t, u32 n, u32 lf_milli, u32 bc, u32 flush, u3
     }
     const u32 row = t.hot_list[k];
     const DirEntry de = t.dir[row];
-    const u64 d = t.deg[row];
+    const u64 d = *deg_at(t, row);
     if (adaptive) {  // size class and #buckets by the initial rule (k_initial_buckets)
       u64 v = class_size(flush ? d : 2 * d, lf_milli, set);
       const u32 oc = de.base >> kClassShift;
@@ -156,7 +156,7 @@ __global__ void __launch_bounds__(256) k_tomb_sweep(Tables t, u32 cls) {
     bool tomb = false;
 #pragma unroll
     for (int j = 0; j < LY::SPU; ++j) tomb |= LY::has(g.gl, j) && LY::key(x, j) == kTomb;
-    const u32 owner = g.shfl(x.w, G - 1);
+    const u32 owner = H ? (u32)b : g.shfl(x.w, G - 1);  // (home: word W-1 = degree)
     if (g.ballot(tomb) && g.gl == 0) {
       const u32 bit = 1u << (owner & 31);
       if (!(atomicOr(&t.hot_flags[owner >> 5], bit) & bit)) {

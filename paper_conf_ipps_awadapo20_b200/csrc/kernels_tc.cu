@@ -243,6 +243,9 @@ cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* ds
                                    u32 nparts, u64* ocnt, u32* big, int sms, cudaStream_t s) {
   cudaError_t e = cudaMemsetAsync(big, 0, 4, s);
   if (e != cudaSuccess) return e;
+  // uniform layouts keep degrees in the home buckets: snapshot them into t.deg (one
+  // 32-B sector per row) so the orientation's random degree reads hit a dense array
+  if (t.hw && (e = launch_degrees(t, t.deg, s)) != cudaSuccess) return e;
   k_tc_orient_count<<<(unsigned)sms * 8, 256, 0, s>>>(ro, dst, t.deg, t.rows, part, nparts, ocnt,
                                                       big);
   k_tc_orient_count_big<<<(unsigned)sms * 2, 256, 0, s>>>(ro, dst, t.deg, ocnt, big);
