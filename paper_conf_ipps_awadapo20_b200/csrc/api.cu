@@ -471,10 +471,61 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   return DG_OK;
 }
 
-dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
-                       cudaStream_t s) {
+// Delete batches of at least this many ops are put in locality order before their
+// probe (kernels_order.cu; DG_ORDER_MIN_OPS overrides, 0 = never).
+u64 order_min_ops() {
+  static const u64 v = std::getenv("DG_ORDER_MIN_OPS")
+                           ? std::strtoull(std::getenv("DG_ORDER_MIN_OPS"), nullptr, 10)
+                           : (1ull << 20);
+  return v;
+}
+
+// Locality order of (src, dst[, mirror]) into g->ord: the permuted arrays, or
+// *ordered = false when the batch keeps its own order.  validate: the batch is
+// validated here (by the order's count pass, else k_validate); note: the verdict is
+// snapshot for validation_status() right after it.
+dg_status order_batch(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
+                      bool validate, bool note, const u32** osrc, const u32** odst, bool* ordered,
+                      cudaStream_t s) {
   const u64 n_ops = mirror ? 2 * n : n;
-  if (n_ops == 0) return DG_OK;
+  const u64 lim = order_min_ops();
+  *ordered = lim != 0 && n_ops >= lim && n_ops < (1ull << 32) && g->rows > 1;
+  if (!*ordered) {
+    if (validate) DG_CK(dg::launch_validate(src, dst, n, g->nv, epoch, g->ctl, g->sms, s));
+    if (note) DG_TRY(note_validation(g, s));
+    return DG_OK;
+  }
+  DG_CK(ensure_buf(g->ord[0], dg::order_scratch_bytes(g->sms)));
+  DG_CK(ensure_buf(g->ord[1], n_ops * 4));
+  DG_CK(ensure_buf(g->ord[2], n_ops * 4));
+  dg_status nst = DG_OK;
+  auto between = [&]() -> cudaError_t {
+    if (note) nst = note_validation(g, s);
+    return nst == DG_OK ? cudaSuccess : cudaErrorUnknown;
+  };
+  const cudaError_t e = dg::launch_order(src, dst, n, mirror, g->rows, g->nranks, g->ord[0].p,
+                                         (u32*)g->ord[1].p, (u32*)g->ord[2].p, g->nv, epoch,
+                                         validate ? g->ctl : nullptr, between, g->sms, s);
+  if (nst != DG_OK) return nst;
+  DG_CK(e);
+  *osrc = (const u32*)g->ord[1].p;
+  *odst = (const u32*)g->ord[2].p;
+  return DG_OK;
+}
+
+// validate / note: see order_batch (the router validates its batches itself)
+dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
+                       cudaStream_t s, bool validate, bool note) {
+  u64 n_ops = mirror ? 2 * n : n;
+  if (n_ops == 0) {
+    if (validate) DG_CK(dg::launch_validate(src, dst, n, g->nv, epoch, g->ctl, g->sms, s));
+    if (note) DG_TRY(note_validation(g, s));
+    return DG_OK;
+  }
+  prof_mark(g, PROF_DELETE, s);
+  bool ordered = false;
+  DG_TRY(order_batch(g, src, dst, n, mirror, epoch, validate, note, &src, &dst, &ordered, s));
+  if (ordered) n = n_ops;  // explicit directed ops (mirrors expanded)
   dg::EdgeBatch a{};
   a.src = src;
   a.dst = dst;
@@ -482,7 +533,6 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
   a.n_ops = n_ops;
   a.epoch = epoch;
   a.nv = g->nv;
-  prof_mark(g, PROF_DELETE, s);
   DG_CK(dg::launch_delete(g->lay, g->tables(), a, g->sms, s));
   prof_mark(g, PROF_DELETE, s);
   return DG_OK;
@@ -990,9 +1040,7 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
     // host inputs, no count requested: as in dg_insert_edges
     DG_TRY(upload_async(g, 11, src, n * 4, s, &ds));
     DG_TRY(upload_async(g, 12, dst, n * 4, s, &dd));
-    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
-    DG_TRY(note_validation(g, s));
-    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s));
+    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s, true, true));
     DG_TRY(release_slots(g, 11, 13, s));
     return validation_status(g, epoch);
   }
@@ -1001,8 +1049,7 @@ dg_status dg_delete_edges(dg_graph g, const uint32_t* src, const uint32_t* dst, 
   if (g->router) {
     DG_TRY(dg::router_delete(g, (const u32*)ds, (const u32*)dd, n, epoch, s));
   } else {
-    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
-    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s));
+    DG_TRY(dg::local_delete(g, (const u32*)ds, (const u32*)dd, n, !g->directed, epoch, s, true, false));
   }
   if (n_removed || host) {
     if (g->snap_pending) DG_CK(cudaEventSynchronize(g->snap_event));

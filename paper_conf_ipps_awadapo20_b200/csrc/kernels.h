@@ -1,6 +1,7 @@
 // kernels.h — host-callable launchers of the sm_100a kernels.
 #pragma once
 #include <cstdint>
+#include <functional>
 #include <cuda_runtime.h>
 
 #include "dg_common.cuh"
@@ -44,6 +45,15 @@ struct EdgeBatch {
 // for the degree-adaptive layout (G = 8 lanes, size class per bucket id)
 // (keys only); launchers that take `G` are layout-independent.
 // edge ops (kernels_edges.cu)
+// locality order of a delete batch (kernels_order.cu): partitions by local row >> shift,
+// at most kMaxOrderParts partitions of 2^shift rows
+constexpr u32 kOrderPartBits = 8;
+constexpr u32 kMaxOrderParts = 256;
+u32 order_shift(u64 rows);
+size_t order_scratch_bytes(int sms);
+cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64 rows, u32 nranks,
+                         void* scratch, u32* osrc, u32* odst, u64 nv, u32 epoch, DevCtl* ctl,
+                         const std::function<cudaError_t()>& between, int sms, cudaStream_t s);
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
                             int sms, cudaStream_t s);
 cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);

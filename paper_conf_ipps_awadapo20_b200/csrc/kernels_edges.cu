@@ -970,22 +970,38 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Ta
 // Validation (Q7) for mutating batches: any endpoint >= capacity rejects the
 // batch; also resets the per-batch counters (they are only written by kernels
 // that run after this one on the stream).
-__global__ void k_validate(const u32* __restrict__ src, const u32* __restrict__ dst, u64 n,
-                           u64 nv, u32 epoch, DevCtl* ctl) {
+__global__ void __launch_bounds__(256) k_validate(const u32* __restrict__ src,
+                                                 const u32* __restrict__ dst, u64 n, u64 nv,
+                                                 u32 epoch, DevCtl* ctl) {
+  constexpr int kItems = 8;  // loads issued before any is consumed
   if (blockIdx.x == 0 && threadIdx.x == 0) {
     ctl->count = 0;
     ctl->retry_count = 0;
   }
+  const u32 lane = threadIdx.x & 31u;
   bool bad = false, unsorted = false;
-  const u64 stride = (u64)gridDim.x * blockDim.x;
-  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += stride) {
-    const u32 u = src[i];
-    bad |= ((u64)u >= nv) | ((u64)dst[i] >= nv);
-    unsorted |= i > 0 && u < src[i - 1];  // (the neighbour's line is the same or cached)
+  const u64 step = (u64)gridDim.x * blockDim.x * kItems;
+  for (u64 i0 = (u64)blockIdx.x * blockDim.x * kItems; i0 < n; i0 += step) {
+    u32 us[kItems], vs[kItems], prev[kItems];
+#pragma unroll
+    for (int k = 0; k < kItems; ++k) {
+      const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
+      us[k] = i < n ? src[i] : 0u;
+      vs[k] = i < n ? dst[i] : 0u;
+      prev[k] = lane == 0 && i > 0 && i < n ? src[i - 1] : 0u;  // (the warp's left neighbour)
+    }
+#pragma unroll
+    for (int k = 0; k < kItems; ++k) {
+      const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
+      const u32 left = __shfl_up_sync(0xFFFFFFFFu, us[k], 1);
+      if (i < n) {
+        bad |= ((u64)us[k] >= nv) | ((u64)vs[k] >= nv);
+        unsorted |= i > 0 && us[k] < (lane == 0 ? prev[k] : left);
+      }
+    }
   }
-  if (__any_sync(0xFFFFFFFFu, bad) && (threadIdx.x & 31) == 0) atomicMax(&ctl->fail_epoch, epoch);
-  if (__any_sync(0xFFFFFFFFu, unsorted) && (threadIdx.x & 31) == 0)
-    atomicMax(&ctl->unsorted_epoch, epoch);
+  if (__any_sync(0xFFFFFFFFu, bad) && lane == 0) atomicMax(&ctl->fail_epoch, epoch);
+  if (__any_sync(0xFFFFFFFFu, unsorted) && lane == 0) atomicMax(&ctl->unsorted_epoch, epoch);
 }
 
 // After an insert phase: drop the popped entries from each class's free stack,
@@ -1116,7 +1132,7 @@ u64 max_groups(int G, int sms) {
 
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
                             int sms, cudaStream_t s) {
-  u64 blocks = (n + 255) / 256;
+  u64 blocks = (n + 2047) / 2048;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   if (blocks == 0) blocks = 1;
   k_validate<<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl); note_kernel(1);

@@ -744,7 +744,7 @@ __global__ void __launch_bounds__(256) k_vdel_clear(Tables t, const u32* dedup, 
       base_bucket = false;
       b = next;
     }
-    if (A && j == 0 && g.gl == 0) t.deg[row] = 0;
+    if (!t.hw && j == 0 && g.gl == 0) t.deg[row] = 0;  // (else the home-word store above)
   }
 }
 

@@ -676,7 +676,7 @@ dg_status router_delete(dg_graph g, const u32* src, const u32* dst, u64 n, u32 e
   if ((st = route_ops(g, src, dst, nullptr, n, !g->directed, false, false, s, &rx, &win)) != DG_OK)
     return st;
   if ((st = reset_counters(g, s)) != DG_OK) return st;
-  return local_delete(g, rx.src, rx.dst, r.roff[r.P], false, epoch, s);
+  return local_delete(g, rx.src, rx.dst, r.roff[r.P], false, epoch, s, false, false);
 }
 
 // Out-of-range queries (Q7/Q19) behave as at P = 1: they are not routed and answer 0,
