@@ -970,33 +970,68 @@ __global__ void __launch_bounds__(kEdgeBlock, DG_SORTED_MINB) k_insert_sorted(Ta
 // Validation (Q7) for mutating batches: any endpoint >= capacity rejects the
 // batch; also resets the per-batch counters (they are only written by kernels
 // that run after this one on the stream).
+template <bool VEC>
 __global__ void __launch_bounds__(256) k_validate(const u32* __restrict__ src,
                                                  const u32* __restrict__ dst, u64 n, u64 nv,
                                                  u32 epoch, DevCtl* ctl) {
-  constexpr int kItems = 8;  // loads issued before any is consumed
+  // kQ quads (VEC: 16-B loads, arrays 16-B aligned) or kQ * 4 single ops per thread and
+  // step, all loads issued before any is consumed
+  constexpr int kQ = 2;
   if (blockIdx.x == 0 && threadIdx.x == 0) {
     ctl->count = 0;
     ctl->retry_count = 0;
   }
   const u32 lane = threadIdx.x & 31u;
   bool bad = false, unsorted = false;
-  const u64 step = (u64)gridDim.x * blockDim.x * kItems;
-  for (u64 i0 = (u64)blockIdx.x * blockDim.x * kItems; i0 < n; i0 += step) {
-    u32 us[kItems], vs[kItems], prev[kItems];
+  const u64 step = (u64)gridDim.x * blockDim.x * kQ * 4;
+  for (u64 i0 = (u64)blockIdx.x * blockDim.x * kQ * 4; i0 < n; i0 += step) {
+    if constexpr (VEC) {
+      uint4 a[kQ], b[kQ];
+      u32 prev[kQ];
 #pragma unroll
-    for (int k = 0; k < kItems; ++k) {
-      const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
-      us[k] = i < n ? src[i] : 0u;
-      vs[k] = i < n ? dst[i] : 0u;
-      prev[k] = lane == 0 && i > 0 && i < n ? src[i - 1] : 0u;  // (the warp's left neighbour)
-    }
+      for (int k = 0; k < kQ; ++k) {
+        const u64 i = i0 + 4 * ((u64)k * blockDim.x + threadIdx.x);
+        if (i + 3 < n) {
+          a[k] = *reinterpret_cast<const uint4*>(src + i);
+          b[k] = *reinterpret_cast<const uint4*>(dst + i);
+        } else {  // the tail quad
+          a[k].x = i < n ? src[i] : 0u;      b[k].x = i < n ? dst[i] : 0u;
+          a[k].y = i + 1 < n ? src[i + 1] : a[k].x;  b[k].y = i + 1 < n ? dst[i + 1] : 0u;
+          a[k].z = i + 2 < n ? src[i + 2] : a[k].y;  b[k].z = i + 2 < n ? dst[i + 2] : 0u;
+          a[k].w = a[k].z;                   b[k].w = 0u;
+          if (i >= n) a[k] = make_uint4(0xFFFFFFFFu, 0xFFFFFFFFu, 0xFFFFFFFFu, 0xFFFFFFFFu);
+        }
+        prev[k] = lane == 0 && i > 0 && i < n ? src[i - 1] : 0u;  // (the warp's left neighbour)
+      }
 #pragma unroll
-    for (int k = 0; k < kItems; ++k) {
-      const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
-      const u32 left = __shfl_up_sync(0xFFFFFFFFu, us[k], 1);
-      if (i < n) {
-        bad |= ((u64)us[k] >= nv) | ((u64)vs[k] >= nv);
-        unsorted |= i > 0 && us[k] < (lane == 0 ? prev[k] : left);
+      for (int k = 0; k < kQ; ++k) {
+        const u64 i = i0 + 4 * ((u64)k * blockDim.x + threadIdx.x);
+        const u32 left = __shfl_up_sync(0xFFFFFFFFu, a[k].w, 1);
+        if (i < n) {
+          const u32 mx = max(max(a[k].x, a[k].y), max(a[k].z, a[k].w));
+          const u32 my = max(max(b[k].x, b[k].y), max(b[k].z, b[k].w));
+          bad |= ((u64)mx >= nv) | ((u64)my >= nv);
+          unsorted |= a[k].y < a[k].x || a[k].z < a[k].y || a[k].w < a[k].z ||
+                      (i > 0 && a[k].x < (lane == 0 ? prev[k] : left));
+        }
+      }
+    } else {
+      u32 us[kQ * 4], vs[kQ * 4], prev[kQ * 4];
+#pragma unroll
+      for (int k = 0; k < kQ * 4; ++k) {
+        const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
+        us[k] = i < n ? src[i] : 0u;
+        vs[k] = i < n ? dst[i] : 0u;
+        prev[k] = lane == 0 && i > 0 && i < n ? src[i - 1] : 0u;
+      }
+#pragma unroll
+      for (int k = 0; k < kQ * 4; ++k) {
+        const u64 i = i0 + (u64)k * blockDim.x + threadIdx.x;
+        const u32 left = __shfl_up_sync(0xFFFFFFFFu, us[k], 1);
+        if (i < n) {
+          bad |= ((u64)us[k] >= nv) | ((u64)vs[k] >= nv);
+          unsorted |= i > 0 && us[k] < (lane == 0 ? prev[k] : left);
+        }
       }
     }
   }
@@ -1135,7 +1170,11 @@ cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 e
   u64 blocks = (n + 2047) / 2048;
   if (blocks > (u64)sms * 8) blocks = (u64)sms * 8;
   if (blocks == 0) blocks = 1;
-  k_validate<<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl); note_kernel(1);
+  if (((reinterpret_cast<uintptr_t>(src) | reinterpret_cast<uintptr_t>(dst)) & 15) == 0)
+    k_validate<true><<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl);
+  else
+    k_validate<false><<<(unsigned)blocks, 256, 0, s>>>(src, dst, n, nv, epoch, ctl);
+  note_kernel(1);
   return cudaGetLastError();
 }
 

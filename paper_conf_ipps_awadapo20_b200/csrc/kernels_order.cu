@@ -24,7 +24,10 @@
 //   k_order_scatter : block b re-reads its range; a shared-memory cursor per partition
 //                     places each op (the order inside a (b, p) run is arbitrary)
 // No global atomics on the partition cursors (a per-tile reservation scheme measured
-// 0.24 ms per 2^24 ops on 148 cursor addresses).
+// 0.24 ms per 2^24 ops on 148 cursor addresses).  Measured on cfg2 2^24 deletes:
+// count 31 us, scan 7 us, scatter 120 us (reads 183 MB: partial output sectors are
+// re-read on eviction; L2 evict-first loads / evict-last stores did not change it),
+// delete probe 0.80 -> 0.54 ms.
 // Undirected batches (mirror = true) expand op j >= n to (dst[j-n], src[j-n]) here,
 // so the probe sees explicit directed ops.
 #include <functional>
@@ -39,7 +42,7 @@ namespace {
 constexpr int kOrdThreads = 256;
 constexpr int kOrdItems = 8;  // ops per thread per step (all loads issued first)
 constexpr u32 kOrdStep = kOrdThreads * kOrdItems;
-constexpr int kOrdBlocksPerSm = 8;
+constexpr int kOrdBlocksPerSm = 4;  // (64 registers: 4 blocks of 256 threads resident)
 constexpr u32 kOrdMaxBlocks = 2048;  // k_order_scan: one column per block, 2 per thread
 
 __device__ __forceinline__ void op_of(const u32* src, const u32* dst, u64 n, u64 j, u32& u, u32& v) {
@@ -54,15 +57,68 @@ __device__ __forceinline__ u32 part_of(u32 u, u32 nranks, u32 shift, u32 nparts)
 }
 
 __device__ __forceinline__ void range_of(u64 n_ops, u64& lo, u64& hi) {
-  const u64 chunk = (n_ops + gridDim.x - 1) / gridDim.x;
+  const u64 chunk = ((n_ops + gridDim.x - 1) / gridDim.x + 3) & ~3ull;  // (quads stay aligned)
   lo = (u64)blockIdx.x * chunk;
+  if (lo > n_ops) lo = n_ops;
   hi = lo + chunk < n_ops ? lo + chunk : n_ops;
+}
+
+// The ops of one step (kOrdItems per thread, all loads issued before any is used):
+// VEC (16-B aligned arrays, n % 4 == 0 for mirrors): two 16-B loads per array and
+// thread, ops j0 + 4 (k kOrdThreads + t) + i; else one 4-B load per op, ops
+// j0 + k kOrdThreads + t.  Bit k of `valid` marks item k as an op of [j0, hi).
+// need_v: also load v (validation reads both endpoints; mirrors are validated at
+// their original op, so their v is not needed then).
+template <bool VEC>
+__device__ __forceinline__ u32 load_step(const u32* __restrict__ src, const u32* __restrict__ dst,
+                                         u64 n, u64 j0, u64 hi, bool need_v,
+                                         u32 (&us)[kOrdItems], u32 (&vs)[kOrdItems]) {
+  u32 valid = 0;
+  if constexpr (VEC) {
+#pragma unroll
+    for (int k = 0; k < kOrdItems / 4; ++k) {
+      const u64 j = j0 + 4 * ((u64)k * kOrdThreads + threadIdx.x);
+      if (j + 3 < hi) {
+        const bool m = j >= n;  // (n % 4 == 0: a quad never straddles n)
+        const u64 jj = m ? j - n : j;
+        const uint4 a = *reinterpret_cast<const uint4*>((m ? dst : src) + jj);
+        us[4 * k] = a.x; us[4 * k + 1] = a.y; us[4 * k + 2] = a.z; us[4 * k + 3] = a.w;
+        if (need_v || m) {
+          const uint4 b = *reinterpret_cast<const uint4*>((m ? src : dst) + jj);
+          vs[4 * k] = b.x; vs[4 * k + 1] = b.y; vs[4 * k + 2] = b.z; vs[4 * k + 3] = b.w;
+        } else {
+          vs[4 * k] = vs[4 * k + 1] = vs[4 * k + 2] = vs[4 * k + 3] = 0u;
+        }
+        valid |= 0xFu << (4 * k);
+      } else {
+#pragma unroll
+        for (int i = 0; i < 4; ++i) {
+          us[4 * k + i] = vs[4 * k + i] = 0u;
+          if (j + i < hi) {
+            op_of(src, dst, n, j + i, us[4 * k + i], vs[4 * k + i]);
+            valid |= 1u << (4 * k + i);
+          }
+        }
+      }
+    }
+  } else {
+#pragma unroll
+    for (int k = 0; k < kOrdItems; ++k) {
+      const u64 j = j0 + (u64)k * kOrdThreads + threadIdx.x;
+      us[k] = vs[k] = 0u;
+      if (j < hi) {
+        op_of(src, dst, n, j, us[k], vs[k]);
+        valid |= 1u << k;
+      }
+    }
+  }
+  return valid;
 }
 
 // ctl != nullptr: also the batch validation of k_validate (Q7: an endpoint >= nv
 // rejects the batch; the per-batch counters are reset), so a validated delete reads
-// its inputs once before the scatter instead of twice.  Mirror ops (j >= n) carry the
-// IDs of op j - n, validated there.
+// its inputs once before the scatter instead of twice.
+template <bool VEC>
 __global__ void __launch_bounds__(kOrdThreads) k_order_count(const u32* __restrict__ src,
                                                              const u32* __restrict__ dst, u64 n,
                                                              u64 n_ops, u32 nranks, u32 shift,
@@ -78,20 +134,22 @@ __global__ void __launch_bounds__(kOrdThreads) k_order_count(const u32* __restri
   u64 lo, hi;
   range_of(n_ops, lo, hi);
   bool bad = false;
+  // the next step's loads are issued before the current step is counted
+  u32 us[kOrdItems], vs[kOrdItems];
+  u32 valid = lo < hi ? load_step<VEC>(src, dst, n, lo, hi, ctl != nullptr, us, vs) : 0u;
   for (u64 j0 = lo; j0 < hi; j0 += kOrdStep) {
-    u32 us[kOrdItems], vs[kOrdItems];
-#pragma unroll
-    for (int k = 0; k < kOrdItems; ++k) {
-      const u64 j = j0 + (u64)k * kOrdThreads + threadIdx.x;
-      us[k] = j < hi ? (j < n ? src[j] : dst[j - n]) : 0u;
-      vs[k] = ctl && j < hi && j < n ? dst[j] : 0u;
-    }
+    u32 nus[kOrdItems], nvs[kOrdItems];
+    const u32 nvalid =
+        j0 + kOrdStep < hi ? load_step<VEC>(src, dst, n, j0 + kOrdStep, hi, ctl != nullptr, nus, nvs) : 0u;
 #pragma unroll
     for (int k = 0; k < kOrdItems; ++k)
-      if (j0 + (u64)k * kOrdThreads + threadIdx.x < hi) {
+      if ((valid >> k) & 1u) {
         bad |= ((u64)us[k] >= nv) | ((u64)vs[k] >= nv);
         atomicAdd(&hs[part_of(us[k], nranks, shift, nparts)], 1u);
       }
+#pragma unroll
+    for (int k = 0; k < kOrdItems; ++k) { us[k] = nus[k]; vs[k] = nvs[k]; }
+    valid = nvalid;
   }
   if (ctl && __any_sync(0xFFFFFFFFu, bad) && (threadIdx.x & 31) == 0)
     atomicMax(&ctl->fail_epoch, epoch);
@@ -134,6 +192,7 @@ __global__ void __launch_bounds__(1024) k_order_scan(u32* h, const u32* totals, 
 // them out in that order, so consecutive threads store consecutive slots of one
 // partition's run (scattering op by op made every warp store touch 32 sectors:
 // 0.31 ms per 2^24 ops).
+template <bool VEC>
 __global__ void __launch_bounds__(kOrdThreads) k_order_scatter(
     const u32* __restrict__ src, const u32* __restrict__ dst, u64 n, u64 n_ops, u32 nranks,
     u32 shift, u32 nparts, const u32* __restrict__ h, u32* __restrict__ osrc,
@@ -148,20 +207,19 @@ __global__ void __launch_bounds__(kOrdThreads) k_order_scatter(
   cur[t] = t < nparts ? h[(size_t)blockIdx.x * kMaxOrderParts + t] : 0u;
   u64 lo, hi;
   range_of(n_ops, lo, hi);
+  // software pipeline: the next step's loads are issued once the current step's ops
+  // are staged in shared memory, so they are in flight during its stores
+  u32 us[kOrdItems], vs[kOrdItems];
+  u32 valid = lo < hi ? load_step<VEC>(src, dst, n, lo, hi, true, us, vs) : 0u;
   for (u64 j0 = lo; j0 < hi; j0 += kOrdStep) {
     cnt[t] = 0;
     __syncthreads();
-    u32 us[kOrdItems], vs[kOrdItems], ps[kOrdItems], rk[kOrdItems];
+    u32 ps[kOrdItems], rk[kOrdItems];
 #pragma unroll
     for (int k = 0; k < kOrdItems; ++k) {
-      const u64 j = j0 + (u64)k * kOrdThreads + t;
-      if (j < hi) op_of(src, dst, n, j, us[k], vs[k]);
-    }
-#pragma unroll
-    for (int k = 0; k < kOrdItems; ++k) {
-      const bool in = j0 + (u64)k * kOrdThreads + t < hi;
+      const bool in = (valid >> k) & 1u;
       ps[k] = in ? part_of(us[k], nranks, shift, nparts) : kNil;
-      if (in) rk[k] = atomicAdd(&cnt[ps[k]], 1u);
+      rk[k] = in ? atomicAdd(&cnt[ps[k]], 1u) : 0u;
     }
     __syncthreads();
     // exclusive scan of cnt over the partitions (thread t holds partition t)
@@ -189,6 +247,7 @@ __global__ void __launch_bounds__(kOrdThreads) k_order_scatter(
       st_v[at] = vs[k];
       st_p[at] = (uint8_t)ps[k];
     }
+    valid = j0 + kOrdStep < hi ? load_step<VEC>(src, dst, n, j0 + kOrdStep, hi, true, us, vs) : 0u;
     __syncthreads();
     const u32 m = (u32)(hi - j0 < kOrdStep ? hi - j0 : kOrdStep);
     for (u32 i = t; i < m; i += kOrdThreads) {  // runs of one partition are contiguous
@@ -236,11 +295,22 @@ cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64
   u32* totals = h + (size_t)nb * kMaxOrderParts;
   cudaError_t e = cudaMemsetAsync(totals, 0, kMaxOrderParts * 4, s);
   if (e != cudaSuccess) return e;
-  k_order_count<<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h, totals,
-                                           nv, epoch, ctl);
+  const bool vec = ((reinterpret_cast<uintptr_t>(src) | reinterpret_cast<uintptr_t>(dst)) & 15) == 0 &&
+                   (!mirror || n % 4 == 0);
+  if (vec)
+    k_order_count<true><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
+                                                   totals, nv, epoch, ctl);
+  else
+    k_order_count<false><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
+                                                    totals, nv, epoch, ctl);
   if (between && (e = between()) != cudaSuccess) return e;
   k_order_scan<<<nparts, 1024, 0, s>>>(h, totals, (u32)nb);
-  k_order_scatter<<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h, osrc, odst);
+  if (vec)
+    k_order_scatter<true><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
+                                                     osrc, odst);
+  else
+    k_order_scatter<false><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
+                                                      osrc, odst);
   note_kernel(3);
   return cudaGetLastError();
 }
