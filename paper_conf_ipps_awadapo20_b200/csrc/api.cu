@@ -330,8 +330,11 @@ dg_status plan_capacity(dg_graph g, u64 need, cudaStream_t s, bool* retry_mode) 
     // size, so that back-to-back calls do not come back here (a synchronisation)
     // before the cursors published by earlier launches catch up (refresh_bound).
     if (!limit) limit = std::min<u64>(4ull << 30, device_free_bytes() / 2);
+    // (64 launches of headroom: a host running ahead of the device synchronises once
+    // per 64 small batches, not once per 8 — 2^16-op inserts back to back: 81 -> 29 us
+    // per call, tools/call_overhead.py; the mapped headroom is capped at 2 GB)
     const u64 room = std::max<u64>(
-        std::min<u64>(8 * need, std::min<u64>(limit, 2ull << 30) / g->cbytes(c)), 65536);
+        std::min<u64>(64 * need, std::min<u64>(limit, 2ull << 30) / g->cbytes(c)), 65536);
     if (free_exact >= need + room) continue;
     if (free_exact >= need) {  // enough for this batch: top up the headroom if cheap
       if (!no_upfront) {
@@ -472,11 +475,13 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
 }
 
 // Delete batches of at least this many ops are put in locality order before their
-// probe (kernels_order.cu; DG_ORDER_MIN_OPS overrides, 0 = never).
+// probe (kernels_order.cu; DG_ORDER_MIN_OPS overrides, 0 = never).  Measured break-even
+// on cfg2 and cfg3 (profiles/r02/order/sweep.txt): 2^20 ops lose (0.086 -> 0.100 ms),
+// 2^21 break even, 2^22 / 2^23 / 2^24 gain 6 / 10 / 15%.
 u64 order_min_ops() {
   static const u64 v = std::getenv("DG_ORDER_MIN_OPS")
                            ? std::strtoull(std::getenv("DG_ORDER_MIN_OPS"), nullptr, 10)
-                           : (1ull << 20);
+                           : (1ull << 21);
   return v;
 }
 
