@@ -384,7 +384,7 @@ dg_status prepare_insert(dg_graph g, u64 n_ops, cudaStream_t s) {
 
 // insert n edges already resident on this GPU (their sources are local rows)
 dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n, bool mirror,
-                       u32 epoch, cudaStream_t s) {
+                       u32 epoch, cudaStream_t s, bool fuse_validate) {
   dg::Tables t = g->tables();
   const u64 n_ops = mirror ? 2 * n : n;
   if (n_ops == 0) return DG_OK;
@@ -423,6 +423,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
   // instead of two; a large batch returns more spare buckets than one block copies fast)
   const bool fused = !g->adaptive && !retry_mode && !a.sorted_path && n_ops <= (1u << 18);
   a.pub = fused ? g->d_hot : nullptr;
+  a.fuse_validate = fuse_validate ? 1u : 0u;
   prof_mark(g, PROF_INSERT, s);
   DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
   prof_mark(g, PROF_INSERT, s);
@@ -465,6 +466,7 @@ dg_status local_insert(dg_graph g, const u32* src, const u32* dst, const u32* w,
     a.n_ops = whole ? n_ops : failed;
     a.sorted_path = 0;  // re-runs go through k_edges
     a.pub = nullptr;
+    a.fuse_validate = 0;  // (validated by the first launch)
     a.retry_out = g->retry[cur ^ 1];
     a.retry_cap = next_cap;
     DG_CK(dg::launch_insert(g->lay, t, a, g->sms, s));
@@ -489,14 +491,18 @@ u64 order_min_ops() {
 // *ordered = false when the batch keeps its own order.  validate: the batch is
 // validated here (by the order's count pass, else k_validate); note: the verdict is
 // snapshot for validation_status() right after it.
+// *fused: a small batch left to the probe kernel's own validation (EdgeBatch
+// fuse_validate; not when the verdict must be snapshot before the probe).
 dg_status order_batch(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
                       bool validate, bool note, const u32** osrc, const u32** odst, bool* ordered,
-                      cudaStream_t s) {
+                      bool* fused, cudaStream_t s) {
   const u64 n_ops = mirror ? 2 * n : n;
   const u64 lim = order_min_ops();
   *ordered = lim != 0 && n_ops >= lim && n_ops < (1ull << 32) && g->rows > 1;
+  *fused = false;
   if (!*ordered) {
-    if (validate) DG_CK(dg::launch_validate(src, dst, n, g->nv, epoch, g->ctl, g->sms, s));
+    *fused = validate && !note && n_ops < dg::kFuseValidateMaxOps;
+    if (validate && !*fused) DG_CK(dg::launch_validate(src, dst, n, g->nv, epoch, g->ctl, g->sms, s));
     if (note) DG_TRY(note_validation(g, s));
     return DG_OK;
   }
@@ -528,8 +534,8 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
     return DG_OK;
   }
   prof_mark(g, PROF_DELETE, s);
-  bool ordered = false;
-  DG_TRY(order_batch(g, src, dst, n, mirror, epoch, validate, note, &src, &dst, &ordered, s));
+  bool ordered = false, fused = false;
+  DG_TRY(order_batch(g, src, dst, n, mirror, epoch, validate, note, &src, &dst, &ordered, &fused, s));
   if (ordered) n = n_ops;  // explicit directed ops (mirrors expanded)
   dg::EdgeBatch a{};
   a.src = src;
@@ -538,6 +544,7 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
   a.n_ops = n_ops;
   a.epoch = epoch;
   a.nv = g->nv;
+  a.fuse_validate = fused ? 1u : 0u;
   DG_CK(dg::launch_delete(g->lay, g->tables(), a, g->sms, s));
   prof_mark(g, PROF_DELETE, s);
   return DG_OK;
@@ -1013,10 +1020,15 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   if (g->router) {
     DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
   } else {
-    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
-    g->validated_epoch = epoch;
+    // a small batch validates inside its insert launch (one launch instead of two; no
+    // sortedness verdict: the src-sorted path is for batches >= 2^18)
+    const bool fuse = n > 0 && (g->directed ? n : 2 * n) < dg::kFuseValidateMaxOps;
+    if (!fuse) {
+      DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
+      g->validated_epoch = epoch;
+    }
     DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
-                            epoch, s));
+                            epoch, s, fuse));
   }
   if (n_added || host) {
     DG_TRY(read_ctl(g, s));

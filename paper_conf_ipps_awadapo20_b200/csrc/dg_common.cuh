@@ -76,6 +76,8 @@ struct DevCtl {
   u32 route_timeout; // a fused-exchange wait gave up on a peer (router.cu)
   u32 unsorted_epoch; // highest validated batch epoch whose sources were not sorted
   u32 fixup_done;     // blocks of k_fixup finished (last-block pattern; reset by the last)
+  u32 bar_count;      // grid barrier of a small k_edges launch with fused validation:
+  u32 bar_gen;        //   arrivals, generation (kernels_edges.cu grid_barrier)
 };
 
 struct Tables {

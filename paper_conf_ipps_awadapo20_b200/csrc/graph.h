@@ -146,8 +146,9 @@ void prof_mark(dg_graph g, int k, cudaStream_t s);
 dg_status grow_pool(dg_graph g, int c, uint64_t min_buckets, cudaStream_t s);
 dg_status rehash_hot(dg_graph g, cudaStream_t s);
 dg_status rehash_rows(dg_graph g, uint32_t n, bool flush, cudaStream_t s);
+// fuse_validate: the insert launch validates the batch itself (small batches, EdgeBatch)
 dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
-                       uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s);
+                       uint64_t n, bool mirror, uint32_t epoch, cudaStream_t s, bool fuse_validate = false);
 // the allocation part of local_insert for n_ops ops, done ahead (the router calls it
 // before the exchange so nothing device-synchronising runs after its scatter)
 dg_status prepare_insert(dg_graph g, uint64_t n_ops, cudaStream_t s);

@@ -39,7 +39,12 @@ struct EdgeBatch {
   u32* pub;              // insert, uniform layouts: when set, the last block of k_edges
                          // does the allocator fixup and publishes to pub (small batches:
                          // one launch instead of two)
+  u32 fuse_validate;     // insert / delete of a small batch (one pass of the grid): the
+                         // kernel validates the batch itself (k_validate's job) before a
+                         // grid barrier, instead of a separate launch
 };
+// largest batch (ops) whose insert / delete validates inside the probe launch
+constexpr u64 kFuseValidateMaxOps = 1ull << 18;
 
 // `lay` = DG_LAYA(G, S, A): G 16-B units per bucket, S = 1 for the set variant, A = 1
 // for the degree-adaptive layout (G = 8 lanes, size class per bucket id)

@@ -522,10 +522,53 @@ struct MinBlocks {
 // the allocator fixup of k_fixup by ONE block (the last of k_edges, small batches)
 __device__ __forceinline__ void fixup_block(const Tables& t, u32* pub, u32 epoch);
 
+// Software grid barrier (every block of the launch is resident: launch_g caps the grid
+// at the occupancy bound): arrivals on ctl->bar_count, the last arrival bumps the
+// generation.  A barrier that is not complete after ~4 s traps (a CUDA error that
+// makes the handle sticky-bad) instead of hanging.
+__device__ __forceinline__ void grid_barrier(DevCtl* c) {
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    volatile u32* gen = &c->bar_gen;
+    const u32 g0 = *gen;
+    __threadfence();
+    if (atomicAdd(&c->bar_count, 1u) == gridDim.x - 1) {
+      c->bar_count = 0;
+      __threadfence();
+      atomicAdd(&c->bar_gen, 1u);
+    } else {
+      const long long t0 = clock64();
+      while (*gen == g0) {
+        __nanosleep(64);
+        if (clock64() - t0 > (8ll << 30)) __trap();
+      }
+    }
+    __threadfence();
+  }
+  __syncthreads();
+}
+
+// Fused validation of a small mutating batch (Q7, k_validate's job): every block
+// checks a share of the batch, then a grid barrier, so no block mutates before the
+// whole batch is known to be in range.
+__device__ __forceinline__ void fused_validate(const EdgeBatch& a, DevCtl* c) {
+  bool bad = false;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < a.n; i += stride)
+    bad |= ((u64)a.src[i] >= a.nv) | ((u64)a.dst[i] >= a.nv);
+  if (__syncthreads_or(bad) && threadIdx.x == 0) atomicMax(&c->fail_epoch, a.epoch);
+  if (blockIdx.x == 0 && threadIdx.x == 0) {  // (no block adds to them before the barrier)
+    c->count = 0;
+    c->retry_count = 0;
+  }
+  grid_barrier(c);
+}
+
 template <int G, int S, int OP, bool A>
 __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t, EdgeBatch a) {
   constexpr u32 FULL = 0xFFFFFFFFu;
   const Group<Lanes<G, OP>::L> g;
+  if (OP != OP_QUERY && a.fuse_validate) fused_validate(a, t.ctl);
   bool skip = false;
   if (OP != OP_QUERY) {
     if (ld_relaxed_u32(&t.ctl->fail_epoch) == a.epoch) skip = true;  // batch rejected (Q7)
