@@ -644,9 +644,9 @@ def run_ours(args, cfg):
                 "peak_source": peak_src,
                 "kernel_share_of_step": kmsl[dom] / total_ms if total_ms else None}
     # context beside the copy peak: the measured random-op ceiling of this GPU for the
-    # dominant op's access pattern (tools/gather_ceiling.cu, profiles/r01/gather_ceiling.json):
+    # dominant op's access pattern (tools/gather_ceiling.cu, profiles/r02/gather_ceiling.json):
     # insert/delete = 128-B gather + CAS + counter atomic, query = 128-B gather
-    cpath = os.path.join(ROOT, "profiles", "r01", "gather_ceiling.json")
+    cpath = os.path.join(ROOT, "profiles", "r02", "gather_ceiling.json")
     if os.path.exists(cpath) and S == 128:
         try:
             cj = json.load(open(cpath))["G_ops_s_S128"]
@@ -656,7 +656,7 @@ def run_ours(args, cfg):
                 "pattern": "128-B gather" if dk == "query" else "128-B gather + 64-bit CAS + counter atomic",
                 "G_ops_s": ceil, "achieved_G_ops_s": gops,
                 "frac": gops / ceil if ceil else None,
-                "source": "tools/gather_ceiling.cu (profiles/r01/gather_ceiling.json)"}
+                "source": "tools/gather_ceiling.cu (profiles/r02/gather_ceiling.json)"}
         except (ValueError, KeyError):
             pass
     ops = {}

@@ -3,7 +3,7 @@
 D=gpurun_out/ncu_r2; mkdir -p $D
 timeout 900 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file $D/launches_bench_cfg2.csv \
    python bench.py --steps 3 --warmup 3 --no-e2e --no-cpu-baseline > $D/launches.log 2>&1; echo launches rc=$?
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:"k_edges|k_insert_sorted" -c 12 \
+timeout 900 ncu --set full --clock-control none --import-source on -k regex:"k_edges|k_insert_sorted|k_order|k_validate" -c 24 \
    -o $D/cfg2 -f python tools/prof_cfg.py --config cfg2 > $D/cfg2.log 2>&1; echo cfg2 rc=$?
 timeout 900 ncu --set full --clock-control none --import-source on -k regex:"k_edges" -c 8 \
    -o $D/cfg3 -f python tools/prof_cfg.py --config cfg3 --no-sorted > $D/cfg3.log 2>&1; echo cfg3 rc=$?
