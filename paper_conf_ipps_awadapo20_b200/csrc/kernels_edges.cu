@@ -50,6 +50,12 @@ enum { OP_INSERT = 0, OP_DELETE = 1, OP_QUERY = 2 };
 #ifndef DG_SLOT_WALK
 #define DG_SLOT_WALK 1
 #endif
+// Speculative chain-0 probe in the MAIN round, bit OP (insert 1, delete 2, query 4):
+// measured slower on B200 (profiles/r02/ab/spec/: cfg2 query 0.633 -> 0.837 ms, insert
+// 1.21 -> 1.34 ms; cfg3, where every key is in chain 0, 0.577 -> 0.587 ms): off
+#ifndef DG_SPEC_HOME
+#define DG_SPEC_HOME 0
+#endif
 #ifndef DG_SLOT_WALK_ONCE
 #define DG_SLOT_WALK_ONCE 1
 #endif
@@ -241,9 +247,17 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
   const u32 row = (t.nranks == 1) ? u : u / t.nranks;
   u32 head = 0;
   u32 nbase = 0;
+  // MAIN round, uniform layouts: speculate that the key hashes to chain 0 — the home
+  // bucket's loads go out together with the chain-count byte's instead of after it;
+  // an op whose key hashes to another chain is deferred to the backlog
+  constexpr bool SPEC = MAIN && !A && ((DG_SPEC_HOME >> OP) & 1);
+  u32 nbb_spec = 0;
   if (pend) {
     // base/nb never change during an edge phase; only deg is written (atomics)
-    if constexpr (A) {
+    if constexpr (SPEC) {
+      nbb_spec = __ldg(t.nbs + row);
+      head = kHomeBit | row;
+    } else if constexpr (A) {
       const uint2 de = (OP == OP_QUERY) ? ld_nc_dir(t.dir + row) : ld_dir(t.dir + row);
       head = de.x + bucket_of(v, de.y);
       nbase = de.y;
@@ -289,12 +303,19 @@ __device__ __forceinline__ bool run_ops(const Tables& t, const EdgeBatch& a,
         else q[r][c] = make_uint4(kEmpty, kEmpty, kEmpty, kEmpty);
       }
     }
+    // the ops decided this round (speculation: those whose key hashes to chain 0)
+    u32 pmd = pm;
+    if constexpr (SPEC) {
+      const bool ok = !pend || (nbb_spec < 255u && bucket_of(v, nbb_spec) == 0u);
+      pmd = pm & __ballot_sync(FULL, ok);
+      nbase = nbb_spec;
+    }
     // b. decide: each lane scans its 2K slots in order, the group combines by ballot
     int act = ACT_NONE;
 #pragma unroll
     for (int r = 0; r < L; ++r) {
       const u32 srcl = g.base + r;
-      const bool pr = (pm >> srcl) & 1u;
+      const bool pr = (pmd >> srcl) & 1u;
       const u32 vr = __shfl_sync(FULL, v, srcl);
       const u32 cr = __shfl_sync(FULL, cur, srcl);
       const u32 units = units_of<G, A>(cr);
