@@ -1431,10 +1431,23 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   u32* oadj = reinterpret_cast<u32*>(g->tc[4].p);
   u32* oend = reinterpret_cast<u32*>(g->tc[5].p);
   DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, big, g->sms, s));
-  // (3) one edgeExist per wedge
+  // (3) probe order: entries sorted by the probed vertex (kernels_tc.cu; off unless
+  // DG_TC_ORDER=1: measured on cfg5 it cuts the wedge kernel's DRAM reads 380 -> 52 GB
+  // but mixes entries of very different candidate counts in a warp, 64 -> 150 G
+  // instructions, 111 -> 237 ms)
+  const u32* perm = nullptr;
+  static const bool tc_order = std::getenv("DG_TC_ORDER") != nullptr &&
+                               std::atoi(std::getenv("DG_TC_ORDER")) != 0;
+  if (tc_order) {
+    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8));
+    DG_CK(ensure_buf(g->tc[7], mo * 8 + 8));
+    DG_CK(dg::launch_tc_probe_order(oadj, mo, rows, (u32*)g->tc[6].p, (u32*)g->tc[7].p, &perm,
+                                    &g->scan_temp, &g->scan_bytes, s));
+  }
+  // (4) one edgeExist per wedge
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);
-  DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, mo,
+  DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, perm, mo,
                              reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
   dg::prof_mark(g, dg::PROF_TC, s);
   DG_TRY(read_ctl(g, s));

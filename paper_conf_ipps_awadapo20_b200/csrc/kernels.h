@@ -149,7 +149,11 @@ cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* ds
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
                                   u32 nparts, const u64* oro, u32* oadj, u32* oend,
                                   const u32* big, int sms, cudaStream_t s);
-cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
+cudaError_t launch_tc_probe_order(const u32* oadj, u64 n_units, u64 rows, u32* keys, u32* vals,
+                                  const u32** perm, void** temp, size_t* temp_bytes,
+                                  cudaStream_t s);
+cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend,
+                             const u32* perm, u64 n_units,
                              unsigned long long* count, int sms, cudaStream_t s);
 
 // per-vertex re-sizing of long-chained tables (kernels_rehash.cu)

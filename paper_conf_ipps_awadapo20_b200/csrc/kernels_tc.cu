@@ -15,6 +15,8 @@
 //   k_tc_wedges       : one thread per oriented entry e = (u, i): probe the hash
 //                       table of v_i for every later v_j of N+(u); whole buckets
 //                       are read with 16-B loads, hits reduced per warp.
+#include <cub/device/device_radix_sort.cuh>
+
 #include "dg_common.cuh"
 #include "kernels.h"
 
@@ -150,9 +152,18 @@ __global__ void __launch_bounds__(256) k_tc_orient_fill_big(const u64* ro, const
 // 16-B load per lane per candidate), then decides all G with group ballots.  Warp
 // loops are warp-uniform so every intrinsic uses the full mask.  The rare probes
 // whose key may sit further down a chain are walked by their own lane.
+__global__ void k_iota(u32* out, u64 n) {
+  for (u64 i = (u64)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (u64)gridDim.x * blockDim.x)
+    out[i] = (u32)i;
+}
+
+// perm (nullable): the entries in probe order — sorted by the probed vertex v, so the
+// probes into one table A_v run close together in time and its buckets are read from
+// DRAM about once instead of once per probe (launch_tc_probe_order)
 template <int G, int S, bool A>
 __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __restrict__ oadj,
-                                                      const u32* __restrict__ oend, u64 n_units,
+                                                      const u32* __restrict__ oend,
+                                                      const u32* __restrict__ perm, u64 n_units,
                                                       unsigned long long* count) {
   typedef Lay<G, S> LY;
   typedef Geo<G, S, A> GEO;
@@ -164,8 +175,9 @@ __global__ void __launch_bounds__(256, 4) k_tc_wedges(Tables t, const u32* __res
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
   for (u64 e0 = warp * PER_WARP; e0 < n_units; e0 += nwarps * PER_WARP) {
-    const u64 e = e0 + g.lane / G;                // this group's entry
-    const bool ev = e < n_units;
+    const u64 ei = e0 + g.lane / G;               // this group's entry
+    const bool ev = ei < n_units;
+    const u64 e = (perm && ev) ? (u64)__ldg(perm + ei) : ei;
     const u32 v = ev ? __ldg(oadj + e) : 0u;
     const u32 ncand = ev ? __ldg(oend + e) - (u32)e - 1u : 0u;
     const uint2 dv = ev ? ld_nc_dir(t.dir + v) : make_uint2(0, 1);
@@ -264,8 +276,39 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
   return cudaGetLastError();
 }
 
-cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend, u64 n_units,
-                             unsigned long long* count, int sms, cudaStream_t s) {
+// Probe order of the wedge kernel: the oriented entries sorted by their probed vertex
+// oadj[e] (CUB radix sort of (v, e) pairs over the bits of the row count).  keys /
+// vals: 2 x n_units u32 each (double buffers); returns the sorted entry ids in *perm.
+cudaError_t launch_tc_probe_order(const u32* oadj, u64 n_units, u64 rows, u32* keys, u32* vals,
+                                  const u32** perm, void** temp, size_t* temp_bytes,
+                                  cudaStream_t s) {
+  if (n_units == 0 || n_units >= (1ull << 31)) { *perm = nullptr; return cudaSuccess; }
+  const int n = (int)n_units;
+  int bits = 1;
+  while (bits < 32 && (1ull << bits) < rows) ++bits;
+  cudaError_t e = cudaMemcpyAsync(keys, oadj, n_units * 4, cudaMemcpyDeviceToDevice, s);
+  if (e != cudaSuccess) return e;
+  k_iota<<<(unsigned)((n_units + 255) / 256 < 65535 ? (n_units + 255) / 256 : 65535), 256, 0, s>>>(vals, n_units);
+  cub::DoubleBuffer<u32> kb(keys, keys + n_units), vb(vals, vals + n_units);
+  size_t need = 0;
+  e = cub::DeviceRadixSort::SortPairs(nullptr, need, kb, vb, n, 0, bits, s);
+  if (e != cudaSuccess) return e;
+  if (need > *temp_bytes) {
+    if (*temp) cudaFree(*temp);
+    *temp = nullptr;
+    *temp_bytes = 0;
+    if ((e = cudaMalloc(temp, need)) != cudaSuccess) return e;
+    *temp_bytes = need;
+  }
+  e = cub::DeviceRadixSort::SortPairs(*temp, need, kb, vb, n, 0, bits, s);
+  note_kernel(2);
+  *perm = vb.Current();
+  return e;
+}
+
+cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u32* oend,
+                             const u32* perm, u64 n_units, unsigned long long* count, int sms,
+                             cudaStream_t s) {
   if (n_units == 0) return cudaSuccess;
   const int G = lay & 31;
   u64 blocks = (n_units * G + 255) / 256;
@@ -273,7 +316,7 @@ cudaError_t launch_tc_wedges(int lay, const Tables& t, const u32* oadj, const u3
   switch (lay) {
 #define DG_CASE(G_, S_, A_)                                                                 \
   case DG_LAYA(G_, S_, A_):                                                                 \
-    k_tc_wedges<G_, S_, A_><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, n_units, count); \
+    k_tc_wedges<G_, S_, A_><<<(unsigned)blocks, 256, 0, s>>>(t, oadj, oend, perm, n_units, count); \
     break;
     DG_FOR_LAYOUTS_A(DG_CASE)
 #undef DG_CASE
