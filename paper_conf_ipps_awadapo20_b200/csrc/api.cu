@@ -1444,11 +1444,34 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
     DG_CK(dg::launch_tc_probe_order(oadj, mo, rows, (u32*)g->tc[6].p, (u32*)g->tc[7].p, &perm,
                                     &g->scan_temp, &g->scan_bytes, s));
   }
-  // (4) one edgeExist per wedge
+  // (4) one edgeExist per wedge: uniform layouts number the wedges and give every lane
+  // one (k_tc_wedges_flat, DG_TC_FLAT=0: the per-entry kernel); the adaptive layout
+  // keeps the per-entry kernel
+  static const bool tc_flat = std::getenv("DG_TC_FLAT") == nullptr ||
+                              std::atoi(std::getenv("DG_TC_FLAT")) != 0;
+  const bool flat = tc_flat && !g->adaptive && mo < (1ull << 31);
+  u32* list = nullptr;
+  u64* woff = nullptr;
+  unsigned long long* nlist_dev = nullptr;
+  if (flat) {
+    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8));  // (shared with the probe order's keys)
+    DG_CK(ensure_buf(g->tc[8], mo * 4 + 4));
+    DG_CK(ensure_buf(g->tc[9], mo * 8 + 16));
+    list = (u32*)g->tc[8].p;
+    woff = (u64*)g->tc[9].p;
+    nlist_dev = (unsigned long long*)((char*)g->tc[6].p + mo * 8);
+    u64 nl = 0;
+    DG_CK(dg::launch_tc_flat_prepare(oend, perm, mo, list, woff, nlist_dev, &nl, &g->scan_temp,
+                                     &g->scan_bytes, s));
+  }
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);
-  DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, perm, mo,
-                             reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
+  if (flat)
+    DG_CK(dg::launch_tc_wedges_flat(g->lay, t, oadj, list, woff, nlist_dev,
+                                    reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
+  else
+    DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, perm, mo,
+                               reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
   dg::prof_mark(g, dg::PROF_TC, s);
   DG_TRY(read_ctl(g, s));
   *count = g->hctl->count;

@@ -16,6 +16,10 @@
 //                       table of v_i for every later v_j of N+(u); whole buckets
 //                       are read with 16-B loads, hits reduced per warp.
 #include <cub/device/device_radix_sort.cuh>
+#include <cub/device/device_scan.cuh>
+#include <cub/device/device_select.cuh>
+#include <thrust/iterator/counting_iterator.h>
+#include <thrust/iterator/transform_iterator.h>
 
 #include "dg_common.cuh"
 #include "kernels.h"
@@ -273,6 +277,172 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
                                                      oend);
   k_tc_orient_fill_big<<<(unsigned)sms * 2, 256, 0, s>>>(ro, dst, t.deg, oro, oadj, oend, big);
   note_kernel(2);
+  return cudaGetLastError();
+}
+
+// ---------------------------------------------------------- flat wedges ----
+// Load-balanced form of the wedge probes: the wedges of all entries with at least one
+// candidate are numbered 0 .. W-1 in entry order (woff = exclusive scan of the entries'
+// candidate counts over the compacted entry list `list`), every warp takes one
+// contiguous range of W / warps wedges and every LANE probes one wedge: w = the
+// candidate, A_v its entry's table, the lane reading the whole bucket with 16-B loads.
+// No warp waits on its longest entry (the per-entry kernel above runs each warp to the
+// largest candidate count of its 32 / G entries) and there is no per-entry setup.
+// Lanes find their entry with one load per lane: lane j reads the start of entry
+// k0 + 1 + j; the bits of the starts that fall inside the 32-wedge window give every
+// lane its entry by a popcount (entries are non-empty, so starts are distinct).
+template <int G, int S>
+__global__ void __launch_bounds__(256) k_tc_wedges_flat(Tables t, const u32* __restrict__ oadj,
+                                                        const u32* __restrict__ list,
+                                                        const u64* __restrict__ woff,
+                                                        const unsigned long long* n_list_dev,
+                                                        unsigned long long* count) {
+  typedef Lay<G, S> LY;
+  typedef Geo<G, S, false> GEO;
+  constexpr u32 FULL = 0xFFFFFFFFu;
+  const u64 n_list = *n_list_dev;
+  if (n_list == 0) return;
+  const u64 W = woff[n_list];
+  const u32 lane = threadIdx.x & 31u;
+  const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+  const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
+  // this warp's wedges [x_lo, x_hi), in whole 32-wedge windows
+  const u64 per = ((W + nwarps - 1) / nwarps + 31) & ~31ull;
+  const u64 x_lo = warp * per;
+  const u64 x_hi = x_lo + per < W ? x_lo + per : W;
+  if (x_lo >= x_hi) return;
+  // k0: the entry holding wedge x_lo (largest k with woff[k] <= x_lo), one search per warp
+  u64 k0 = 0;
+  if (lane == 0) {
+    u64 lo = 0, hi = n_list;
+    while (hi - lo > 1) {
+      const u64 mid = (lo + hi) >> 1;
+      if (woff[mid] <= x_lo) lo = mid;
+      else hi = mid;
+    }
+    k0 = lo;
+  }
+  k0 = __shfl_sync(FULL, k0, 0);
+  u32 hits = 0;
+  for (u64 x0 = x_lo; x0 < x_hi; x0 += 32) {
+    const u64 kj = k0 + 1 + lane;
+    u32 bit = 0;
+    if (kj < n_list) {
+      const u64 sj = woff[kj] - x0;
+      if (sj < 32) bit = 1u << sj;
+    }
+    const u32 M = __reduce_or_sync(FULL, bit);
+    const u64 x = x0 + lane;
+    const u64 k = k0 + __popc(M & (lane == 31 ? FULL : ((2u << lane) - 1u)));
+    if (x < x_hi) {
+      const u32 e = __ldg(list + k);
+      const u64 c = x - woff[k];
+      const u32 v = __ldg(oadj + e);
+      const u32 w = __ldg(oadj + e + 1 + c);
+      const uint2 dv = ld_nc_dir(t.dir + v);
+      u32 b = chain_head<false>(dv.x, v, bucket_of(w, dv.y));
+      // edgeExist: the chain of A_v that w hashes to
+      while (b != kNil) {
+        const uint4* bp = reinterpret_cast<const uint4*>(GEO(t, b).p);
+        uint4 y[G];
+#pragma unroll
+        for (int c2 = 0; c2 < G; ++c2) y[c2] = __ldg(bp + c2);
+        bool found = false, ended = false;
+#pragma unroll
+        for (int c2 = 0; c2 < G; ++c2) {
+#pragma unroll
+          for (int j = 0; j < LY::SPU; ++j) {
+            if (!LY::has(c2, j)) continue;
+            found |= LY::key(y[c2], j) == w;
+            ended |= LY::key(y[c2], j) == kEmpty;
+          }
+        }
+        if (found) { ++hits; break; }
+        if (ended) break;
+        b = y[G - 1].z;
+      }
+    }
+    // the entry holding the next window's first wedge
+    k0 += __popc(M);
+    if (k0 + 1 < n_list && woff[k0 + 1] <= x0 + 32) ++k0;  // (an entry starting at x0 + 32)
+  }
+  const u32 tot = __reduce_add_sync(FULL, hits);
+  if (lane == 0 && tot) atomicAdd(count, (unsigned long long)tot);
+}
+
+namespace {
+struct HasCand {  // entry e of the oriented lists has at least one later candidate
+  const u32* oend;
+  __host__ __device__ bool operator()(u32 e) const { return oend[e] > e + 1; }
+};
+struct CandOf {  // candidates of the k-th listed entry
+  const u32* oend;
+  const u32* list;
+  u64 n;
+  __host__ __device__ u64 operator()(u64 k) const {
+    return k < n ? (u64)(oend[list[k]] - list[k] - 1) : 0ull;
+  }
+};
+}  // namespace
+
+// list: entries with >= 1 candidate, in `order` (nullable: entry order); woff: their
+// wedge offsets (n_list + 1); n_list_dev / *n_list: their number.  Synchronises s.
+cudaError_t launch_tc_flat_prepare(const u32* oend, const u32* order, u64 n_units, u32* list,
+                                   u64* woff, unsigned long long* n_list_dev, u64* n_list,
+                                   void** temp, size_t* temp_bytes, cudaStream_t s) {
+  *n_list = 0;
+  if (n_units == 0 || n_units >= (1ull << 31)) return cudaSuccess;
+  const int n = (int)n_units;
+  size_t need = 0;
+  cudaError_t e;
+  auto grow = [&](size_t want) -> cudaError_t {
+    if (want <= *temp_bytes) return cudaSuccess;
+    if (*temp) cudaFree(*temp);
+    *temp = nullptr;
+    *temp_bytes = 0;
+    cudaError_t r = cudaMalloc(temp, want);
+    if (r == cudaSuccess) *temp_bytes = want;
+    return r;
+  };
+  if (order) {
+    e = cub::DeviceSelect::If(nullptr, need, order, list, n_list_dev, n, HasCand{oend}, s);
+    if (e != cudaSuccess || (e = grow(need)) != cudaSuccess) return e;
+    e = cub::DeviceSelect::If(*temp, need, order, list, n_list_dev, n, HasCand{oend}, s);
+  } else {
+    thrust::counting_iterator<u32> it(0);
+    e = cub::DeviceSelect::If(nullptr, need, it, list, n_list_dev, n, HasCand{oend}, s);
+    if (e != cudaSuccess || (e = grow(need)) != cudaSuccess) return e;
+    e = cub::DeviceSelect::If(*temp, need, it, list, n_list_dev, n, HasCand{oend}, s);
+  }
+  if (e != cudaSuccess) return e;
+  unsigned long long nl = 0;
+  if ((e = cudaMemcpyAsync(&nl, n_list_dev, 8, cudaMemcpyDeviceToHost, s)) != cudaSuccess) return e;
+  if ((e = cudaStreamSynchronize(s)) != cudaSuccess) return e;
+  *n_list = nl;
+  auto it = thrust::make_transform_iterator(thrust::counting_iterator<u64>(0),
+                                            CandOf{oend, list, (u64)nl});
+  need = 0;
+  e = cub::DeviceScan::ExclusiveSum(nullptr, need, it, woff, (int64_t)(nl + 1), s);
+  if (e != cudaSuccess || (e = grow(need)) != cudaSuccess) return e;
+  e = cub::DeviceScan::ExclusiveSum(*temp, need, it, woff, (int64_t)(nl + 1), s);
+  note_kernel(3);
+  return e;
+}
+
+cudaError_t launch_tc_wedges_flat(int lay, const Tables& t, const u32* oadj, const u32* list,
+                                  const u64* woff, const unsigned long long* n_list_dev,
+                                  unsigned long long* count, int sms, cudaStream_t s) {
+  switch (lay) {
+#define DG_CASE(G_, S_)                                                                     \
+  case DG_LAY(G_, S_):                                                                      \
+    k_tc_wedges_flat<G_, S_><<<(unsigned)sms * 8, 256, 0, s>>>(t, oadj, list, woff,          \
+                                                             n_list_dev, count);           \
+    break;
+    DG_FOR_LAYOUTS(DG_CASE)
+#undef DG_CASE
+    default: return cudaErrorInvalidValue;
+  }
+  note_kernel(1);
   return cudaGetLastError();
 }
 
