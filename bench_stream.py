@@ -285,7 +285,7 @@ def run_tc(args, cfg):
     Sb = S or st_["table_bytes"] / max(1, st_["base_buckets"] + st_["overflow_buckets"])
     bytes_per_probe = Sb + 4
     # wk covers the nl timed launches (one per step); their probes are sum(wedges)
-    roofline = {"bound": "hbm", "kernel": f"k_tc_wedges<{S // 16 if S else 'adaptive'},{variant}>",
+    roofline = {"bound": "hbm", "kernel": (f"k_tc_wedges_flat<{S // 16},{variant}>" if S else "k_tc_wedges<adaptive,{variant}>"),
                 "unit": "GB/s",
                 "achieved": sum(wedges) / world * bytes_per_probe / (wk * 1e-3) / 1e9,
                 "peak": peak, "peak_source": peak_src, "traffic": None,

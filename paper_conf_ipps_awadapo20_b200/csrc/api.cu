@@ -1450,24 +1450,30 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   static const bool tc_flat = std::getenv("DG_TC_FLAT") == nullptr ||
                               std::atoi(std::getenv("DG_TC_FLAT")) != 0;
   const bool flat = tc_flat && !g->adaptive && mo < (1ull << 31);
-  u32* list = nullptr;
+  uint2* list = nullptr;
   u64* woff = nullptr;
+  u32* chunk_k = nullptr;
   unsigned long long* nlist_dev = nullptr;
   if (flat) {
     DG_CK(ensure_buf(g->tc[6], mo * 8 + 8));  // (shared with the probe order's keys)
-    DG_CK(ensure_buf(g->tc[8], mo * 4 + 4));
+    DG_CK(ensure_buf(g->tc[8], mo * 8 + 8));
     DG_CK(ensure_buf(g->tc[9], mo * 8 + 16));
-    list = (u32*)g->tc[8].p;
+    list = (uint2*)g->tc[8].p;
     woff = (u64*)g->tc[9].p;
     nlist_dev = (unsigned long long*)((char*)g->tc[6].p + mo * 8);
     u64 nl = 0;
-    DG_CK(dg::launch_tc_flat_prepare(oend, perm, mo, list, woff, nlist_dev, &nl, &g->scan_temp,
+    DG_CK(dg::launch_tc_flat_prepare(oadj, oend, perm, mo, list, woff, nlist_dev, &nl, &g->scan_temp,
                                      &g->scan_bytes, s));
+    u64 wedges = 0;  // (sizes the chunk table)
+    DG_CK(cudaMemcpyAsync(&wedges, woff + nl, 8, cudaMemcpyDeviceToHost, s));
+    DG_CK(cudaStreamSynchronize(s));
+    DG_CK(ensure_buf(g->tc[10], dg::tc_chunk_count(wedges) * 4 + 4));
+    chunk_k = (u32*)g->tc[10].p;
   }
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);
   if (flat)
-    DG_CK(dg::launch_tc_wedges_flat(g->lay, t, oadj, list, woff, nlist_dev,
+    DG_CK(dg::launch_tc_wedges_flat(g->lay, t, oadj, list, woff, chunk_k, nlist_dev,
                                     reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
   else
     DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, perm, mo,

@@ -149,11 +149,13 @@ cudaError_t launch_tc_orient_count(const Tables& t, const u64* ro, const u32* ds
 cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst, u32 part,
                                   u32 nparts, const u64* oro, u32* oadj, u32* oend,
                                   const u32* big, int sms, cudaStream_t s);
-cudaError_t launch_tc_flat_prepare(const u32* oend, const u32* order, u64 n_units, u32* list,
-                                   u64* woff, unsigned long long* n_list_dev, u64* n_list,
-                                   void** temp, size_t* temp_bytes, cudaStream_t s);
-cudaError_t launch_tc_wedges_flat(int lay, const Tables& t, const u32* oadj, const u32* list,
-                                  const u64* woff, const unsigned long long* n_list_dev,
+cudaError_t launch_tc_flat_prepare(const u32* oadj, const u32* oend, const u32* order, u64 n_units,
+                                   uint2* list, u64* woff, unsigned long long* n_list_dev,
+                                   u64* n_list, void** temp, size_t* temp_bytes, cudaStream_t s);
+u64 tc_chunk_count(u64 wedges);
+cudaError_t launch_tc_wedges_flat(int lay, const Tables& t, const u32* oadj, const uint2* list,
+                                  const u64* woff, u32* chunk_k,
+                                  const unsigned long long* n_list_dev,
                                   unsigned long long* count, int sms, cudaStream_t s);
 cudaError_t launch_tc_probe_order(const u32* oadj, u64 n_units, u64 rows, u32* keys, u32* vals,
                                   const u32** perm, void** temp, size_t* temp_bytes,

@@ -283,18 +283,37 @@ cudaError_t launch_tc_orient_fill(const Tables& t, const u64* ro, const u32* dst
 // ---------------------------------------------------------- flat wedges ----
 // Load-balanced form of the wedge probes: the wedges of all entries with at least one
 // candidate are numbered 0 .. W-1 in entry order (woff = exclusive scan of the entries'
-// candidate counts over the compacted entry list `list`), every warp takes one
-// contiguous range of W / warps wedges and every LANE probes one wedge: w = the
-// candidate, A_v its entry's table, the lane reading the whole bucket with 16-B loads.
-// No warp waits on its longest entry (the per-entry kernel above runs each warp to the
-// largest candidate count of its 32 / G entries) and there is no per-entry setup.
-// Lanes find their entry with one load per lane: lane j reads the start of entry
-// k0 + 1 + j; the bits of the starts that fall inside the 32-wedge window give every
-// lane its entry by a popcount (entries are non-empty, so starts are distinct).
+// candidate counts over the compacted entry list `list` of (entry, probed vertex v)
+// pairs), split into chunks of kTcChunk wedges taken grid-stride by the warps (so the
+// warps work on neighbouring wedges at any moment: with the probe order the tables
+// they probe are the same few), and every LANE probes one wedge: w = the candidate,
+// A_v its entry's table, the lane reading the whole bucket with 16-B loads.  No warp waits on its longest entry (the per-entry
+// kernel above runs each warp to the largest candidate count of its 32 / G entries)
+// and there is no per-entry setup.
+// Entry of each lane: lane j reads the start of entry k0 + 1 + j; the starts inside
+// the 32-wedge window (and one at its end, bit 32) form a mask whose popcounts give
+// every lane its entry and whose highest set bit its entry's start (entries are
+// non-empty, so starts are distinct).  The next window's starts are loaded before the
+// current window's probes run.
+constexpr u32 kTcChunk = 256;  // wedges per chunk (8 windows of 32)
+
+// chunk_k[c] = the entry holding wedge c * kTcChunk (every entry writes the chunks
+// whose first wedge it holds)
+__global__ void k_tc_chunk_entries(const u64* __restrict__ woff,
+                                   const unsigned long long* n_list_dev, u32* chunk_k) {
+  const u64 n_list = *n_list_dev;
+  const u64 stride = (u64)gridDim.x * blockDim.x;
+  for (u64 k = (u64)blockIdx.x * blockDim.x + threadIdx.x; k < n_list; k += stride) {
+    const u64 a = woff[k], b = woff[k + 1];
+    for (u64 c = (a + kTcChunk - 1) / kTcChunk; c * kTcChunk < b; ++c) chunk_k[c] = (u32)k;
+  }
+}
+
 template <int G, int S>
 __global__ void __launch_bounds__(256) k_tc_wedges_flat(Tables t, const u32* __restrict__ oadj,
-                                                        const u32* __restrict__ list,
+                                                        const uint2* __restrict__ list,
                                                         const u64* __restrict__ woff,
+                                                        const u32* __restrict__ chunk_k,
                                                         const unsigned long long* n_list_dev,
                                                         unsigned long long* count) {
   typedef Lay<G, S> LY;
@@ -306,90 +325,101 @@ __global__ void __launch_bounds__(256) k_tc_wedges_flat(Tables t, const u32* __r
   const u32 lane = threadIdx.x & 31u;
   const u64 warp = ((u64)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
   const u64 nwarps = ((u64)gridDim.x * blockDim.x) >> 5;
-  // this warp's wedges [x_lo, x_hi), in whole 32-wedge windows
-  const u64 per = ((W + nwarps - 1) / nwarps + 31) & ~31ull;
-  const u64 x_lo = warp * per;
-  const u64 x_hi = x_lo + per < W ? x_lo + per : W;
-  if (x_lo >= x_hi) return;
-  // k0: the entry holding wedge x_lo (largest k with woff[k] <= x_lo), one search per warp
-  u64 k0 = 0;
-  if (lane == 0) {
-    u64 lo = 0, hi = n_list;
-    while (hi - lo > 1) {
-      const u64 mid = (lo + hi) >> 1;
-      if (woff[mid] <= x_lo) lo = mid;
-      else hi = mid;
-    }
-    k0 = lo;
-  }
-  k0 = __shfl_sync(FULL, k0, 0);
+  const u64 nchunks = (W + kTcChunk - 1) / kTcChunk;
   u32 hits = 0;
-  for (u64 x0 = x_lo; x0 < x_hi; x0 += 32) {
-    const u64 kj = k0 + 1 + lane;
-    u32 bit = 0;
+  for (u64 ch = warp; ch < nchunks; ch += nwarps) {
+  // this chunk's wedges [x_lo, x_hi) in 32-wedge windows; k0 holds x_lo, s0 its start
+  const u64 x_lo = ch * kTcChunk;
+  const u64 x_hi = x_lo + kTcChunk < W ? x_lo + kTcChunk : W;
+  u64 k0 = __ldg(chunk_k + ch);
+  u64 s0 = woff[k0];
+  const u32 upto = lane == 31 ? FULL : ((2u << lane) - 1u);
+  // starts of entries k0+1 .. k0+32 relative to x0: bits 0..31 (lo) and bit 32 (hi)
+  auto window = [&](u64 k0w, u64 x0, u32& mlo, u32& mhi) {
+    const u64 kj = k0w + 1 + lane;
+    u64 bit = 0;
     if (kj < n_list) {
       const u64 sj = woff[kj] - x0;
-      if (sj < 32) bit = 1u << sj;
+      if (sj <= 32) bit = 1ull << sj;
     }
-    const u32 M = __reduce_or_sync(FULL, bit);
+    mlo = __reduce_or_sync(FULL, (u32)bit);
+    mhi = __reduce_or_sync(FULL, (u32)(bit >> 32));
+  };
+  u32 mlo, mhi;
+  window(k0, x_lo, mlo, mhi);
+  for (u64 x0 = x_lo; x0 < x_hi; x0 += 32) {
     const u64 x = x0 + lane;
-    const u64 k = k0 + __popc(M & (lane == 31 ? FULL : ((2u << lane) - 1u)));
+    const u32 mine = mlo & upto;
+    const u64 k = k0 + __popc(mine);
+    const u64 start = mine ? x0 + 31 - __clz(mine) : s0;
+    // the next window: entry, start, and its starts' loads in flight during the probes
+    const u64 k0n = k0 + __popc(mlo) + (mhi & 1u);
+    const u64 s0n = (mhi & 1u) ? x0 + 32 : (mlo ? x0 + 31 - __clz(mlo) : s0);
+    u32 nlo = 0, nhi = 0;
+    if (x0 + 32 < x_hi) window(k0n, x0 + 32, nlo, nhi);
     if (x < x_hi) {
-      const u32 e = __ldg(list + k);
-      const u64 c = x - woff[k];
-      const u32 v = __ldg(oadj + e);
-      const u32 w = __ldg(oadj + e + 1 + c);
-      const uint2 dv = ld_nc_dir(t.dir + v);
-      u32 b = chain_head<false>(dv.x, v, bucket_of(w, dv.y));
+      const uint2 ev = __ldg(list + k);  // (entry, probed vertex)
+      const u32 w = __ldg(oadj + ev.x + 1 + (x - start));
+      const uint2 dv = ld_nc_dir(t.dir + ev.y);
+      u32 b = chain_head<false>(dv.x, ev.y, bucket_of(w, dv.y));
       // edgeExist: the chain of A_v that w hashes to
       while (b != kNil) {
         const uint4* bp = reinterpret_cast<const uint4*>(GEO(t, b).p);
         uint4 y[G];
 #pragma unroll
         for (int c2 = 0; c2 < G; ++c2) y[c2] = __ldg(bp + c2);
-        bool found = false, ended = false;
+        bool found = false;
 #pragma unroll
         for (int c2 = 0; c2 < G; ++c2) {
 #pragma unroll
           for (int j = 0; j < LY::SPU; ++j) {
             if (!LY::has(c2, j)) continue;
             found |= LY::key(y[c2], j) == w;
-            ended |= LY::key(y[c2], j) == kEmpty;
           }
         }
         if (found) { ++hits; break; }
-        if (ended) break;
+        // EMPTY slots form the chain's suffix: the chain ends in this
+        // bucket iff its last slot is EMPTY (one compare instead of one per slot)
+        if (LY::key(y[G - 1], LY::SPU / 2 - 1) == kEmpty) break;
         b = y[G - 1].z;
       }
     }
-    // the entry holding the next window's first wedge
-    k0 += __popc(M);
-    if (k0 + 1 < n_list && woff[k0 + 1] <= x0 + 32) ++k0;  // (an entry starting at x0 + 32)
+    k0 = k0n;
+    s0 = s0n;
+    mlo = nlo;
+    mhi = nhi;
+  }
   }
   const u32 tot = __reduce_add_sync(FULL, hits);
   if (lane == 0 && tot) atomicAdd(count, (unsigned long long)tot);
 }
 
 namespace {
-struct HasCand {  // entry e of the oriented lists has at least one later candidate
+struct EntryPair {  // entry e -> (e, probed vertex oadj[e])
+  const u32* oadj;
+  __host__ __device__ uint2 operator()(u32 e) const { return make_uint2(e, oadj[e]); }
+};
+struct HasCand {  // the entry has at least one later candidate
   const u32* oend;
-  __host__ __device__ bool operator()(u32 e) const { return oend[e] > e + 1; }
+  __host__ __device__ bool operator()(const uint2& p) const { return oend[p.x] > p.x + 1; }
 };
 struct CandOf {  // candidates of the k-th listed entry
   const u32* oend;
-  const u32* list;
+  const uint2* list;
   u64 n;
   __host__ __device__ u64 operator()(u64 k) const {
-    return k < n ? (u64)(oend[list[k]] - list[k] - 1) : 0ull;
+    return k < n ? (u64)(oend[list[k].x] - list[k].x - 1) : 0ull;
   }
 };
 }  // namespace
 
+u64 tc_chunk_count(u64 wedges) { return wedges / kTcChunk + 1; }
+
 // list: entries with >= 1 candidate, in `order` (nullable: entry order); woff: their
 // wedge offsets (n_list + 1); n_list_dev / *n_list: their number.  Synchronises s.
-cudaError_t launch_tc_flat_prepare(const u32* oend, const u32* order, u64 n_units, u32* list,
-                                   u64* woff, unsigned long long* n_list_dev, u64* n_list,
-                                   void** temp, size_t* temp_bytes, cudaStream_t s) {
+cudaError_t launch_tc_flat_prepare(const u32* oadj, const u32* oend, const u32* order, u64 n_units,
+                                   uint2* list, u64* woff, unsigned long long* n_list_dev,
+                                   u64* n_list, void** temp, size_t* temp_bytes, cudaStream_t s) {
   *n_list = 0;
   if (n_units == 0 || n_units >= (1ull << 31)) return cudaSuccess;
   const int n = (int)n_units;
@@ -405,14 +435,15 @@ cudaError_t launch_tc_flat_prepare(const u32* oend, const u32* order, u64 n_unit
     return r;
   };
   if (order) {
-    e = cub::DeviceSelect::If(nullptr, need, order, list, n_list_dev, n, HasCand{oend}, s);
+    auto in = thrust::make_transform_iterator(order, EntryPair{oadj});
+    e = cub::DeviceSelect::If(nullptr, need, in, list, n_list_dev, n, HasCand{oend}, s);
     if (e != cudaSuccess || (e = grow(need)) != cudaSuccess) return e;
-    e = cub::DeviceSelect::If(*temp, need, order, list, n_list_dev, n, HasCand{oend}, s);
+    e = cub::DeviceSelect::If(*temp, need, in, list, n_list_dev, n, HasCand{oend}, s);
   } else {
-    thrust::counting_iterator<u32> it(0);
-    e = cub::DeviceSelect::If(nullptr, need, it, list, n_list_dev, n, HasCand{oend}, s);
+    auto in = thrust::make_transform_iterator(thrust::counting_iterator<u32>(0), EntryPair{oadj});
+    e = cub::DeviceSelect::If(nullptr, need, in, list, n_list_dev, n, HasCand{oend}, s);
     if (e != cudaSuccess || (e = grow(need)) != cudaSuccess) return e;
-    e = cub::DeviceSelect::If(*temp, need, it, list, n_list_dev, n, HasCand{oend}, s);
+    e = cub::DeviceSelect::If(*temp, need, in, list, n_list_dev, n, HasCand{oend}, s);
   }
   if (e != cudaSuccess) return e;
   unsigned long long nl = 0;
@@ -429,13 +460,17 @@ cudaError_t launch_tc_flat_prepare(const u32* oend, const u32* order, u64 n_unit
   return e;
 }
 
-cudaError_t launch_tc_wedges_flat(int lay, const Tables& t, const u32* oadj, const u32* list,
-                                  const u64* woff, const unsigned long long* n_list_dev,
+// chunk_k: (total wedges / kTcChunk + 1) u32 (tc_chunk_count)
+cudaError_t launch_tc_wedges_flat(int lay, const Tables& t, const u32* oadj, const uint2* list,
+                                  const u64* woff, u32* chunk_k,
+                                  const unsigned long long* n_list_dev,
                                   unsigned long long* count, int sms, cudaStream_t s) {
+  k_tc_chunk_entries<<<(unsigned)sms * 8, 256, 0, s>>>(woff, n_list_dev, chunk_k);
+  note_kernel(1);
   switch (lay) {
 #define DG_CASE(G_, S_)                                                                     \
   case DG_LAY(G_, S_):                                                                      \
-    k_tc_wedges_flat<G_, S_><<<(unsigned)sms * 8, 256, 0, s>>>(t, oadj, list, woff,          \
+    k_tc_wedges_flat<G_, S_><<<(unsigned)sms * 8, 256, 0, s>>>(t, oadj, list, woff, chunk_k, \
                                                              n_list_dev, count);           \
     break;
     DG_FOR_LAYOUTS(DG_CASE)
