@@ -52,7 +52,14 @@ constexpr u64 kFuseValidateMaxOps = 1ull << 18;
 // edge ops (kernels_edges.cu)
 // locality order of a delete batch (kernels_order.cu): partitions by local row >> shift,
 // at most kMaxOrderParts partitions of 2^shift rows
-constexpr u32 kOrderPartBits = 8;
+// (measured on cfg2 / cfg3 2^24 deletes, profiles/r02/order/partbits.txt: at most
+// 256 / 128 / 64 / 32 partitions -> scatter 122 / 79 us, delete call 0.711 / 0.673 /
+// 0.670 / 0.665 ms on cfg2, 0.772 / 0.714 / 0.702 ms on cfg3; 64 keeps a partition's
+// rows within L2 on cfg3's 24 M rows)
+#ifndef DG_ORDER_PART_BITS
+#define DG_ORDER_PART_BITS 6
+#endif
+constexpr u32 kOrderPartBits = DG_ORDER_PART_BITS;
 constexpr u32 kMaxOrderParts = 256;
 u32 order_shift(u64 rows);
 size_t order_scratch_bytes(int sms);

@@ -40,7 +40,10 @@ namespace dg {
 namespace {
 
 constexpr int kOrdThreads = 256;
-constexpr int kOrdItems = 8;  // ops per thread per step (all loads issued first)
+#ifndef DG_ORDER_ITEMS
+#define DG_ORDER_ITEMS 8
+#endif
+constexpr int kOrdItems = DG_ORDER_ITEMS;  // ops per thread per step (all loads issued first)
 constexpr u32 kOrdStep = kOrdThreads * kOrdItems;
 constexpr int kOrdBlocksPerSm = 4;  // (64 registers: 4 blocks of 256 threads resident)
 constexpr u32 kOrdMaxBlocks = 2048;  // k_order_scan: one column per block, 2 per thread
