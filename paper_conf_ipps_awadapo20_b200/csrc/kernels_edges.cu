@@ -692,8 +692,10 @@ __global__ void __launch_bounds__(kEdgeBlock, MinBlocks<OP>::v) k_edges(Tables t
 // one warp walk a long run alone) go through the lock-free per-op path of k_edges
 // (run_ops) in every chunk, as in unsorted batches.
 //
+// resident blocks per SM (measured on the cfg2 src-sorted bulk build, kernel ms: 3 blocks
+// at 80 registers 3.59; 4: 3.22; 5: 3.16; 6 (40 registers + spills): 3.10; 8: 3.11)
 #ifndef DG_SORTED_MINB
-#define DG_SORTED_MINB 3
+#define DG_SORTED_MINB 6
 #endif
 #ifndef DG_SORTED_PREMATCH
 #define DG_SORTED_PREMATCH 1
