@@ -45,7 +45,12 @@ constexpr int kOrdThreads = 256;
 #endif
 constexpr int kOrdItems = DG_ORDER_ITEMS;  // ops per thread per step (all loads issued first)
 constexpr u32 kOrdStep = kOrdThreads * kOrdItems;
-constexpr int kOrdBlocksPerSm = 4;  // (64 registers: 4 blocks of 256 threads resident)
+// (measured, cfg2 2^24 delete: 4 / 6 / 8 blocks -> scatter 71 / 75 / 90 us: more
+// block ranges leave more partial runs)
+#ifndef DG_ORDER_BLOCKS
+#define DG_ORDER_BLOCKS 4
+#endif
+constexpr int kOrdBlocksPerSm = DG_ORDER_BLOCKS;  // resident blocks of 256 threads per SM
 constexpr u32 kOrdMaxBlocks = 2048;  // k_order_scan: one column per block, 2 per thread
 
 __device__ __forceinline__ void op_of(const u32* src, const u32* dst, u64 n, u64 j, u32& u, u32& v) {
@@ -122,7 +127,7 @@ __device__ __forceinline__ u32 load_step(const u32* __restrict__ src, const u32*
 // rejects the batch; the per-batch counters are reset), so a validated delete reads
 // its inputs once before the scatter instead of twice.
 template <bool VEC>
-__global__ void __launch_bounds__(kOrdThreads) k_order_count(const u32* __restrict__ src,
+__global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_count(const u32* __restrict__ src,
                                                              const u32* __restrict__ dst, u64 n,
                                                              u64 n_ops, u32 nranks, u32 shift,
                                                              u32 nparts, u32* h, u32* totals,
@@ -196,7 +201,7 @@ __global__ void __launch_bounds__(1024) k_order_scan(u32* h, const u32* totals, 
 // partition's run (scattering op by op made every warp store touch 32 sectors:
 // 0.31 ms per 2^24 ops).
 template <bool VEC>
-__global__ void __launch_bounds__(kOrdThreads) k_order_scatter(
+__global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_scatter(
     const u32* __restrict__ src, const u32* __restrict__ dst, u64 n, u64 n_ops, u32 nranks,
     u32 shift, u32 nparts, const u32* __restrict__ h, u32* __restrict__ osrc,
     u32* __restrict__ odst) {
