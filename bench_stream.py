@@ -233,6 +233,7 @@ def run_tc(args, cfg):
     IB = 1 << 22
     t_ins = t_tc = 0.0
     wedges = []  # edgeExist probes of each timed TC, counted on the graph it ran on
+    tc_steps = []  # device ms of each timed TC (this rank)
     tri = []
     clock = None
     # warm-up steps count triangles on the bulk-built graph only; the timed steps are
@@ -261,6 +262,7 @@ def run_tc(args, cfg):
         if timed:
             t_ins += e0.elapsed_time(e1)
             t_tc += e1.elapsed_time(e2)
+            tc_steps.append(e1.elapsed_time(e2))
             tri.append(c)
             # the graph grows every step: count this TC's probes now (untimed, host)
             wedges.append(_wedges(g, rank, world))
@@ -318,6 +320,7 @@ def run_tc(args, cfg):
                    "l2": "flushed (256 MiB write) before every step",
                    "parallelism": parallelism_label(world, f"replicas, wedges split by u mod {world},")},
         "tc": {"triangles_per_step": tri, "tc_ms_per_step": t_tc / K,
+               "tc_ms_steps": [round(x, 3) for x in tc_steps],
                "insert_ms_per_step": t_ins / K, "wedges_per_tc": wedges,
                "wedge_G_per_s": sum(wedges) / (t_tc * 1e-3) / 1e9,
                "insert_M_edges_s": 2 * IB / (t_ins / K * 1e3)},
