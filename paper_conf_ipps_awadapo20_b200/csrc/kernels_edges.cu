@@ -544,8 +544,8 @@ struct MinBlocks {
 __device__ __forceinline__ void fixup_block(const Tables& t, u32* pub, u32 epoch);
 
 // Software grid barrier (every block of the launch is resident: launch_g caps the grid
-// at the occupancy bound): arrivals on ctl->bar_count, the last arrival bumps the
-// generation.  A barrier that is not complete after ~4 s traps (a CUDA error that
+// at the occupancy bound and launches it cooperatively): arrivals on ctl->bar_count,
+// the last arrival bumps the generation.  A barrier that is not complete after ~4 s traps (a CUDA error that
 // makes the handle sticky-bad) instead of hanging.
 __device__ __forceinline__ void grid_barrier(DevCtl* c) {
   __syncthreads();
@@ -1188,6 +1188,18 @@ static cudaError_t launch_g(const Tables& t, const EdgeBatch& a, int sms, cudaSt
     if (e != cudaSuccess) return e;
   } else {
     ab.sorted_path = 0;
+  }
+  if (OP != OP_QUERY && ab.fuse_validate) {
+    // the fused validation's grid barrier needs every block resident: a cooperative
+    // launch guarantees it even when other kernels (another handle's, another
+    // stream's) hold part of the GPU
+    Tables tt = t;
+    void* args[] = {&tt, &ab};
+    const cudaError_t e = cudaLaunchCooperativeKernel((const void*)k_edges<G, S, OP, A>,
+                                                      dim3((unsigned)blocks), dim3(kEdgeBlock),
+                                                      args, 0, s);
+    note_kernel(1);
+    return e;
   }
   k_edges<G, S, OP, A><<<(unsigned)blocks, kEdgeBlock, 0, s>>>(t, ab); note_kernel(1);
   return cudaGetLastError();

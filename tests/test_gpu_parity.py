@@ -852,3 +852,47 @@ def test_src_sorted_batch_beyond_2_24_rows():
     assert g.insert_edges(cuda(s), cuda(d), cuda(w), count=True) == o.insert_edges(s, d, w)[1]
     check_against_oracle(g, o, "sorted batch, 2^24+ rows")
     g.close()
+
+
+def test_concurrent_fused_small_batches():
+    """Two handles on one GPU, each fed small mutating batches (one launch each: the
+    validation runs inside the probe kernel before a grid barrier) on
+    its own stream, enqueued interleaved so the two kernels can overlap.  The
+    cooperative launch keeps every block of each grid resident, so neither barrier
+    can wait on blocks the other kernel holds; both graphs end equal to their oracles
+    (a rejected batch on one of them changes nothing)."""
+    from paper_conf_ipps_awadapo20_b200 import Graph
+    nv = 1 << 16
+    B = 1 << 17  # a near-full grid per launch (the fused path is < 2^18 ops)
+    graphs = [Graph(nv), Graph(nv)]
+    oracles = [Oracle(nv), Oracle(nv)]
+    streams = [torch.cuda.Stream(), torch.cuda.Stream()]
+    batches = {}
+    for b in range(6):
+        for k in range(2):
+            s, d, w = wl.uniform_edges(40 + k, b, B, nv)
+            if k == 1 and b == 3:
+                s = s.copy()
+                s[777] = nv  # out of range: this batch is rejected on graph 1 only
+            batches[(b, k)] = (s, d, w)
+    dev = [[cuda(x) for x in batches[(b, k)]] for b in range(6) for k in range(2)]
+    torch.cuda.synchronize()
+    for b in range(6):
+        for k in range(2):
+            S, D, W = dev[2 * b + k]
+            with torch.cuda.stream(streams[k]):
+                if b % 2 == 0:
+                    graphs[k].insert_edges(S, D, W)
+                else:
+                    graphs[k].delete_edges(S[: B // 2], D[: B // 2])
+    torch.cuda.synchronize()
+    for b in range(6):
+        for k in range(2):
+            s, d, w = batches[(b, k)]
+            if b % 2 == 0:
+                oracles[k].insert_edges(s, d, w)
+            else:
+                oracles[k].delete_edges(s[: B // 2], d[: B // 2])
+    for k in range(2):
+        check_against_oracle(graphs[k], oracles[k], f"graph {k}")
+        graphs[k].close()
