@@ -493,12 +493,14 @@ u64 order_min_ops() {
 // snapshot for validation_status() right after it.
 // *fused: a small batch left to the probe kernel's own validation (EdgeBatch
 // fuse_validate; not when the verdict must be snapshot before the probe).
-dg_status order_batch(dg_graph g, const u32* src, const u32* dst, u64 n, bool mirror, u32 epoch,
-                      bool validate, bool note, const u32** osrc, const u32** odst, bool* ordered,
-                      bool* fused, cudaStream_t s) {
+// w (nullable, insert batches): the weights, permuted with their ops into *ow.
+// want: the caller's decision to order (delete_order_wanted / insert_order_wanted).
+dg_status order_batch(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n, bool mirror,
+                      u32 epoch, bool validate, bool note, bool want, const u32** osrc,
+                      const u32** odst, const u32** ow, bool* ordered, bool* fused,
+                      cudaStream_t s) {
   const u64 n_ops = mirror ? 2 * n : n;
-  const u64 lim = order_min_ops();
-  *ordered = lim != 0 && n_ops >= lim && n_ops < (1ull << 32) && g->rows > 1;
+  *ordered = want;
   *fused = false;
   if (!*ordered) {
     *fused = validate && !note && n_ops < dg::kFuseValidateMaxOps;
@@ -509,19 +511,66 @@ dg_status order_batch(dg_graph g, const u32* src, const u32* dst, u64 n, bool mi
   DG_CK(ensure_buf(g->ord[0], dg::order_scratch_bytes(g->sms)));
   DG_CK(ensure_buf(g->ord[1], n_ops * 4));
   DG_CK(ensure_buf(g->ord[2], n_ops * 4));
+  if (w) DG_CK(ensure_buf(g->ord[3], n_ops * 4));
   dg_status nst = DG_OK;
   auto between = [&]() -> cudaError_t {
     if (note) nst = note_validation(g, s);
     return nst == DG_OK ? cudaSuccess : cudaErrorUnknown;
   };
-  const cudaError_t e = dg::launch_order(src, dst, n, mirror, g->rows, g->nranks, g->ord[0].p,
-                                         (u32*)g->ord[1].p, (u32*)g->ord[2].p, g->nv, epoch,
+  const cudaError_t e = dg::launch_order(src, dst, w, n, mirror, g->rows, g->nranks, g->ord[0].p,
+                                         (u32*)g->ord[1].p, (u32*)g->ord[2].p,
+                                         w ? (u32*)g->ord[3].p : nullptr, g->nv, epoch,
                                          validate ? g->ctl : nullptr, between, g->sms, s);
   if (nst != DG_OK) return nst;
   DG_CK(e);
   *osrc = (const u32*)g->ord[1].p;
   *odst = (const u32*)g->ord[2].p;
+  if (ow) *ow = w ? (const u32*)g->ord[3].p : nullptr;
   return DG_OK;
+}
+
+bool delete_order_wanted(dg_graph g, u64 n_ops) {
+  const u64 lim = order_min_ops();
+  return lim != 0 && n_ops >= lim && n_ops < (1ull << 32) && g->rows > 1;
+}
+
+// Inserts are ordered only when ops of one row rarely meet in flight: at most
+// DG_ORDER_INSERT_PER_ROW (default 1.0) ops per local row on average (measured with the
+// reorder untimed, tools/locality_probe.py: cfg3's 2^24 batch over 24 M rows, 0.7 per
+// row, 1.50 -> 0.95 ms; cfg2's over 4.85 M rows, 3.5 per row, 1.18 -> 1.15 ms: ops
+// of one row then race for the same free slot).
+bool insert_order_wanted(dg_graph g, u64 n_ops);
+
+// An insert batch of this rank (not routed): validation, then the insert — a small
+// batch validates inside its insert launch (one launch instead of two; no sortedness
+// verdict: the src-sorted path is for batches >= 2^18); a large batch over many rows
+// is put in locality order (its count pass validates; an ordered batch is not
+// src-sorted); otherwise k_validate (with the sortedness verdict) and the insert.
+// note: snapshot the verdict for validation_status() (host-buffer calls).
+dg_status validated_insert(dg_graph g, const u32* src, const u32* dst, const u32* w, u64 n,
+                           u32 epoch, bool note, cudaStream_t s) {
+  const bool mirror = !g->directed;
+  const u64 n_ops = mirror ? 2 * n : n;
+  if (insert_order_wanted(g, n_ops)) {
+    const u32 *os = nullptr, *od = nullptr, *ow = nullptr;
+    bool ordered = false, fused = false;
+    DG_TRY(order_batch(g, src, dst, w, n, mirror, epoch, true, note, true, &os, &od, &ow, &ordered,
+                       &fused, s));
+    return local_insert(g, os, od, ow, n_ops, false, epoch, s, false);
+  }
+  const bool fuse = !note && n > 0 && n_ops < kFuseValidateMaxOps;
+  if (!fuse) {
+    DG_CK(launch_validate(src, dst, n, g->nv, epoch, g->ctl, g->sms, s));
+    g->validated_epoch = epoch;
+  }
+  if (note) DG_TRY(note_validation(g, s));
+  return local_insert(g, src, dst, w, n, mirror, epoch, s, fuse);
+}
+
+bool insert_order_wanted(dg_graph g, u64 n_ops) {
+  static const double per_row = std::getenv("DG_ORDER_INSERT_PER_ROW")
+                                    ? std::atof(std::getenv("DG_ORDER_INSERT_PER_ROW")) : 1.0;
+  return delete_order_wanted(g, n_ops) && (double)n_ops <= per_row * (double)g->rows;
 }
 
 // validate / note: see order_batch (the router validates its batches itself)
@@ -535,7 +584,8 @@ dg_status local_delete(dg_graph g, const u32* src, const u32* dst, u64 n, bool m
   }
   prof_mark(g, PROF_DELETE, s);
   bool ordered = false, fused = false;
-  DG_TRY(order_batch(g, src, dst, n, mirror, epoch, validate, note, &src, &dst, &ordered, &fused, s));
+  DG_TRY(order_batch(g, src, dst, nullptr, n, mirror, epoch, validate, note,
+                     delete_order_wanted(g, n_ops), &src, &dst, nullptr, &ordered, &fused, s));
   if (ordered) n = n_ops;  // explicit directed ops (mirrors expanded)
   dg::EdgeBatch a{};
   a.src = src;
@@ -1006,11 +1056,8 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
     DG_TRY(upload_async(g, 8, src, n * 4, s, &ds));
     DG_TRY(upload_async(g, 9, dst, n * 4, s, &dd));
     DG_TRY(upload_async(g, 10, weight, weight ? n * 4 : 0, s, &dw));
-    DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
-    g->validated_epoch = epoch;
-    DG_TRY(note_validation(g, s));
-    DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
-                            epoch, s));
+    DG_TRY(dg::validated_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, true,
+                                s));
     DG_TRY(release_slots(g, 8, 11, s));
     return validation_status(g, epoch);
   }
@@ -1020,15 +1067,8 @@ dg_status dg_insert_edges(dg_graph g, const uint32_t* src, const uint32_t* dst,
   if (g->router) {
     DG_TRY(dg::router_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, s));
   } else {
-    // a small batch validates inside its insert launch (one launch instead of two; no
-    // sortedness verdict: the src-sorted path is for batches >= 2^18)
-    const bool fuse = n > 0 && (g->directed ? n : 2 * n) < dg::kFuseValidateMaxOps;
-    if (!fuse) {
-      DG_CK(dg::launch_validate((const u32*)ds, (const u32*)dd, n, g->nv, epoch, g->ctl, g->sms, s));
-      g->validated_epoch = epoch;
-    }
-    DG_TRY(dg::local_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, !g->directed,
-                            epoch, s, fuse));
+    DG_TRY(dg::validated_insert(g, (const u32*)ds, (const u32*)dd, (const u32*)dw, n, epoch, false,
+                                s));
   }
   if (n_added || host) {
     DG_TRY(read_ctl(g, s));

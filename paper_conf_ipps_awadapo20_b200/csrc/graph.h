@@ -81,8 +81,8 @@ struct dg_graph_s {
   cudaEvent_t val_event = nullptr;  // batch validated (status readable)
   uint32_t* h_fail = nullptr;       // pinned copy of ctl->fail_epoch
   Buf tc[11];  // triangle counting scratch (CSR, orientation, probe order, flat wedge list)
-  Buf ord[3];  // locality order of large delete batches: per-block partition counts /
-               // offsets, permuted src, dst (kernels_order.cu)
+  Buf ord[4];  // locality order of large batches: per-block partition counts / offsets,
+               // permuted src, dst, weights (kernels_order.cu)
   Buf rh[4];  // re-sizing scratch
   Buf big;    // hub-row list (export, stats, TC orientation)
   // per-vertex re-sizing of long chains
@@ -154,6 +154,9 @@ dg_status local_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, con
 dg_status prepare_insert(dg_graph g, uint64_t n_ops, cudaStream_t s);
 // validate: run the batch validation (Q7) first; note: snapshot its verdict for
 // validation_status() (api.cu order_batch)
+// validation + insert of a local (not routed) batch, in locality order when it pays
+dg_status validated_insert(dg_graph g, const uint32_t* src, const uint32_t* dst, const uint32_t* w,
+                           uint64_t n, uint32_t epoch, bool note, cudaStream_t s);
 dg_status local_delete(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,
                        bool mirror, uint32_t epoch, cudaStream_t s, bool validate, bool note);
 dg_status local_query(dg_graph g, const uint32_t* src, const uint32_t* dst, uint64_t n,

@@ -63,9 +63,10 @@ constexpr u32 kOrderPartBits = DG_ORDER_PART_BITS;
 constexpr u32 kMaxOrderParts = 256;
 u32 order_shift(u64 rows);
 size_t order_scratch_bytes(int sms);
-cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64 rows, u32 nranks,
-                         void* scratch, u32* osrc, u32* odst, u64 nv, u32 epoch, DevCtl* ctl,
-                         const std::function<cudaError_t()>& between, int sms, cudaStream_t s);
+cudaError_t launch_order(const u32* src, const u32* dst, const u32* w, u64 n, bool mirror, u64 rows,
+                         u32 nranks, void* scratch, u32* osrc, u32* odst, u32* ow, u64 nv,
+                         u32 epoch, DevCtl* ctl, const std::function<cudaError_t()>& between,
+                         int sms, cudaStream_t s);
 cudaError_t launch_validate(const u32* src, const u32* dst, u64 n, u64 nv, u32 epoch, DevCtl* ctl,
                             int sms, cudaStream_t s);
 cudaError_t launch_insert(int lay, const Tables& t, const EdgeBatch& a, int sms, cudaStream_t s);

@@ -10,12 +10,13 @@
 // any moment cover a window of rows whose buckets fit in L2, so repeated touches of a
 // bucket hit L2 and consecutive DRAM requests fall into nearby pages.  Measured on
 // cfg2 2^24 batches (tools/locality_probe.py, the reorder itself untimed): delete
-// 0.80 -> 0.54 ms, query 0.62 -> 0.49 ms.  Only deletes use it: they are
-// order-independent (each key is removed once, the count is of keys that existed:
-// Q5), so the permuted batch is probed as is.  Inserts gain nothing (ops of one row
-// then race for the same free slot), and queries lose more than they gain (answers
-// written back to the caller's positions scatter 1- and 4-B stores: 7x the DRAM
-// write bytes; measured 0.64 -> 0.78 ms for the probe alone).
+// 0.80 -> 0.54 ms, query 0.62 -> 0.49 ms.  Deletes use it (order-independent: each
+// key is removed once, the count is of keys that existed, Q5), and inserts with at
+// most ~1 op per row (cfg3: 1.50 -> 0.95 ms; with more ops per row they gain nothing:
+// ops of one row then race for the same free slot); the weights move with their ops.
+// Queries lose more than they gain (answers written back to the caller's positions
+// scatter 1- and 4-B stores: 7x the DRAM write bytes; measured 0.64 -> 0.78 ms for
+// the probe alone).
 //
 // The batch is split into one contiguous range per block (B = 4 per SM):
 //   k_order_count   : block b's shared histogram of its range -> h[b][p], totals[p]
@@ -123,6 +124,32 @@ __device__ __forceinline__ u32 load_step(const u32* __restrict__ src, const u32*
   return valid;
 }
 
+// The weights of one step's ops, in load_step's order (mirror op j >= n: w[j - n]).
+template <bool VEC>
+__device__ __forceinline__ void load_w_step(const u32* __restrict__ w, u64 n, u64 j0, u64 hi,
+                                            u32 (&ws)[kOrdItems]) {
+  if constexpr (VEC) {
+#pragma unroll
+    for (int k = 0; k < kOrdItems / 4; ++k) {
+      const u64 j = j0 + 4 * ((u64)k * kOrdThreads + threadIdx.x);
+      if (j + 3 < hi) {
+        const uint4 a = *reinterpret_cast<const uint4*>(w + (j >= n ? j - n : j));
+        ws[4 * k] = a.x; ws[4 * k + 1] = a.y; ws[4 * k + 2] = a.z; ws[4 * k + 3] = a.w;
+      } else {
+#pragma unroll
+        for (int i = 0; i < 4; ++i)
+          ws[4 * k + i] = j + i < hi ? w[j + i >= n ? j + i - n : j + i] : 0u;
+      }
+    }
+  } else {
+#pragma unroll
+    for (int k = 0; k < kOrdItems; ++k) {
+      const u64 j = j0 + (u64)k * kOrdThreads + threadIdx.x;
+      ws[k] = j < hi ? w[j >= n ? j - n : j] : 0u;
+    }
+  }
+}
+
 // ctl != nullptr: also the batch validation of k_validate (Q7: an endpoint >= nv
 // rejects the batch; the per-batch counters are reset), so a validated delete reads
 // its inputs once before the scatter instead of twice.
@@ -200,14 +227,16 @@ __global__ void __launch_bounds__(1024) k_order_scan(u32* h, const u32* totals, 
 // them out in that order, so consecutive threads store consecutive slots of one
 // partition's run (scattering op by op made every warp store touch 32 sectors:
 // 0.31 ms per 2^24 ops).
-template <bool VEC>
+// WT: the batch carries weights (an insert batch), moved with their ops.
+template <bool VEC, bool WT>
 __global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_scatter(
-    const u32* __restrict__ src, const u32* __restrict__ dst, u64 n, u64 n_ops, u32 nranks,
-    u32 shift, u32 nparts, const u32* __restrict__ h, u32* __restrict__ osrc,
-    u32* __restrict__ odst) {
+    const u32* __restrict__ src, const u32* __restrict__ dst, const u32* __restrict__ w, u64 n,
+    u64 n_ops, u32 nranks, u32 shift, u32 nparts, const u32* __restrict__ h,
+    u32* __restrict__ osrc, u32* __restrict__ odst, u32* __restrict__ ow) {
   __shared__ u32 cur[kMaxOrderParts];   // next output slot of each partition
   __shared__ u32 cnt[kMaxOrderParts];   // this step: ops per partition, then their offsets
   __shared__ u32 st_u[kOrdStep], st_v[kOrdStep];
+  __shared__ u32 st_w[WT ? kOrdStep : 1];
   __shared__ uint8_t st_p[kOrdStep];
   __shared__ u32 wsum[kOrdThreads / 32];
   static_assert(kMaxOrderParts == kOrdThreads, "one partition per thread in the scan");
@@ -217,8 +246,9 @@ __global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_scatter(
   range_of(n_ops, lo, hi);
   // software pipeline: the next step's loads are issued once the current step's ops
   // are staged in shared memory, so they are in flight during its stores
-  u32 us[kOrdItems], vs[kOrdItems];
+  u32 us[kOrdItems], vs[kOrdItems], ws[kOrdItems];
   u32 valid = lo < hi ? load_step<VEC>(src, dst, n, lo, hi, true, us, vs) : 0u;
+  if (WT && lo < hi) load_w_step<VEC>(w, n, lo, hi, ws);
   for (u64 j0 = lo; j0 < hi; j0 += kOrdStep) {
     cnt[t] = 0;
     __syncthreads();
@@ -253,9 +283,11 @@ __global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_scatter(
       const u32 at = cnt[ps[k]] + rk[k];
       st_u[at] = us[k];
       st_v[at] = vs[k];
+      if (WT) st_w[at] = ws[k];
       st_p[at] = (uint8_t)ps[k];
     }
     valid = j0 + kOrdStep < hi ? load_step<VEC>(src, dst, n, j0 + kOrdStep, hi, true, us, vs) : 0u;
+    if (WT && j0 + kOrdStep < hi) load_w_step<VEC>(w, n, j0 + kOrdStep, hi, ws);
     __syncthreads();
     const u32 m = (u32)(hi - j0 < kOrdStep ? hi - j0 : kOrdStep);
     for (u32 i = t; i < m; i += kOrdThreads) {  // runs of one partition are contiguous
@@ -263,6 +295,7 @@ __global__ void __launch_bounds__(kOrdThreads, kOrdBlocksPerSm) k_order_scatter(
       const u32 at = cur[p] + (i - cnt[p]);
       osrc[at] = st_u[i];
       odst[at] = st_v[i];
+      if (WT) ow[at] = st_w[i];
     }
     __syncthreads();
     if (t < nparts) cur[t] += c;
@@ -290,9 +323,11 @@ size_t order_scratch_bytes(int sms) {
 // ctl != nullptr: the count pass validates the batch (k_validate's job); `between`,
 // when set, runs on the stream after that pass and before the scatter (the caller's
 // snapshot of the verdict).
-cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64 rows, u32 nranks,
-                         void* scratch, u32* osrc, u32* odst, u64 nv, u32 epoch, DevCtl* ctl,
-                         const std::function<cudaError_t()>& between, int sms, cudaStream_t s) {
+// w / ow (nullable): the batch's weights and their permuted copy (insert batches)
+cudaError_t launch_order(const u32* src, const u32* dst, const u32* w, u64 n, bool mirror, u64 rows,
+                         u32 nranks, void* scratch, u32* osrc, u32* odst, u32* ow, u64 nv,
+                         u32 epoch, DevCtl* ctl, const std::function<cudaError_t()>& between,
+                         int sms, cudaStream_t s) {
   const u64 n_ops = mirror ? 2 * n : n;
   const u32 shift = order_shift(rows);
   u32 nparts = (u32)(((rows ? rows : 1) + (1ull << shift) - 1) >> shift);
@@ -303,7 +338,8 @@ cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64
   u32* totals = h + (size_t)nb * kMaxOrderParts;
   cudaError_t e = cudaMemsetAsync(totals, 0, kMaxOrderParts * 4, s);
   if (e != cudaSuccess) return e;
-  const bool vec = ((reinterpret_cast<uintptr_t>(src) | reinterpret_cast<uintptr_t>(dst)) & 15) == 0 &&
+  const bool vec = ((reinterpret_cast<uintptr_t>(src) | reinterpret_cast<uintptr_t>(dst) |
+                     reinterpret_cast<uintptr_t>(w)) & 15) == 0 &&
                    (!mirror || n % 4 == 0);
   if (vec)
     k_order_count<true><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
@@ -313,12 +349,15 @@ cudaError_t launch_order(const u32* src, const u32* dst, u64 n, bool mirror, u64
                                                     totals, nv, epoch, ctl);
   if (between && (e = between()) != cudaSuccess) return e;
   k_order_scan<<<nparts, 1024, 0, s>>>(h, totals, (u32)nb);
-  if (vec)
-    k_order_scatter<true><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
-                                                     osrc, odst);
-  else
-    k_order_scatter<false><<<nb, kOrdThreads, 0, s>>>(src, dst, n, n_ops, nranks, shift, nparts, h,
-                                                      osrc, odst);
+#define DG_SCATTER(V_, W_)                                                                   \
+  k_order_scatter<V_, W_><<<nb, kOrdThreads, 0, s>>>(src, dst, w, n, n_ops, nranks, shift, nparts, \
+                                                     h, osrc, odst, ow)
+  if (w) {
+    if (vec) DG_SCATTER(true, true); else DG_SCATTER(false, true);
+  } else {
+    if (vec) DG_SCATTER(true, false); else DG_SCATTER(false, false);
+  }
+#undef DG_SCATTER
   note_kernel(3);
   return cudaGetLastError();
 }
