@@ -21,8 +21,8 @@ import time
 import numpy as np
 
 import workloads as wl
-from bench import (METRIC, UNIT, ClockSampler, config_block, dist_env, load_peaks, make_coll,
-                   model_bytes, parallelism_label, slice_of)
+from bench import (L2_NOTE, METRIC, UNIT, ClockSampler, L2Flush, config_block, dist_env,
+                   load_peaks, make_coll, model_bytes, parallelism_label, slice_of)
 
 
 def _setup(args):
@@ -85,7 +85,7 @@ def run_mixed(args, cfg):
     torch.cuda.synchronize()
     bulk_ms = _max(torch, pg, dev, [a0.elapsed_time(a1)])[0]
     del BS, BD, BW
-    flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
+    flush = L2Flush(dev)
     IB, QB, DB, VB, RB = 1 << 22, 1 << 22, 1 << 21, 1 << 12, 1 << 16
     names = ["insert", "query", "delete", "delete_vertices", "reinsert"]
     tot = dict.fromkeys(names, 0.0)
@@ -133,7 +133,7 @@ def run_mixed(args, cfg):
             torch.cuda.synchronize()
             if pg:
                 pg.barrier()
-            flush.zero_()
+            flush()
             e0, e1 = ev(), ev()
             e0.record()
             fn(inp)
@@ -187,7 +187,7 @@ def run_mixed(args, cfg):
                                f"insert {IB:,} + query {QB:,} + delete {DB:,} edges + delete "
                                f"{VB:,} vertices + re-insert {RB:,} edges (global)",
                    "bucket_bytes": S, "load_factor": args.load_factor,
-                   "l2": "flushed (256 MiB write) before every timed op; tables >> L2",
+                   "l2": L2_NOTE,
                    "parallelism": parallelism_label(world)},
         "ops": ops, "bulk_build": {"insert_ms": bulk_ms, "unique_added": int(added0)},
         "roofline": roofline, "gpu_launches": prof["launches"], "clocks": clocks,
@@ -229,7 +229,7 @@ def run_tc(args, cfg):
     torch.cuda.synchronize()
     bulk_ms = a0.elapsed_time(a1)
     del BS, BD
-    flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
+    flush = L2Flush(dev)
     IB = 1 << 22
     t_ins = t_tc = 0.0
     wedges = []  # edgeExist probes of each timed TC, counted on the graph it ran on
@@ -251,7 +251,7 @@ def run_tc(args, cfg):
         torch.cuda.synchronize()
         if pg:
             pg.barrier()
-        flush.zero_()
+        flush()
         e0, e1, e2 = ev(), ev(), ev()
         e0.record()
         g.insert_edges(S1, D1)
@@ -317,7 +317,7 @@ def run_tc(args, cfg):
                                f"(edge ops counted: 2 directed inserts per edge + 1 edgeExist "
                                f"per wedge)",
                    "bucket_bytes": S, "load_factor": args.load_factor, "variant": variant,
-                   "l2": "flushed (256 MiB write) before every step",
+                   "l2": L2_NOTE + " (before every step)",
                    "parallelism": parallelism_label(world, f"replicas, wedges split by u mod {world},")},
         "tc": {"triangles_per_step": tri, "tc_ms_per_step": t_tc / K,
                "tc_ms_steps": [round(x, 3) for x in tc_steps],
