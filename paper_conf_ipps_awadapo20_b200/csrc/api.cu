@@ -1,3 +1,4 @@
+#include <chrono>
 // api.cu — the C ABI (include/dg.h) on top of the sm_100a kernels.
 #include <algorithm>
 #include <cmath>
@@ -47,14 +48,17 @@ bool is_device_ptr(const void* p) {
 }
 
 // grow-only scratch buffer
-cudaError_t ensure_buf(dg_graph_s::Buf& b, size_t bytes) {
+cudaError_t ensure_buf(dg_graph_s::Buf& b, size_t bytes, bool big_slack = false) {
   if (bytes <= b.bytes) return cudaSuccess;
   if (b.p) cudaFree(b.p);
   b.p = nullptr;
   b.bytes = 0;
   // geometric headroom: buffers that track a growing graph (TC scratch, export
-  // staging) are not re-allocated (cudaFree synchronises the device) every call
-  size_t want = std::max<size_t>(bytes + bytes / 4, 1 << 20);
+  // staging) are not re-allocated (cudaFree synchronises the device) every call;
+  // big_slack (the triangle-count scratch, re-sized as the graph grows every dynamic
+  // step): 2x — a cudaFree + cudaMalloc of a multi-GB buffer measured 40-600 ms on
+  // cfg5's growing graph (DG_TRACE_TC)
+  size_t want = std::max<size_t>(big_slack ? 2 * bytes : bytes + bytes / 4, 1 << 20);
   cudaError_t e = cudaMalloc(&b.p, want);
   if (e == cudaSuccess) b.bytes = want;
   return e;
@@ -1441,24 +1445,36 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   if (g->nranks != 1) return DG_ERR_UNSUPPORTED;
   cudaStream_t s = reinterpret_cast<cudaStream_t>(stream);
   *count = 0;
+  // DG_TRACE_TC=1: wall time of each phase (synchronising after each) on stderr
+  static const bool trace = std::getenv("DG_TRACE_TC") != nullptr;
+  auto tprev = std::chrono::steady_clock::now();
+  auto tmark = [&](const char* what) {
+    if (!trace) return;
+    cudaStreamSynchronize(s);
+    const auto now = std::chrono::steady_clock::now();
+    std::fprintf(stderr, "dg tc: %-12s %8.3f ms\n", what,
+                 std::chrono::duration<double, std::milli>(now - tprev).count());
+    tprev = now;
+  };
   const dg::Tables t = g->tables();
   const u64 rows = g->rows;
   // (1) adjacency export (a12): CSR of every A_u
-  DG_CK(ensure_buf(g->tc[0], (rows + 1) * 8));
+  DG_CK(ensure_buf(g->tc[0], (rows + 1) * 8, true));
   u64* ro = reinterpret_cast<u64*>(g->tc[0].p);
   DG_CK(dg::launch_export_offsets(t, ro, &g->scan_temp, &g->scan_bytes, s));
   u64 m = 0;
   DG_CK(cudaMemcpyAsync(&m, ro + rows, 8, cudaMemcpyDeviceToHost, s));
   DG_CK(cudaStreamSynchronize(s));
   if (m >= 0xFFFFFFFFull) return DG_ERR_UNSUPPORTED;
-  DG_CK(ensure_buf(g->tc[1], m * 4 + 4));
+  DG_CK(ensure_buf(g->tc[1], m * 4 + 4, true));
   u32* dst = reinterpret_cast<u32*>(g->tc[1].p);
-  DG_CK(ensure_buf(g->big, (rows + 2) * 4));
+  DG_CK(ensure_buf(g->big, (rows + 2) * 4, true));
   u32* big = reinterpret_cast<u32*>(g->big.p);
   DG_CK(dg::launch_export_fill(g->lay, t, ro, dst, nullptr, big, g->sms, s));
+  tmark("export");
   // (2) orientation by rank = (degree, id)
-  DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8));
-  DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8));
+  DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8, true));
+  DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8, true));
   u64* ocnt = reinterpret_cast<u64*>(g->tc[2].p);
   u64* oro = reinterpret_cast<u64*>(g->tc[3].p);
   DG_CK(dg::launch_tc_orient_count(t, ro, dst, part, nparts, ocnt, big, g->sms, s));
@@ -1466,11 +1482,12 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   u64 mo = 0;
   DG_CK(cudaMemcpyAsync(&mo, oro + rows, 8, cudaMemcpyDeviceToHost, s));
   DG_CK(cudaStreamSynchronize(s));
-  DG_CK(ensure_buf(g->tc[4], mo * 4 + 4));
-  DG_CK(ensure_buf(g->tc[5], mo * 4 + 4));
+  DG_CK(ensure_buf(g->tc[4], mo * 4 + 4, true));
+  DG_CK(ensure_buf(g->tc[5], mo * 4 + 4, true));
   u32* oadj = reinterpret_cast<u32*>(g->tc[4].p);
   u32* oend = reinterpret_cast<u32*>(g->tc[5].p);
   DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, big, g->sms, s));
+  tmark("orient");
   // (3) probe order: entries sorted by the probed vertex (kernels_tc.cu; off unless
   // DG_TC_ORDER=1: measured on cfg5 it cuts the wedge kernel's DRAM reads 380 -> 52 GB
   // but mixes entries of very different candidate counts in a warp, 64 -> 150 G
@@ -1479,8 +1496,8 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   static const bool tc_order = std::getenv("DG_TC_ORDER") != nullptr &&
                                std::atoi(std::getenv("DG_TC_ORDER")) != 0;
   if (tc_order) {
-    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8));
-    DG_CK(ensure_buf(g->tc[7], mo * 8 + 8));
+    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8, true));
+    DG_CK(ensure_buf(g->tc[7], mo * 8 + 8, true));
     DG_CK(dg::launch_tc_probe_order(oadj, mo, rows, (u32*)g->tc[6].p, (u32*)g->tc[7].p, &perm,
                                     &g->scan_temp, &g->scan_bytes, s));
   }
@@ -1495,9 +1512,9 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   u32* chunk_k = nullptr;
   unsigned long long* nlist_dev = nullptr;
   if (flat) {
-    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8));  // (shared with the probe order's keys)
-    DG_CK(ensure_buf(g->tc[8], mo * 8 + 8));
-    DG_CK(ensure_buf(g->tc[9], mo * 8 + 16));
+    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8, true));  // (shared with the probe order's keys)
+    DG_CK(ensure_buf(g->tc[8], mo * 8 + 8, true));
+    DG_CK(ensure_buf(g->tc[9], mo * 8 + 16, true));
     list = (uint2*)g->tc[8].p;
     woff = (u64*)g->tc[9].p;
     nlist_dev = (unsigned long long*)((char*)g->tc[6].p + mo * 8);
@@ -1507,8 +1524,9 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
     u64 wedges = 0;  // (sizes the chunk table)
     DG_CK(cudaMemcpyAsync(&wedges, woff + nl, 8, cudaMemcpyDeviceToHost, s));
     DG_CK(cudaStreamSynchronize(s));
-    DG_CK(ensure_buf(g->tc[10], dg::tc_chunk_count(wedges) * 4 + 4));
+    DG_CK(ensure_buf(g->tc[10], dg::tc_chunk_count(wedges) * 4 + 4, true));
     chunk_k = (u32*)g->tc[10].p;
+  tmark("flat_prep");
   }
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));
   dg::prof_mark(g, dg::PROF_TC, s);
@@ -1519,6 +1537,7 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
     DG_CK(dg::launch_tc_wedges(g->lay, t, oadj, oend, perm, mo,
                                reinterpret_cast<unsigned long long*>(&g->ctl->count), g->sms, s));
   dg::prof_mark(g, dg::PROF_TC, s);
+  tmark("wedges");
   DG_TRY(read_ctl(g, s));
   *count = g->hctl->count;
   return DG_OK;
