@@ -787,8 +787,7 @@ static void destroy_graph(dg_graph g) {
   if (g->small_dev) cudaFree(g->small_dev);
   for (auto& b : g->stage)
     if (b.p) cudaFree(b.p);
-  for (auto& b : g->tc)
-    if (b.p) cudaFree(b.p);
+  for (auto& a : g->tcv) a.release();
   for (auto& b : g->rh)
     if (b.p) cudaFree(b.p);
   if (g->big.p) cudaFree(g->big.p);
@@ -1438,6 +1437,17 @@ dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* stream) 
   return DG_OK;
 }
 
+// Triangle-count scratch k: a growable VMM array (a large virtual range reserved once,
+// physical memory mapped at its end as the graph grows: no free, no copy, no
+// re-allocation of the whole buffer — cudaFree + cudaMalloc of multi-GB scratch cost
+// 40-600 ms on single cfg5 steps).  The contents need not survive growth.
+static dg_status tc_buf(dg_graph g, int k, size_t bytes, cudaStream_t s) {
+  dg::VmmArray& a = g->tcv[k];
+  if (!a.ptr()) DG_CK(a.reserve(g->device, 64ull << 30));
+  DG_CK(a.ensure(bytes, -1, s));
+  return DG_OK;
+}
+
 dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t* count,
                             void* stream) {
   DG_TRY(check_handle(g));
@@ -1459,33 +1469,33 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   const dg::Tables t = g->tables();
   const u64 rows = g->rows;
   // (1) adjacency export (a12): CSR of every A_u
-  DG_CK(ensure_buf(g->tc[0], (rows + 1) * 8, true));
-  u64* ro = reinterpret_cast<u64*>(g->tc[0].p);
+  DG_TRY(tc_buf(g, 0, (rows + 1) * 8, s));
+  u64* ro = reinterpret_cast<u64*>(g->tcv[0].ptr());
   DG_CK(dg::launch_export_offsets(t, ro, &g->scan_temp, &g->scan_bytes, s));
   u64 m = 0;
   DG_CK(cudaMemcpyAsync(&m, ro + rows, 8, cudaMemcpyDeviceToHost, s));
   DG_CK(cudaStreamSynchronize(s));
   if (m >= 0xFFFFFFFFull) return DG_ERR_UNSUPPORTED;
-  DG_CK(ensure_buf(g->tc[1], m * 4 + 4, true));
-  u32* dst = reinterpret_cast<u32*>(g->tc[1].p);
+  DG_TRY(tc_buf(g, 1, m * 4 + 4, s));
+  u32* dst = reinterpret_cast<u32*>(g->tcv[1].ptr());
   DG_CK(ensure_buf(g->big, (rows + 2) * 4, true));
   u32* big = reinterpret_cast<u32*>(g->big.p);
   DG_CK(dg::launch_export_fill(g->lay, t, ro, dst, nullptr, big, g->sms, s));
   tmark("export");
   // (2) orientation by rank = (degree, id)
-  DG_CK(ensure_buf(g->tc[2], (rows + 1) * 8, true));
-  DG_CK(ensure_buf(g->tc[3], (rows + 1) * 8, true));
-  u64* ocnt = reinterpret_cast<u64*>(g->tc[2].p);
-  u64* oro = reinterpret_cast<u64*>(g->tc[3].p);
+  DG_TRY(tc_buf(g, 2, (rows + 1) * 8, s));
+  DG_TRY(tc_buf(g, 3, (rows + 1) * 8, s));
+  u64* ocnt = reinterpret_cast<u64*>(g->tcv[2].ptr());
+  u64* oro = reinterpret_cast<u64*>(g->tcv[3].ptr());
   DG_CK(dg::launch_tc_orient_count(t, ro, dst, part, nparts, ocnt, big, g->sms, s));
   DG_CK(dg::scan_exclusive_u64(ocnt, oro, rows + 1, &g->scan_temp, &g->scan_bytes, s));
   u64 mo = 0;
   DG_CK(cudaMemcpyAsync(&mo, oro + rows, 8, cudaMemcpyDeviceToHost, s));
   DG_CK(cudaStreamSynchronize(s));
-  DG_CK(ensure_buf(g->tc[4], mo * 4 + 4, true));
-  DG_CK(ensure_buf(g->tc[5], mo * 4 + 4, true));
-  u32* oadj = reinterpret_cast<u32*>(g->tc[4].p);
-  u32* oend = reinterpret_cast<u32*>(g->tc[5].p);
+  DG_TRY(tc_buf(g, 4, mo * 4 + 4, s));
+  DG_TRY(tc_buf(g, 5, mo * 4 + 4, s));
+  u32* oadj = reinterpret_cast<u32*>(g->tcv[4].ptr());
+  u32* oend = reinterpret_cast<u32*>(g->tcv[5].ptr());
   DG_CK(dg::launch_tc_orient_fill(t, ro, dst, part, nparts, oro, oadj, oend, big, g->sms, s));
   tmark("orient");
   // (3) probe order: entries sorted by the probed vertex (kernels_tc.cu; off unless
@@ -1496,9 +1506,9 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   static const bool tc_order = std::getenv("DG_TC_ORDER") != nullptr &&
                                std::atoi(std::getenv("DG_TC_ORDER")) != 0;
   if (tc_order) {
-    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8, true));
-    DG_CK(ensure_buf(g->tc[7], mo * 8 + 8, true));
-    DG_CK(dg::launch_tc_probe_order(oadj, mo, rows, (u32*)g->tc[6].p, (u32*)g->tc[7].p, &perm,
+    DG_TRY(tc_buf(g, 6, mo * 8 + 8, s));
+    DG_TRY(tc_buf(g, 7, mo * 8 + 8, s));
+    DG_CK(dg::launch_tc_probe_order(oadj, mo, rows, (u32*)g->tcv[6].ptr(), (u32*)g->tcv[7].ptr(), &perm,
                                     &g->scan_temp, &g->scan_bytes, s));
   }
   // (4) one edgeExist per wedge: uniform layouts number the wedges and give every lane
@@ -1512,20 +1522,19 @@ dg_status dg_triangle_count(dg_graph g, uint32_t part, uint32_t nparts, uint64_t
   u32* chunk_k = nullptr;
   unsigned long long* nlist_dev = nullptr;
   if (flat) {
-    DG_CK(ensure_buf(g->tc[6], mo * 8 + 8, true));  // (shared with the probe order's keys)
-    DG_CK(ensure_buf(g->tc[8], mo * 8 + 8, true));
-    DG_CK(ensure_buf(g->tc[9], mo * 8 + 16, true));
-    list = (uint2*)g->tc[8].p;
-    woff = (u64*)g->tc[9].p;
-    nlist_dev = (unsigned long long*)((char*)g->tc[6].p + mo * 8);
+    DG_TRY(tc_buf(g, 8, mo * 8 + 8, s));
+    DG_TRY(tc_buf(g, 9, mo * 8 + 24, s));
+    list = (uint2*)g->tcv[8].ptr();
+    woff = (u64*)g->tcv[9].ptr();
+    nlist_dev = (unsigned long long*)((char*)g->tcv[9].ptr() + mo * 8 + 8);  // (after woff[mo])
     u64 nl = 0;
     DG_CK(dg::launch_tc_flat_prepare(oadj, oend, perm, mo, list, woff, nlist_dev, &nl, &g->scan_temp,
                                      &g->scan_bytes, s));
     u64 wedges = 0;  // (sizes the chunk table)
     DG_CK(cudaMemcpyAsync(&wedges, woff + nl, 8, cudaMemcpyDeviceToHost, s));
     DG_CK(cudaStreamSynchronize(s));
-    DG_CK(ensure_buf(g->tc[10], dg::tc_chunk_count(wedges) * 4 + 4, true));
-    chunk_k = (u32*)g->tc[10].p;
+    DG_TRY(tc_buf(g, 10, dg::tc_chunk_count(wedges) * 4 + 4, s));
+    chunk_k = (u32*)g->tcv[10].ptr();
   tmark("flat_prep");
   }
   DG_CK(cudaMemsetAsync(&g->ctl->count, 0, 8, s));

@@ -80,7 +80,7 @@ struct dg_graph_s {
   cudaEvent_t slot_ev[16] = {};
   cudaEvent_t val_event = nullptr;  // batch validated (status readable)
   uint32_t* h_fail = nullptr;       // pinned copy of ctl->fail_epoch
-  Buf tc[11];  // triangle counting scratch (CSR, orientation, probe order, flat wedge list)
+  dg::VmmArray tcv[11];  // triangle counting scratch (CSR, orientation, probe order, flat wedge list)
   Buf ord[4];  // locality order of large batches: per-block partition counts / offsets,
                // permuted src, dst, weights (kernels_order.cu)
   Buf rh[4];  // re-sizing scratch
