@@ -1443,7 +1443,12 @@ dg_status dg_flush_tombstones(dg_graph g, uint64_t* rows_rebuilt, void* stream) 
 // 40-600 ms on single cfg5 steps).  The contents need not survive growth.
 static dg_status tc_buf(dg_graph g, int k, size_t bytes, cudaStream_t s) {
   dg::VmmArray& a = g->tcv[k];
-  if (!a.ptr()) DG_CK(a.reserve(g->device, 64ull << 30));
+  if (!a.ptr()) {
+    // first use: map twice the need, so a graph that keeps growing between triangle
+    // counts (cfg5 more than doubles over its 10 steps) maps new memory rarely
+    DG_CK(a.reserve(g->device, 64ull << 30));
+    DG_CK(a.ensure(std::min<size_t>(2 * bytes, a.reserved()), -1, s));
+  }
   DG_CK(a.ensure(bytes, -1, s));
   return DG_OK;
 }
