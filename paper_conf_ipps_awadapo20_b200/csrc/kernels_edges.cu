@@ -533,8 +533,8 @@ struct Prefetch {
 #ifndef DG_MINB_QRY
 #define DG_MINB_QRY 3
 #endif
-#ifndef DG_MINB_DEL
-#define DG_MINB_DEL 4
+#ifndef DG_MINB_DEL  // (round 2, locality-ordered deletes: 5 blocks 0.666 -> 0.652 ms on cfg2,
+#define DG_MINB_DEL 5  //  6 blocks 0.80 ms; profiles/r02/ab/occupancy/)
 #endif
 template <int OP>
 struct MinBlocks {
